@@ -1,0 +1,407 @@
+"""Benchmark of the staged multi-level-tiled hot path (Baskaran et al., PPoPP'08) on B200.
+
+One step = one pass of the whole hot path over one batch:
+  * Jacobi (BASELINE config 3): T = 1024 steps of the fp32 1-D Jacobi stencil over
+    n_local = 2^26 cells per GPU, time-tiled (one launch per time tile);
+  * ME (BASELINE config 4): full-search SAD motion estimation of a 64-pair batch of
+    1920x1080 uint8 frames, +-32, 16x16 macroblocks, per GPU.
+Multi-GPU (torchrun, one process per GPU): weak scaling.  Jacobi's global domain is the
+concatenation of the ranks' slabs with a halo exchange (NCCL send/recv inside libsp) once
+per time tile; ME ranks search their own 64-pair shard of a 64*N-pair batch (no data-path
+collective).  `value` = Jacobi point-updates of all ranks / max-over-ranks device time;
+ME's throughput is reported in the `me` object with its own roofline.
+
+  python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference] [--time-tile Tt]
+"""
+from __future__ import annotations
+
+import argparse
+import json
+import os
+import statistics
+import subprocess
+import sys
+import threading
+import time
+
+import numpy as np
+
+ROOT = os.path.dirname(os.path.abspath(__file__))
+sys.path.insert(0, ROOT)
+
+METRIC = "Jacobi GPoint-updates/s & ME SAD/s; %HBM roofline at 1/2/4/8 B200"
+JAC_N_LOCAL = 1 << 26
+JAC_T = 1024
+ME_W, ME_H, ME_R, ME_PAIRS = 1920, 1080, 32, 64
+VABSDIFF4_PER_CLK_SM = 64  # measured issue rate (profiles/r01_ubench_issue_rates.txt)
+
+
+def me_valid_sads(width, height, r, pairs):
+    tot = 0
+    for by in range(height // 16):
+        y0 = 16 * by
+        ny = min(r, height - 16 - y0) - max(-r, -y0) + 1
+        for bx in range(width // 16):
+            x0 = 16 * bx
+            tot += (min(r, width - 16 - x0) - max(-r, -x0) + 1) * ny
+    return tot * pairs
+
+
+def peaks():
+    p = {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0, "source": "fallback (B200_PROFILING.md)"}
+    try:
+        with open(os.path.join(ROOT, "MEASURED_PEAKS.json")) as f:
+            m = json.load(f)
+        p = {"hbm_gbs": float(m["hbm_gbs"]), "sm_max_mhz": float(m.get("sm_max_mhz", 1965.0)),
+             "source": "measured (MEASURED_PEAKS.json)"}
+    except Exception:
+        pass
+    return p
+
+
+class ClockSampler:
+    """nvidia-smi clocks and throttle reasons sampled during the timed region."""
+
+    def __init__(self, device: int):
+        self.device = device
+        self.proc = None
+        self.lines: list[str] = []
+
+    def __enter__(self):
+        try:
+            self.proc = subprocess.Popen(
+                ["nvidia-smi", "-i", str(self.device), "--query-gpu=clocks.sm,clocks.max.sm,clocks_event_reasons.active,"
+                 "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
+                 "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap",
+                 "--format=csv,noheader,nounits", "-lms", "100"],
+                stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
+            self.t = threading.Thread(target=self._read, daemon=True)
+            self.t.start()
+        except Exception:
+            self.proc = None
+        return self
+
+    def _read(self):
+        for line in self.proc.stdout:
+            self.lines.append(line.strip())
+
+    def __exit__(self, *a):
+        if self.proc:
+            self.proc.terminate()
+            try:
+                self.proc.wait(timeout=5)
+            except Exception:
+                self.proc.kill()
+            self.t.join(timeout=2)
+
+    def summary(self):
+        sm, mx, reasons = [], None, set()
+        for ln in self.lines:
+            f = [x.strip() for x in ln.split(",")]
+            if len(f) < 7:
+                continue
+            try:
+                sm.append(float(f[0]))
+                mx = float(f[1])
+            except ValueError:
+                continue
+            for name, v in zip(["hw_slowdown", "hw_thermal_slowdown", "sw_thermal_slowdown", "sw_power_cap"], f[3:7]):
+                if v.lower() == "active":
+                    reasons.add(name)
+        if not sm:
+            return {"sm_mhz": None, "sm_max_mhz": None, "reasons": [], "samples": 0}
+        return {"sm_mhz": statistics.median(sm), "sm_max_mhz": mx, "reasons": sorted(reasons), "samples": len(sm)}
+
+
+def traffic_from_profiles():
+    """dram read+write bytes per launch from the committed ncu summary, if present."""
+    try:
+        with open(os.path.join(ROOT, "profiles", "ncu_traffic.json")) as f:
+            return json.load(f)
+    except Exception:
+        return {}
+
+
+# ---------------------------------------------------------------------------------------
+# reference arm: the CPU oracle, as it stands, on the host cores
+# ---------------------------------------------------------------------------------------
+def oracle_samples(rng_seed=0):
+    """Bounded samples of the bench workload for the oracle (~2-4 s of CPU per call)."""
+    import oracle
+    import sp_inputs
+    cores = len(os.sched_getaffinity(0))
+    oracle.set_threads(cores)
+    # Jacobi: the full 2^26-cell state, 16 of the 1024 steps
+    a = sp_inputs.jacobi_input(JAC_N_LOCAL, seed=sp_inputs.JACOBI_BENCH_SEED)
+    js = 16
+    t0 = time.perf_counter()
+    oracle.jacobi1d(a, js)
+    tj = time.perf_counter() - t0
+    jac = (JAC_N_LOCAL - 2) * js / tj
+    # ME: 2 macroblock rows (interior) of one 1080p pair at +-32
+    fr0 = sp_inputs.me_frame(0, ME_W, ME_H, ME_R)
+    fr1 = sp_inputs.me_frame(1, ME_W, ME_H, ME_R)
+    mbx = ME_W // 16
+    mbs = np.arange(30 * mbx, 32 * mbx, dtype=np.int32)
+    t0 = time.perf_counter()
+    oracle.me_search(fr0, fr1, ME_W, ME_H, ME_R, mbs=mbs)
+    tm = time.perf_counter() - t0
+    me = len(mbs) * (2 * ME_R + 1) ** 2 / tm
+    return {"jacobi_ups": jac, "me_sads": me, "cores": oracle.get_threads(), "jacobi_s": tj, "me_s": tm,
+            "sample": f"Jacobi: N=2^26 cells x {js} steps (of T=1024); ME: {len(mbs)} interior macroblocks "
+                      f"(2 MB rows) of one 1920x1080 pair at +-32"}
+
+
+def run_reference(args, rank, world):
+    if rank != 0:
+        return 0
+    for _ in range(args.warmup):
+        oracle_samples()
+    js, ms, tot = [], [], 0.0
+    t_start = time.perf_counter()
+    last = None
+    for _ in range(args.steps):
+        last = oracle_samples()
+        js.append(last["jacobi_ups"])
+        ms.append(last["me_sads"])
+    tot = time.perf_counter() - t_start
+    val = statistics.median(js) / 1e9
+    line = {
+        "impl": "reference", "metric": METRIC, "value": val, "unit": "GPoint-updates/s", "n_gpus": args.gpus,
+        "steps": args.steps, "warmup": args.warmup, "ms_per_step": tot / max(1, args.steps) * 1e3,
+        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
+        "config": {"workload": "J3 (Jacobi fp32 N=2^26, T=1024) + M4 (ME 1920x1080 +-32 uint8)",
+                   "note": "oracle timed on bounded samples of the workload (see cpu_baseline.sample)"},
+        "me": {"value": statistics.median(ms) / 1e9, "unit": "GSAD/s"},
+        "cpu_baseline": {"value": val, "unit": "GPoint-updates/s", "cores": last["cores"], "kind": "oracle",
+                         "sample": last["sample"], "me_value": statistics.median(ms) / 1e9, "me_unit": "GSAD/s"},
+        "e2e": {"value": val, "unit": "GPoint-updates/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
+    }
+    print(json.dumps(line), flush=True)
+    return 0
+
+
+# ---------------------------------------------------------------------------------------
+# our arm
+# ---------------------------------------------------------------------------------------
+def run_ours(args, rank, world, local_rank):
+    import torch
+    import torch.distributed as dist
+
+    import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
+    import sp_inputs
+
+    dev = torch.device("cuda", local_rank)
+    torch.cuda.set_device(dev)
+    stream = torch.cuda.current_stream()
+    tt = args.time_tile
+    H = sp.halo_of(tt)
+    pk = peaks()
+
+    # ---- Jacobi state: this rank's slab [x_begin, x_begin + n_local) of the global domain
+    n_local = JAC_N_LOCAL
+    n_global = n_local * world
+    x_begin = rank * n_local
+    comm = None
+    if world == 1:
+        a_host = sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED)
+        a = torch.from_numpy(a_host).to(dev)
+        work = torch.empty_like(a)
+    else:
+        lo, hi = max(0, x_begin - H), min(n_global, x_begin + n_local + H)
+        a = torch.zeros(n_local + 2 * H, dtype=torch.float32, device=dev)
+        a[lo - (x_begin - H): hi - (x_begin - H)] = torch.from_numpy(
+            sp_inputs.jacobi_input(hi - lo, seed=sp_inputs.JACOBI_BENCH_SEED, begin=lo)).to(dev)
+        work = torch.empty_like(a)
+        uid = torch.zeros(128, dtype=torch.uint8, device=dev)
+        if rank == 0:
+            uid.copy_(torch.frombuffer(bytearray(sp.get_unique_id()), dtype=torch.uint8))
+        dist.broadcast(uid, 0)
+        comm = sp.Comm(bytes(uid.cpu().numpy().tobytes()), world, rank, local_rank)
+
+    def jacobi_step():
+        if comm is None:
+            sp.jacobi1d_timetiled(a, JAC_T, tt, 0, work=work)
+        else:
+            comm.jacobi1d_timetiled_dist(a, work, n_global, x_begin, n_local, JAC_T, tt, 0)
+
+    # ---- ME batch: this rank's 64 pairs = frames [64 r, 64 r + 65) of the sequence
+    f0 = ME_PAIRS * rank
+    frames_host = np.stack([sp_inputs.me_frame(f0 + f, ME_W, ME_H, ME_R) for f in range(ME_PAIRS + 1)])
+    frames = torch.from_numpy(frames_host).to(dev)
+    mbx, mby = ME_W // 16, ME_H // 16
+    me_out = (torch.empty((ME_PAIRS, mby, mbx, 2), dtype=torch.int16, device=dev),
+              torch.empty((ME_PAIRS, mby, mbx), dtype=torch.int32, device=dev), None)
+
+    def me_step():
+        sp.me_search_sequence(frames, ME_W, ME_H, ME_R, out=me_out)
+
+    def barrier():
+        if world > 1:
+            dist.barrier()
+        torch.cuda.synchronize()
+
+    # ---- warm-up
+    for _ in range(args.warmup):
+        jacobi_step()
+        me_step()
+    barrier()
+
+    # ---- timed region: K steps, device events on the launching stream
+    K = args.steps
+    ev = [[torch.cuda.Event(enable_timing=True) for _ in range(3)] for _ in range(K)]
+    with ClockSampler(local_rank) as clk:
+        barrier()
+        e_start = torch.cuda.Event(enable_timing=True)
+        e_end = torch.cuda.Event(enable_timing=True)
+        e_start.record(stream)
+        for k in range(K):
+            ev[k][0].record(stream)
+            jacobi_step()
+            ev[k][1].record(stream)
+            me_step()
+            ev[k][2].record(stream)
+        e_end.record(stream)
+        torch.cuda.synchronize()
+        barrier()
+    total_ms = e_start.elapsed_time(e_end)
+    jac_ms = sum(ev[k][0].elapsed_time(ev[k][1]) for k in range(K))
+    me_ms = sum(ev[k][1].elapsed_time(ev[k][2]) for k in range(K))
+
+    def max_over_ranks(x):
+        if world == 1:
+            return x
+        t = torch.tensor([x], dtype=torch.float64, device=dev)
+        dist.all_reduce(t, op=dist.ReduceOp.MAX)
+        return float(t.item())
+
+    total_ms, jac_ms, me_ms = max_over_ranks(total_ms), max_over_ranks(jac_ms), max_over_ranks(me_ms)
+    updates = (n_global - 2) * JAC_T * K
+    sads = me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * world * K
+    jac_val = updates / (jac_ms * 1e-3) / 1e9
+    me_val = sads / (me_ms * 1e-3) / 1e9
+
+    # ---- per-launch kernel durations (CUDA events on the launching stream) for the roofline
+    plan = sp.jacobi1d_plan(n_local, JAC_T, tt, 0)
+    reps = 8
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    torch.cuda.synchronize()
+    e0.record(stream)
+    for _ in range(reps):
+        if comm is None:
+            sp.jacobi1d_timetiled(a, 2 * tt, tt, 0, work=work)  # 2 full-height launches
+        else:
+            comm.jacobi1d_timetiled_dist(a, work, n_global, x_begin, n_local, 2 * tt, tt, 0)
+    e1.record(stream)
+    torch.cuda.synchronize()
+    jac_launch_ms = e0.elapsed_time(e1) / (2 * reps)
+    jac_bytes = 8.0 * n_local  # algorithmic: each cell read once and written once per pass
+    jac_achieved = jac_bytes / (jac_launch_ms * 1e-3) / 1e9
+    e0.record(stream)
+    for _ in range(3):
+        me_step()
+    e1.record(stream)
+    torch.cuda.synchronize()
+    me_launch_ms = e0.elapsed_time(e1) / 3
+    me_ops = me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * 256.0
+    me_achieved = me_ops / (me_launch_ms * 1e-3) / 1e12
+    alu_peak = 148 * VABSDIFF4_PER_CLK_SM * 4 * pk["sm_max_mhz"] * 1e6 / 1e12
+    tr = traffic_from_profiles()
+    roof_jac = {"kernel": "jacobi1d_pass_kernel", "bound": "hbm", "achieved": round(jac_achieved, 1),
+                "peak": pk["hbm_gbs"], "unit": "GB/s", "frac": round(jac_achieved / pk["hbm_gbs"], 4),
+                "traffic": tr.get("jacobi1d_pass_kernel"), "peak_source": pk["source"],
+                "per_launch_ms": round(jac_launch_ms, 4), "algorithmic_bytes_per_launch": jac_bytes}
+    roof_me = {"kernel": "me_sad_kernel", "bound": "alu", "achieved": round(me_achieved, 2), "peak": round(alu_peak, 2),
+               "unit": "Tabsdiff/s", "frac": round(me_achieved / alu_peak, 4), "traffic": tr.get("me_sad_kernel"),
+               "peak_source": f"148 SM x {VABSDIFF4_PER_CLK_SM} VABSDIFF4/clk (measured) x 4 x sm_max_mhz",
+               "per_launch_ms": round(me_launch_ms, 4), "algorithmic_ops_per_launch": me_ops}
+    dominant = roof_jac if jac_ms >= me_ms else roof_me
+
+    # ---- end-to-end through the public API with host buffers (N = 1: pinned H2D/D2H in the timed region)
+    e2e = None
+    me_e2e = None
+    if world == 1:
+        a_pin = torch.from_numpy(sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED)).pin_memory()
+        f_pin = torch.from_numpy(frames_host).pin_memory()
+        for _ in range(1):
+            sp.jacobi1d(a_pin, JAC_T, tt)
+            sp.me_search(f_pin, ME_W, ME_H, ME_R)
+        torch.cuda.synchronize()
+        ke = max(1, min(K, 3))
+        tj = tm = 0.0
+        for _ in range(ke):
+            t0 = time.perf_counter()
+            sp.jacobi1d(a_pin, JAC_T, tt)
+            torch.cuda.synchronize()
+            t1 = time.perf_counter()
+            sp.me_search(f_pin, ME_W, ME_H, ME_R)
+            torch.cuda.synchronize()
+            t2 = time.perf_counter()
+            tj += t1 - t0
+            tm += t2 - t1
+        e2e = {"value": (n_local - 2) * JAC_T * ke / tj / 1e9, "unit": "GPoint-updates/s",
+               "h2d_bytes_per_step": 4 * n_local + frames_host.nbytes,
+               "d2h_bytes_per_step": 4 * n_local + ME_PAIRS * mby * mbx * (4 + 4)}
+        me_e2e = {"value": me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * ke / tm / 1e9, "unit": "GSAD/s",
+                  "h2d_bytes_per_step": frames_host.nbytes, "d2h_bytes_per_step": ME_PAIRS * mby * mbx * 8}
+
+    # ---- CPU baseline: the oracle on a bounded sample (rank 0, N = 1 only)
+    cpu = None
+    if world == 1 and not args.no_cpu_baseline:
+        s = oracle_samples()
+        cpu = {"value": s["jacobi_ups"] / 1e9, "unit": "GPoint-updates/s", "cores": s["cores"], "kind": "oracle",
+               "sample": s["sample"], "me_value": s["me_sads"] / 1e9, "me_unit": "GSAD/s"}
+
+    launches_per_step = plan["passes"] + 1  # Jacobi passes + one ME launch
+    line = {
+        "metric": METRIC, "value": round(jac_val, 2), "unit": "GPoint-updates/s", "n_gpus": world, "steps": K,
+        "warmup": args.warmup, "ms_per_step": round(total_ms / K, 4), "higher_is_better": True, "scaling": "weak",
+        "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
+        "config": {"workload": f"J3: Jacobi fp32 N=2^26 cells/GPU, T={JAC_T}, time tile {tt} (halo {H}) + "
+                               f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs/GPU",
+                   "jacobi_global_n": n_global, "time_tile": tt, "space_tile": plan["space_tile"],
+                   "me_pairs_global": ME_PAIRS * world,
+                   "l2": "inputs larger than L2 (256 MiB Jacobi state per GPU, 135 MB frame batch); no flush",
+                   "parallelism": f"weak scaling over {world} GPU(s); Jacobi halo exchange per time tile"},
+        "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4)},
+        "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
+               "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},
+        "roofline": dominant, "roofline_jacobi": roof_jac,
+        "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches_per_step * K, "clocks": clk.summary(),
+    }
+    if rank == 0:
+        print(json.dumps(line), flush=True)
+    if comm is not None:
+        comm.destroy()
+    return 0
+
+
+def main():
+    ap = argparse.ArgumentParser()
+    ap.add_argument("--gpus", type=int, default=1)
+    ap.add_argument("--steps", type=int, default=10)
+    ap.add_argument("--warmup", type=int, default=3)
+    ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
+    ap.add_argument("--time-tile", type=int, default=32)
+    ap.add_argument("--no-cpu-baseline", action="store_true")
+    args = ap.parse_args()
+    world = int(os.environ.get("WORLD_SIZE", "1"))
+    rank = int(os.environ.get("RANK", "0"))
+    local_rank = int(os.environ.get("LOCAL_RANK", "0"))
+    if args.impl == "reference":
+        return run_reference(args, rank, world)
+    if world > 1:
+        import torch
+        import torch.distributed as dist
+        torch.cuda.set_device(local_rank)
+        dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
+    try:
+        return run_ours(args, rank, world, local_rank)
+    finally:
+        if world > 1:
+            import torch.distributed as dist
+            dist.destroy_process_group()
+
+
+if __name__ == "__main__":
+    sys.exit(main())

@@ -1,0 +1,266 @@
+/*
+ * sp.h — C ABI of libsp, a B200-native (sm_100a) implementation of the data-parallel
+ * hot path of Baskaran, Bondhugula, Krishnamoorthy, Ramanujam, Rountev, Sadayappan,
+ * "Automatic Data Movement and Computation Mapping for Multi-level Parallel
+ * Architectures with Explicitly Managed Memories", PPoPP'08.
+ *
+ * Citations "P:Lx-y" are lines of the paper text; "R-xx" are the readings of
+ * garbled or silent passages listed in DESIGN.md.
+ *
+ * Conventions (every entry point):
+ *   - plain C types only; every integer is fixed width; no exception crosses the ABI;
+ *   - the return value is a status code (SP_OK or a negative SP_ERR_*);
+ *   - the caller owns every array and stream; the library never frees caller memory,
+ *     keeps no pointer after return, and makes no device allocation on a hot path;
+ *   - `stream` arguments are cudaStream_t passed as void* (NULL = legacy default stream);
+ *     device entry points are stream-ordered and asynchronous: argument and launch
+ *     errors are returned immediately, device faults surface at the caller's next sync;
+ *   - there is no CPU fallback: on a machine without a usable sm_100 device the device
+ *     entry points return SP_ERR_CUDA.
+ */
+#ifndef SP_H_
+#define SP_H_
+
+#include <stdint.h>
+
+#ifdef __cplusplus
+extern "C" {
+#endif
+
+#define SP_OK 0
+#define SP_ERR_INVALID_ARG -1 /* bad sizes, null required pointer, misalignment */
+#define SP_ERR_UNBOUNDED -2   /* planner: a statement domain is unbounded */
+#define SP_ERR_CAPACITY -3    /* caller output array too small; required count written back */
+#define SP_ERR_OVERFLOW -4    /* int64 overflow in bounds / sizes / coefficients */
+#define SP_ERR_UNSUPPORTED -5 /* outside the supported envelope (see each function) */
+#define SP_ERR_SMEM_LIMIT -6  /* planner: total staged size exceeds opts->mup_elems */
+#define SP_ERR_CUDA -7        /* CUDA error; sp_last_cuda_error() gives the cudaError_t */
+#define SP_ERR_NCCL -8        /* NCCL error; sp_last_nccl_error() gives the ncclResult_t */
+
+/* Human-readable name of a status code (static storage). */
+const char* sp_status_string(int status);
+/* cudaError_t / ncclResult_t of the last failing call on this host thread (0 if none). */
+int sp_last_cuda_error(void);
+int sp_last_nccl_error(void);
+/* Library version, major*10000 + minor*100 + patch. */
+int sp_version(void);
+
+/* =====================================================================================
+ * 1. Planner — the paper's data-management framework for one program block
+ *    ("takes as input the iteration spaces of all statements in a program
+ *    block as well as the access functions of all array references"; §3.1, Alg. 1,
+ *    Alg. 2, §3.1.2, §3.1.3).  Host-only, pure, thread-safe, synchronous.
+ * ===================================================================================== */
+#define SP_MAX_RANK 8  /* max array dimensionality */
+#define SP_MAX_DEPTH 8 /* max loop depth of a statement */
+#define SP_MAX_PARAMS 8
+
+/* Iteration-space polytope of a statement (§2): every integer vector i with
+ * row . (i, p, 1) >= 0 for each of the n_rows rows; `rows` is row-major
+ * [n_rows][depth + n_params + 1].  The domain must be bounded (else SP_ERR_UNBOUNDED). */
+typedef struct {
+    int32_t depth;
+    int32_t n_rows;
+    const int64_t* rows;
+} sp_domain;
+
+/* Affine array reference A[F . (i, p, 1)] (§2): `rows` is row-major
+ * [rank][depth_of_stmt + n_params + 1]; subscript k = rows[k] . (i, p, 1).
+ * `array` is a caller-chosen array id; every reference to one array has the same rank. */
+typedef struct {
+    int32_t stmt;
+    int32_t array;
+    int32_t is_write;
+    int32_t rank;
+    const int64_t* rows;
+} sp_ref;
+
+typedef struct {
+    int32_t n_params;
+    int32_t n_stmts;
+    int32_t n_refs;
+    int32_t reserved;       /* must be 0 */
+    const int64_t* params;  /* [n_params] concrete parameter values */
+    const sp_domain* stmts; /* [n_stmts] */
+    const sp_ref* refs;     /* [n_refs] */
+} sp_block;
+
+enum {
+    SP_PLAN_PER_ARRAY = 0,  /* one buffer per array: the bounding box of all its data
+                               spaces — what Figure 1 prints (reading R-P1) */
+    SP_PLAN_COMPONENTS = 1  /* one buffer per connected component of the overlap graph
+                               (Alg. 2 step 5) */
+};
+
+typedef struct {
+    int32_t mode;          /* SP_PLAN_PER_ARRAY or SP_PLAN_COMPONENTS */
+    int32_t reuse_filter;  /* 1: stage only partitions Alg. 1 marks beneficial (GPU rule,
+                              P:L349-351); refs of other partitions map to -1 */
+    double delta;          /* Alg. 1 constant-reuse threshold, 0.30 in the paper */
+    int64_t mup_elems;     /* M_up in elements; 0 = unlimited.  If the staged
+                              buffers' total size exceeds it: SP_ERR_SMEM_LIMIT */
+    int64_t max_points;    /* enumeration budget (integer points over all statements);
+                              0 = default 2^27; exceeding it: SP_ERR_UNSUPPORTED */
+} sp_plan_opts;
+
+/* One local-memory buffer = one partition of an array's data spaces (Alg. 2 output). */
+typedef struct {
+    int32_t array;       /* array id */
+    int32_t rank;        /* dimensionality n of the local array (= that of the global
+                            array: every dimension is kept, reading R-P5) */
+    int32_t beneficial;  /* Alg. 1 verdict */
+    int32_t n_refs;      /* references in the partition */
+    int64_t lb[SP_MAX_RANK]; /* lower bound per dimension = offset g */
+    int64_t ub[SP_MAX_RANK]; /* upper bound per dimension; empty buffer: lb = 0, ub = -1 */
+    int64_t size;            /* prod (ub_k - lb_k + 1) elements */
+    int64_t v_in_ub;         /* upper bound on the move-in volume */
+    int64_t v_out_ub;        /* upper bound on the move-out volume */
+    int64_t in_lb[SP_MAX_RANK], in_ub[SP_MAX_RANK]; /* bbox of the move-in set = union of
+                                                       read data spaces */
+    int64_t in_count;        /* |union of read data spaces| (0: nothing to move in) */
+    int64_t out_lb[SP_MAX_RANK], out_ub[SP_MAX_RANK]; /* bbox of the move-out set */
+    int64_t out_count;       /* |union of write data spaces| */
+    int32_t in_dense;        /* in_count == volume of the in bbox (a box copy is exact) */
+    int32_t out_dense;       /* out_count == volume of the out bbox */
+    int64_t overlap;         /* sum over reference pairs of |D_r ∩ D_r'| (Alg. 1 line 7) */
+    int64_t union_count;     /* |union of the partition's data spaces| */
+} sp_buffer;
+
+/* Plan the local buffers of one program block.
+ *   bufs[cap_bufs]  : output buffers ordered by (array id, smallest ref index in the
+ *                     partition).  If more than cap_bufs are needed, *n_bufs receives the
+ *                     required count and SP_ERR_CAPACITY is returned (nothing else written).
+ *   ref_buf[n_refs] : buffer index of each reference, -1 if not staged (nullable).
+ *   local_rows      : sum over refs of rank x (depth + n_params + 1) int64, in ref order:
+ *                     the local access function F' - g; unchanged F for
+ *                     unstaged refs (nullable).
+ * Empty statement domains are not errors: they yield empty (size-0) data spaces. */
+int sp_plan_buffers(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, int32_t cap_bufs,
+                    int32_t* n_bufs, int32_t* ref_buf, int64_t* local_rows);
+
+/* =====================================================================================
+ * 2. Time-tiled 1-D Jacobi
+ *
+ *   for t in [0, steps): for i in [1, n-2]: a'[i] = ((a[i-1] + a[i]) + a[i+1]) * w
+ *   w = fl32(1/3), every operation rounded to nearest fp32, no contraction; a[0] and
+ *   a[n-1] are fixed (reading R-J1).
+ *
+ * Execution: passes of h = min(time_tile, remaining) steps
+ * (overlapped "concurrent start" tiling, R-J4); a pass splits [0, n) into space tiles of
+ * S cells; a CTA stages each tile's footprint [max(0,x0-H), min(n-1,x0+S-1+H)], H = the
+ * time tile rounded up to a multiple of 4, into shared memory (TMA bulk copy), runs the h
+ * steps in registers (warp shuffles), and writes back only its owned cells
+ * [x0, min(n-1, x0+S-1)] (R-J5).  The kernel boundary is the inter-pass barrier.
+ * ===================================================================================== */
+typedef struct {
+    int64_t n;
+    int32_t steps;
+    int32_t time_tile;   /* Tt: steps per pass */
+    int32_t halo;        /* H: halo cells per side actually staged (Tt rounded up to 4) */
+    int32_t passes;      /* ceil(steps / Tt) */
+    int64_t space_tile;  /* S: owned cells per tile */
+    int64_t tiles;       /* tiles per pass = ceil(n / S) */
+    int32_t grid;        /* CTAs per launch (persistent) */
+    int32_t threads;     /* threads per CTA */
+    int32_t smem_bytes;  /* dynamic shared memory per CTA */
+    int32_t cells_per_thread; /* register cells per thread */
+} sp_jacobi_plan;
+
+/* Geometry the library will use (host-only).  space_tile = 0 selects the default
+ * (largest) tile; otherwise it must be a multiple of 4 not above the default.
+ * time_tile in [1, 128].  Errors: SP_ERR_INVALID_ARG. */
+int sp_jacobi1d_plan(int64_t n, int32_t steps, int32_t time_tile, int32_t space_tile, sp_jacobi_plan* out);
+
+/* Closed-form footprint of tile (x0, S) in a pass of height h: the Alg. 2 bounding box of
+ * the tile's reads of `a`: [max(0, x0-h), min(n-1, x0+S-1+h)]. */
+int sp_jacobi1d_tile_footprint(int64_t n, int32_t h, int64_t x0, int64_t space_tile, int64_t* lb, int64_t* ub);
+
+/* Run `steps` steps on device array a[n] (16-byte aligned), using work[n] (16-byte
+ * aligned, contents clobbered) as the ping-pong buffer.  On completion a holds a^(steps).
+ * n >= 3; steps >= 0 (0 = identity); time_tile in [1, 128]; space_tile 0 or as above.
+ * footprint_log (nullable, device int64): [passes][tiles][2] = (lb, ub) of each tile's
+ * staged footprint as the kernel computed it (for checking against the planner). */
+int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32_t time_tile,
+                          int32_t space_tile, int64_t* footprint_log, void* stream);
+
+/* Segment form (building block of the multi-GPU layer and of its single-GPU loopback
+ * test): one pass of height h over a window of the global domain.
+ *   src/dst : device arrays holding global cells [g0, g0 + len); dst receives the new
+ *             values of the owned cells [own_begin, own_end) only (global indices), which
+ *             must satisfy g0 + H <= own_begin (or own_begin == 0 ... cells < 0 do not
+ *             exist) and own_end + H <= g0 + len (or own_end == n_global); H is the halo
+ *             for time_tile (= h rounded up to 4).  Global cells 0 and n_global-1 are fixed.
+ *   g0 and own_begin must be multiples of 4 (16-byte aligned TMA copies). */
+int sp_jacobi1d_pass_segment(const float* src, float* dst, int64_t n_global, int64_t g0, int64_t len,
+                             int64_t own_begin, int64_t own_end, int32_t h, int32_t time_tile,
+                             int32_t space_tile, void* stream);
+
+/* =====================================================================================
+ * 3. Full-search motion estimation (Fig. 2 with WS = 16)
+ *
+ * Macroblocks (bx, by), x0 = 16 bx, y0 = 16 by, bx < floor(width/16); candidates
+ * (dx, dy) in [-R, R]^2 valid iff the displaced block lies inside the frame
+ * (R-M3); SAD(dx,dy) = sum_{v,u<16} |cur[y0+v][x0+u] - ref[y0+dy+v][x0+dx+u]| (R-M1);
+ * best = lexicographic min of (SAD, |dx|+|dy|, dy, dx) over valid candidates (R-M4).
+ *
+ * Buffers: ref/cur hold rows [row0_global, row0_global + rows_in_buffer) of frames of
+ * `frame_height` rows, row pitch `pitch` bytes (multiple of 16), base 16-byte aligned;
+ * pair p is at ref + p*pair_stride and cur + p*pair_stride (pair_stride multiple of 16).
+ * The band must contain every row a valid candidate of MB rows [mb_row_begin,
+ * mb_row_end) reads: [16*mb_row_begin - R, 16*mb_row_end + R) ∩ [0, frame_height).
+ * Outputs (device), for pair p, MB row r (relative to mb_row_begin), bx:
+ *   mv[((p*rows + r)*mbx + bx)*2 + {0,1}] = (dx, dy)      int16
+ *   best_sad[(p*rows + r)*mbx + bx]                        uint32
+ *   surface (nullable) [...][(2R+1)^2], entry (dy+R)(2R+1) + (dx+R), 0xFFFFFFFF if invalid
+ * block must be 16 (SP_ERR_UNSUPPORTED otherwise); 0 <= range <= 63.
+ * ===================================================================================== */
+int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                     int32_t rows_in_buffer, int32_t row0_global, int32_t frame_height, int32_t n_pairs,
+                     int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
+                     int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream);
+
+/* Reference window the ME kernel stages for macroblock (bx, by): the Alg. 2 bounding box
+ * of ref[y0+dy+v][x0+dx+u] over valid candidates, = [y0-R, y0+15+R] x [x0-R, x0+15+R]
+ * clipped to the frame (lb/ub as (row, col)).  Host-only. */
+int sp_me_ref_window(int32_t width, int32_t frame_height, int32_t range, int32_t bx, int32_t by,
+                     int64_t lb[2], int64_t ub[2]);
+
+/* =====================================================================================
+ * 4. Multi-GPU layer (one process per GPU, NCCL over NVLink / NVSwitch)
+ * Jacobi is partitioned spatially with a halo of depth H exchanged once per time tile;
+ * ME is partitioned by macroblock rows with R-row reference halos (no exchange during
+ * the search; results are all-gathered).
+ * ===================================================================================== */
+typedef struct sp_comm sp_comm;
+
+/* NCCL unique id of the job (rank 0 creates it and broadcasts the 128 bytes). */
+int sp_get_unique_id(uint8_t out_id[128]);
+/* Collective: create the communicator on `device` (cudaSetDevice is called). */
+int sp_comm_init(sp_comm** out, const uint8_t id[128], int32_t nranks, int32_t rank, int32_t device);
+int sp_comm_destroy(sp_comm* c);
+
+/* Distributed time-tiled Jacobi over contiguous slabs.  Rank r owns global cells
+ * [x_begin, x_begin + n_local); a_local/work_local hold [x_begin - H, x_begin + n_local + H)
+ * (H = halo of time_tile; cells outside [0, n_global) unused), 16-byte aligned, x_begin a
+ * multiple of 4.  Per pass the ranks exchange H halo cells with each neighbour (grouped
+ * ncclSend/ncclRecv on `stream`), then run sp_jacobi1d_pass_segment.  On return a_local
+ * holds the rank's slab of a^(steps) (and its halos are stale). */
+int sp_jacobi1d_timetiled_dist(sp_comm* c, float* a_local, float* work_local, int64_t n_global,
+                               int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
+                               int32_t space_tile, void* stream);
+
+/* Single-GPU loopback transport of the same partitioned pass loop: nranks virtual slabs
+ * on the current device (slab r owns [x_begins[r], x_begins[r] + n_locals[r]), slabs tile
+ * [0, n_global) in order, each n_local >= H), halos moved with cudaMemcpyAsync instead of
+ * NCCL.  Test vehicle for the decomposition on a one-GPU box; layouts as above. */
+int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_locals, int32_t nranks, int64_t n_global,
+                                   const int64_t* x_begins, const int64_t* n_locals, int32_t steps,
+                                   int32_t time_tile, int32_t space_tile, void* stream);
+
+/* ncclAllGather of `bytes` per rank (device buffers) — used for the ME results. */
+int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream);
+
+#ifdef __cplusplus
+}
+#endif
+#endif /* SP_H_ */

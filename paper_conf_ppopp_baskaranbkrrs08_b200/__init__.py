@@ -1,0 +1,373 @@
+"""Python binding of libsp (include/sp.h) — argument marshalling only.
+
+B200-native (sm_100a) implementation of the data-parallel hot path of Baskaran et al.,
+"Automatic Data Movement and Computation Mapping for Multi-level Parallel Architectures
+with Explicitly Managed Memories", PPoPP'08: staged multi-level-tiled execution of the
+paper's two GPU workloads (time-tiled 1-D Jacobi, MPEG-4 full-search SAD motion
+estimation) plus the paper's buffer planner (Alg. 1 / Alg. 2 / §3.1.2-3.1.3).
+
+Every step of the path runs in libsp.so (CUDA kernels + C++ host code); this module only
+converts arguments.  PyTorch supplies device memory, streams and process groups.  There is
+no CPU fallback: importing this package without the built library raises ImportError, and
+the device entry points raise SPError when no usable device is present.
+
+C entry point -> Python name (same names, `sp_` prefix dropped):
+  sp_plan_buffers             -> plan_buffers(block, ...)
+  sp_jacobi1d_plan            -> jacobi1d_plan(n, steps, time_tile, space_tile)
+  sp_jacobi1d_tile_footprint  -> jacobi1d_tile_footprint(n, h, x0, space_tile)
+  sp_jacobi1d_timetiled       -> jacobi1d_timetiled(a, steps, ...)     (device tensor, in place)
+  sp_jacobi1d_pass_segment    -> jacobi1d_pass_segment(...)
+  sp_jacobi1d_timetiled_loopback -> jacobi1d_timetiled_loopback(...)
+  sp_jacobi1d_timetiled_dist  -> Comm.jacobi1d_timetiled_dist(...)
+  sp_me_sad_search            -> me_sad_search(ref, cur, ...)          (device tensors)
+  sp_me_ref_window            -> me_ref_window(...)
+  sp_get_unique_id / sp_comm_init / sp_comm_destroy / sp_allgather -> Comm
+Host-buffer convenience (the end-to-end public API used for bench.py's `e2e`):
+  jacobi1d(host_array, steps, ...), me_search(host_frames, ...)
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+import numpy as np
+
+__all__ = [
+    "SPError", "lib", "plan_buffers", "jacobi1d_plan", "jacobi1d_tile_footprint", "jacobi1d_timetiled",
+    "jacobi1d_pass_segment", "jacobi1d_timetiled_loopback", "me_sad_search", "me_ref_window", "me_search_sequence",
+    "jacobi1d", "me_search", "Comm", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
+]
+
+_HERE = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_HERE, "libsp.so")
+
+PER_ARRAY = 0
+COMPONENTS = 1
+MAX_RANK = 8
+
+i32, i64, f64 = ctypes.c_int32, ctypes.c_int64, ctypes.c_double
+vp = ctypes.c_void_p
+
+
+class sp_domain(ctypes.Structure):
+    _fields_ = [("depth", i32), ("n_rows", i32), ("rows", ctypes.POINTER(i64))]
+
+
+class sp_ref(ctypes.Structure):
+    _fields_ = [("stmt", i32), ("array", i32), ("is_write", i32), ("rank", i32), ("rows", ctypes.POINTER(i64))]
+
+
+class sp_block(ctypes.Structure):
+    _fields_ = [("n_params", i32), ("n_stmts", i32), ("n_refs", i32), ("reserved", i32),
+                ("params", ctypes.POINTER(i64)), ("stmts", ctypes.POINTER(sp_domain)), ("refs", ctypes.POINTER(sp_ref))]
+
+
+class sp_plan_opts(ctypes.Structure):
+    _fields_ = [("mode", i32), ("reuse_filter", i32), ("delta", f64), ("mup_elems", i64), ("max_points", i64)]
+
+
+class sp_buffer(ctypes.Structure):
+    _fields_ = [("array", i32), ("rank", i32), ("beneficial", i32), ("n_refs", i32),
+                ("lb", i64 * MAX_RANK), ("ub", i64 * MAX_RANK), ("size", i64), ("v_in_ub", i64), ("v_out_ub", i64),
+                ("in_lb", i64 * MAX_RANK), ("in_ub", i64 * MAX_RANK), ("in_count", i64),
+                ("out_lb", i64 * MAX_RANK), ("out_ub", i64 * MAX_RANK), ("out_count", i64),
+                ("in_dense", i32), ("out_dense", i32), ("overlap", i64), ("union_count", i64)]
+
+
+class sp_jacobi_plan(ctypes.Structure):
+    _fields_ = [("n", i64), ("steps", i32), ("time_tile", i32), ("halo", i32), ("passes", i32), ("space_tile", i64),
+                ("tiles", i64), ("grid", i32), ("threads", i32), ("smem_bytes", i32), ("cells_per_thread", i32)]
+
+
+SYMBOLS = {
+    "sp_status_string": (ctypes.c_char_p, [ctypes.c_int]),
+    "sp_last_cuda_error": (ctypes.c_int, []),
+    "sp_last_nccl_error": (ctypes.c_int, []),
+    "sp_version": (ctypes.c_int, []),
+    "sp_plan_buffers": (ctypes.c_int, [ctypes.POINTER(sp_block), ctypes.POINTER(sp_plan_opts), ctypes.POINTER(sp_buffer),
+                                       i32, ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(i64)]),
+    "sp_jacobi1d_plan": (ctypes.c_int, [i64, i32, i32, i32, ctypes.POINTER(sp_jacobi_plan)]),
+    "sp_jacobi1d_tile_footprint": (ctypes.c_int, [i64, i32, i64, i64, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
+    "sp_jacobi1d_timetiled": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, vp, vp]),
+    "sp_jacobi1d_pass_segment": (ctypes.c_int, [vp, vp, i64, i64, i64, i64, i64, i32, i32, i32, vp]),
+    "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
+    "sp_me_ref_window": (ctypes.c_int, [i32, i32, i32, i32, i32, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
+    "sp_get_unique_id": (ctypes.c_int, [ctypes.POINTER(ctypes.c_uint8)]),
+    "sp_comm_init": (ctypes.c_int, [ctypes.POINTER(vp), ctypes.POINTER(ctypes.c_uint8), i32, i32, i32]),
+    "sp_comm_destroy": (ctypes.c_int, [vp]),
+    "sp_jacobi1d_timetiled_dist": (ctypes.c_int, [vp, vp, vp, i64, i64, i64, i32, i32, i32, vp]),
+    "sp_jacobi1d_timetiled_loopback": (ctypes.c_int, [ctypes.POINTER(vp), ctypes.POINTER(vp), i32, i64,
+                                                      ctypes.POINTER(i64), ctypes.POINTER(i64), i32, i32, i32, vp]),
+    "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
+}
+
+
+def _load():
+    if not os.path.exists(LIB_PATH):
+        raise ImportError(f"libsp.so is not built ({LIB_PATH}); run `python -c 'import __graft_entry__ as g; g.build()'`."
+                          " There is no CPU fallback.")
+    L = ctypes.CDLL(LIB_PATH)
+    for name, (res, args) in SYMBOLS.items():
+        fn = getattr(L, name)
+        fn.restype = res
+        fn.argtypes = args
+    return L
+
+
+lib = _load()
+
+
+class SPError(RuntimeError):
+    def __init__(self, status: int, where: str):
+        self.status = status
+        name = lib.sp_status_string(status).decode()
+        extra = ""
+        if name == "SP_ERR_CUDA":
+            extra = f" (cudaError {lib.sp_last_cuda_error()})"
+        elif name == "SP_ERR_NCCL":
+            extra = f" (ncclResult {lib.sp_last_nccl_error()})"
+        super().__init__(f"{where}: {name}{extra}")
+
+
+def _check(status: int, where: str) -> None:
+    if status != 0:
+        raise SPError(status, where)
+
+
+def _stream(stream):
+    import torch
+    if stream is None:
+        return vp(torch.cuda.current_stream().cuda_stream)
+    if isinstance(stream, int):
+        return vp(stream)
+    return vp(stream.cuda_stream)
+
+
+def _ptr(t):
+    return vp(t.data_ptr()) if t is not None else None
+
+
+def halo_of(time_tile: int) -> int:
+    return (int(time_tile) + 3) & ~3
+
+
+# ---------------------------------------------------------------------------------------
+# Planner
+# ---------------------------------------------------------------------------------------
+def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_filter: bool = False,
+                 mup_elems: int = 0, max_points: int = 0, cap: int = 64) -> dict:
+    """sp_plan_buffers on a block given as {"params": [...], "stmts": [{"depth", "rows"}],
+    "refs": [{"stmt", "array", "is_write", "rank", "rows"}]} (extra keys ignored)."""
+    params = [int(p) for p in block.get("params", [])]
+    P = len(params)
+    keep = []
+    doms = (sp_domain * max(1, len(block["stmts"])))()
+    for k, s in enumerate(block["stmts"]):
+        d = int(s["depth"])
+        rows = np.ascontiguousarray(np.asarray(s["rows"], dtype=np.int64).reshape(-1, d + P + 1))
+        keep.append(rows)
+        doms[k] = sp_domain(d, rows.shape[0], rows.ctypes.data_as(ctypes.POINTER(i64)))
+    refs = (sp_ref * max(1, len(block["refs"])))()
+    for k, r in enumerate(block["refs"]):
+        rows = np.ascontiguousarray(np.asarray(r["rows"], dtype=np.int64))
+        keep.append(rows)
+        refs[k] = sp_ref(int(r["stmt"]), int(r["array"]), int(bool(r["is_write"])), int(r["rank"]),
+                         rows.ctypes.data_as(ctypes.POINTER(i64)))
+    par = np.ascontiguousarray(np.asarray(params if params else [0], dtype=np.int64))
+    blk = sp_block(P, len(block["stmts"]), len(block["refs"]), 0, par.ctypes.data_as(ctypes.POINTER(i64)), doms, refs)
+    opts = sp_plan_opts(int(mode), int(bool(reuse_filter)), float(delta), int(mup_elems), int(max_points))
+    n_refs = len(block["refs"])
+    ref_buf = (i32 * max(1, n_refs))()
+    width = sum(int(r["rank"]) * (int(block["stmts"][int(r["stmt"])]["depth"]) + P + 1) for r in block["refs"])
+    local = (i64 * max(1, width))()
+    n = i32(0)
+    while True:
+        bufs = (sp_buffer * cap)()
+        st = lib.sp_plan_buffers(ctypes.byref(blk), ctypes.byref(opts), bufs, cap, ctypes.byref(n), ref_buf, local)
+        if st == -3 and n.value > cap:  # SP_ERR_CAPACITY: retry with the required count
+            cap = n.value
+            continue
+        break
+    out = {"status": st, "buffers": [], "ref_buf": [], "local_rows": []}
+    if st not in (0, -6):
+        return out
+    for b in bufs[: n.value]:
+        rk = b.rank
+        out["buffers"].append({
+            "array": b.array, "rank": rk, "beneficial": b.beneficial, "n_refs": b.n_refs,
+            "lb": list(b.lb[:rk]), "ub": list(b.ub[:rk]), "size": b.size, "v_in_ub": b.v_in_ub, "v_out_ub": b.v_out_ub,
+            "in_lb": list(b.in_lb[:rk]), "in_ub": list(b.in_ub[:rk]), "in_count": b.in_count, "in_dense": b.in_dense,
+            "out_lb": list(b.out_lb[:rk]), "out_ub": list(b.out_ub[:rk]), "out_count": b.out_count,
+            "out_dense": b.out_dense, "overlap": b.overlap, "union_count": b.union_count,
+        })
+    if st != 0:
+        return out
+    out["ref_buf"] = list(ref_buf[:n_refs])
+    pos = 0
+    for r in block["refs"]:
+        w = int(block["stmts"][int(r["stmt"])]["depth"]) + P + 1
+        rk = int(r["rank"])
+        out["local_rows"].append([list(local[pos + k * w: pos + (k + 1) * w]) for k in range(rk)])
+        pos += rk * w
+    return out
+
+
+# ---------------------------------------------------------------------------------------
+# Jacobi
+# ---------------------------------------------------------------------------------------
+def jacobi1d_plan(n: int, steps: int, time_tile: int = 16, space_tile: int = 0) -> dict:
+    p = sp_jacobi_plan()
+    _check(lib.sp_jacobi1d_plan(int(n), int(steps), int(time_tile), int(space_tile), ctypes.byref(p)), "sp_jacobi1d_plan")
+    return {f: getattr(p, f) for f, _ in sp_jacobi_plan._fields_}
+
+
+def jacobi1d_tile_footprint(n: int, h: int, x0: int, space_tile: int) -> tuple[int, int]:
+    lb, ub = i64(), i64()
+    _check(lib.sp_jacobi1d_tile_footprint(int(n), int(h), int(x0), int(space_tile), ctypes.byref(lb), ctypes.byref(ub)),
+           "sp_jacobi1d_tile_footprint")
+    return lb.value, ub.value
+
+
+def jacobi1d_timetiled(a, steps: int, time_tile: int = 16, space_tile: int = 0, work=None, footprint_log=None,
+                       stream=None):
+    """In place on a CUDA float32 tensor a[n]; work (same shape) is allocated if None."""
+    import torch
+    assert a.is_cuda and a.dtype == torch.float32 and a.is_contiguous()
+    if work is None:
+        work = torch.empty_like(a)
+    _check(lib.sp_jacobi1d_timetiled(_ptr(a), _ptr(work), a.numel(), int(steps), int(time_tile), int(space_tile),
+                                     _ptr(footprint_log), _stream(stream)), "sp_jacobi1d_timetiled")
+    return a
+
+
+def jacobi1d_pass_segment(src, dst, n_global: int, g0: int, own_begin: int, own_end: int, h: int, time_tile: int,
+                          space_tile: int = 0, stream=None):
+    _check(lib.sp_jacobi1d_pass_segment(_ptr(src), _ptr(dst), int(n_global), int(g0), src.numel(), int(own_begin),
+                                        int(own_end), int(h), int(time_tile), int(space_tile), _stream(stream)),
+           "sp_jacobi1d_pass_segment")
+
+
+def jacobi1d_timetiled_loopback(a_locals, work_locals, n_global: int, x_begins, n_locals, steps: int,
+                                time_tile: int = 16, space_tile: int = 0, stream=None):
+    k = len(a_locals)
+    A = (vp * k)(*[t.data_ptr() for t in a_locals])
+    Wk = (vp * k)(*[t.data_ptr() for t in work_locals])
+    xb = (i64 * k)(*[int(v) for v in x_begins])
+    nl = (i64 * k)(*[int(v) for v in n_locals])
+    _check(lib.sp_jacobi1d_timetiled_loopback(A, Wk, k, int(n_global), xb, nl, int(steps), int(time_tile),
+                                              int(space_tile), _stream(stream)), "sp_jacobi1d_timetiled_loopback")
+
+
+def jacobi1d(a_host, steps: int, time_tile: int = 16, space_tile: int = 0, device="cuda"):
+    """End-to-end public call on a host array: H2D copy, time-tiled run, D2H copy.
+    Accepts a numpy array or a (preferably pinned) CPU torch tensor; returns a CPU tensor."""
+    import torch
+    h = torch.from_numpy(np.ascontiguousarray(a_host, dtype=np.float32)) if isinstance(a_host, np.ndarray) else a_host
+    d = h.to(device, non_blocking=True)
+    jacobi1d_timetiled(d, steps, time_tile, space_tile)
+    out = torch.empty(h.shape, dtype=torch.float32, pin_memory=h.is_pinned())
+    out.copy_(d, non_blocking=False)
+    return out
+
+
+# ---------------------------------------------------------------------------------------
+# Motion estimation
+# ---------------------------------------------------------------------------------------
+def me_ref_window(width: int, frame_height: int, search_range: int, bx: int, by: int):
+    lb, ub = (i64 * 2)(), (i64 * 2)()
+    _check(lib.sp_me_ref_window(int(width), int(frame_height), int(search_range), int(bx), int(by), lb, ub),
+           "sp_me_ref_window")
+    return (lb[0], lb[1]), (ub[0], ub[1])
+
+
+def me_sad_search(ref, cur, width: int, frame_height: int, search_range: int, *, row0: int = 0,
+                  mb_row_begin: int = 0, mb_row_end: int | None = None, with_surface: bool = False,
+                  out=None, stream=None):
+    """ref, cur: CUDA uint8 tensors [n_pairs, rows_in_buffer, pitch] (views allowed, e.g.
+    seq[0:64] and seq[1:65]); returns (mv [P, rows, mbx, 2] int16, sad [P, rows, mbx] uint32
+    as int32 bits, surface or None)."""
+    import torch
+    assert ref.is_cuda and cur.is_cuda and ref.dtype == torch.uint8 and cur.dtype == torch.uint8
+    assert ref.dim() == 3 and ref.shape == cur.shape and ref.stride() == cur.stride() and ref.stride(2) == 1
+    n_pairs, rows_in_buffer, _ = ref.shape
+    pitch = ref.stride(1)
+    pair_stride = ref.stride(0) if n_pairs > 1 else pitch * rows_in_buffer
+    mbx = width // 16
+    if mb_row_end is None:
+        mb_row_end = frame_height // 16
+    rows = mb_row_end - mb_row_begin
+    side = 2 * search_range + 1
+    if out is None:
+        mv = torch.empty((n_pairs, rows, mbx, 2), dtype=torch.int16, device=ref.device)
+        sad = torch.empty((n_pairs, rows, mbx), dtype=torch.int32, device=ref.device)
+        surf = torch.empty((n_pairs, rows, mbx, side * side), dtype=torch.int32, device=ref.device) if with_surface else None
+    else:
+        mv, sad, surf = out
+    _check(lib.sp_me_sad_search(_ptr(ref), _ptr(cur), pitch, int(width), int(rows_in_buffer), int(row0),
+                                int(frame_height), int(n_pairs), int(pair_stride), 16, int(search_range),
+                                int(mb_row_begin), int(mb_row_end), _ptr(mv), _ptr(sad), _ptr(surf), _stream(stream)),
+           "sp_me_sad_search")
+    return mv, sad, surf
+
+
+def me_search_sequence(frames, width: int, frame_height: int, search_range: int, **kw):
+    """Pairs (ref = frame p, cur = frame p+1) of a CUDA uint8 sequence [F, H, pitch]."""
+    return me_sad_search(frames[:-1], frames[1:], width, frame_height, search_range, **kw)
+
+
+def me_search(frames_host, width: int, frame_height: int, search_range: int, device="cuda"):
+    """End-to-end public call on a host frame sequence [F, H, pitch] (numpy or pinned
+    tensor): H2D copy, search of the F-1 consecutive pairs, D2H copy of MV and SAD."""
+    import torch
+    h = torch.from_numpy(np.ascontiguousarray(frames_host)) if isinstance(frames_host, np.ndarray) else frames_host
+    d = h.to(device, non_blocking=True)
+    mv, sad, _ = me_search_sequence(d, width, frame_height, search_range)
+    return mv.cpu(), sad.cpu()
+
+
+# ---------------------------------------------------------------------------------------
+# Multi-GPU
+# ---------------------------------------------------------------------------------------
+def _nccl_path():
+    try:
+        import nvidia.nccl
+        d = os.path.join(list(nvidia.nccl.__path__)[0], "lib", "libnccl.so.2")
+        return d if os.path.exists(d) else None
+    except Exception:
+        return None
+
+
+def get_unique_id() -> bytes:
+    if "SP_NCCL_LIB" not in os.environ and _nccl_path():
+        os.environ["SP_NCCL_LIB"] = _nccl_path()
+    buf = (ctypes.c_uint8 * 128)()
+    _check(lib.sp_get_unique_id(buf), "sp_get_unique_id")
+    return bytes(buf)
+
+
+class Comm:
+    """NCCL communicator owned by libsp (one per process / GPU)."""
+
+    def __init__(self, uid: bytes, nranks: int, rank: int, device: int):
+        if "SP_NCCL_LIB" not in os.environ and _nccl_path():
+            os.environ["SP_NCCL_LIB"] = _nccl_path()
+        h = vp()
+        buf = (ctypes.c_uint8 * 128)(*uid)
+        _check(lib.sp_comm_init(ctypes.byref(h), buf, int(nranks), int(rank), int(device)), "sp_comm_init")
+        self.handle = h
+        self.nranks, self.rank, self.device = nranks, rank, device
+
+    def destroy(self):
+        if self.handle:
+            _check(lib.sp_comm_destroy(self.handle), "sp_comm_destroy")
+            self.handle = None
+
+    def jacobi1d_timetiled_dist(self, a_local, work_local, n_global: int, x_begin: int, n_local: int, steps: int,
+                                time_tile: int = 16, space_tile: int = 0, stream=None):
+        _check(lib.sp_jacobi1d_timetiled_dist(self.handle, _ptr(a_local), _ptr(work_local), int(n_global), int(x_begin),
+                                              int(n_local), int(steps), int(time_tile), int(space_tile),
+                                              _stream(stream)), "sp_jacobi1d_timetiled_dist")
+
+    def allgather(self, send, recv, stream=None):
+        nbytes = send.numel() * send.element_size()
+        _check(lib.sp_allgather(self.handle, _ptr(send), _ptr(recv), nbytes, _stream(stream)), "sp_allgather")

@@ -1,0 +1,72 @@
+"""libsp.so loads on a GPU-less host and exports every entry point include/sp.h declares;
+host-only entry points (planner, geometry, footprints, status strings) work without a GPU."""
+import ctypes
+import os
+import re
+
+import pytest
+
+import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
+
+ROOT = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+
+
+def _declared():
+    txt = open(os.path.join(ROOT, "include", "sp.h")).read()
+    txt = re.sub(r"/\*.*?\*/", "", txt, flags=re.S)
+    return sorted(set(re.findall(r"\b(sp_[a-z0-9_]+)\s*\(", txt)))
+
+
+def test_exports_every_declared_symbol():
+    names = _declared()
+    assert len(names) >= 17
+    L = ctypes.CDLL(sp.LIB_PATH)
+    for n in names:
+        assert hasattr(L, n), n
+    # and the binding wires every one of them
+    assert set(names) <= set(sp.SYMBOLS), set(names) - set(sp.SYMBOLS)
+
+
+def test_status_strings_and_version():
+    assert sp.lib.sp_status_string(0) == b"SP_OK"
+    assert sp.lib.sp_status_string(-3) == b"SP_ERR_CAPACITY"
+    assert sp.lib.sp_status_string(-8) == b"SP_ERR_NCCL"
+    assert sp.lib.sp_version() >= 100
+
+
+def test_built_for_sm100a():
+    import subprocess
+    out = subprocess.run(["cuobjdump", "--list-elf", sp.LIB_PATH], capture_output=True, text=True).stdout
+    assert "sm_100a" in out
+
+
+def test_jacobi_plan_geometry_host_only():
+    p = sp.jacobi1d_plan(1 << 26, 1024, 16, 0)
+    assert p["passes"] == 64 and p["halo"] == 16
+    assert p["space_tile"] % 4 == 0 and p["tiles"] == -(-(1 << 26) // p["space_tile"])
+    assert sp.jacobi1d_plan(4096, 64, 16, 256)["space_tile"] == 256
+    with pytest.raises(sp.SPError):
+        sp.jacobi1d_plan(4096, 64, 0, 0)
+    with pytest.raises(sp.SPError):
+        sp.jacobi1d_plan(4096, 64, 16, 6)  # not a multiple of 4
+    with pytest.raises(sp.SPError):
+        sp.jacobi1d_plan(2, 64, 16, 0)
+
+
+def test_jacobi_tile_footprint_closed_form():
+    assert sp.jacobi1d_tile_footprint(100, 5, 0, 16) == (0, 20)
+    assert sp.jacobi1d_tile_footprint(100, 5, 96, 16) == (91, 99)
+    assert sp.jacobi1d_tile_footprint(100, 0, 32, 16) == (32, 47)
+
+
+def test_me_ref_window():
+    assert sp.me_ref_window(352, 288, 16, 0, 0) == ((0, 0), (31, 31))
+    assert sp.me_ref_window(352, 288, 16, 5, 7) == ((112 - 16, 80 - 16), (112 + 31, 80 + 31))
+    assert sp.me_ref_window(1920, 1080, 32, 119, 66) == ((1056 - 32, 1904 - 32), (1079, 1919))
+
+
+def test_device_entry_points_reject_bad_args_without_gpu():
+    # argument validation happens before any CUDA call
+    assert sp.lib.sp_jacobi1d_timetiled(None, None, 10, 1, 16, 0, None, None) == -1
+    assert sp.lib.sp_me_sad_search(None, None, 16, 16, 16, 0, 16, 1, 256, 8, 4, 0, 1, None, None, None, None) == -5
+    assert sp.lib.sp_me_sad_search(None, None, 16, 16, 16, 0, 16, 1, 256, 16, 4, 0, 1, None, None, None, None) == -1

@@ -1,0 +1,24 @@
+"""Minimal launch sequence of one kernel at the bench configuration, for ncu captures:
+   python tools/prof_target.py jacobi [Tt]   |   python tools/prof_target.py me"""
+import sys
+
+import torch
+
+sys.path.insert(0, ".")
+import paper_conf_ppopp_baskaranbkrrs08_b200 as sp  # noqa: E402
+import sp_inputs  # noqa: E402
+
+what = sys.argv[1]
+if what == "jacobi":
+    tt = int(sys.argv[2]) if len(sys.argv) > 2 else 16
+    n = 1 << 26
+    a = torch.from_numpy(sp_inputs.jacobi_input(n)).cuda()
+    w = torch.empty_like(a)
+    sp.jacobi1d_timetiled(a, 4 * tt, tt, 0, work=w)  # 4 launches
+else:
+    W, H, R = 1920, 1080, 32
+    fr = torch.from_numpy(sp_inputs.me_sequence(9, W, H, R)).cuda()
+    for _ in range(2):
+        sp.me_search_sequence(fr, W, H, R)
+torch.cuda.synchronize()
+print("done")
