@@ -66,17 +66,19 @@ class ClockSampler:
         self.device = device
         self.proc = None
         self.lines: list[str] = []
+        self.marks: list[float] = []
 
     def __enter__(self):
         try:
             self.proc = subprocess.Popen(
-                ["nvidia-smi", "-i", str(self.device), "--query-gpu=clocks.sm,clocks.max.sm,clocks_event_reasons.active,"
+                ["nvidia-smi", "-i", str(self.device), "--query-gpu=timestamp,clocks.sm,clocks.max.sm,clocks_event_reasons.active,"
                  "clocks_event_reasons.hw_slowdown,clocks_event_reasons.hw_thermal_slowdown,"
                  "clocks_event_reasons.sw_thermal_slowdown,clocks_event_reasons.sw_power_cap",
                  "--format=csv,noheader,nounits", "-lms", "100"],
                 stdout=subprocess.PIPE, stderr=subprocess.DEVNULL, text=True)
             self.t = threading.Thread(target=self._read, daemon=True)
             self.t.start()
+            time.sleep(1.0)  # let nvidia-smi start sampling before the timed region
         except Exception:
             self.proc = None
         return self
@@ -94,12 +96,26 @@ class ClockSampler:
                 self.proc.kill()
             self.t.join(timeout=2)
 
+    def mark(self):
+        self.marks.append(time.time())
+
     def summary(self):
+        """Samples whose timestamp falls inside [first mark, last mark] (the timed region)."""
+        import datetime
         sm, mx, reasons = [], None, set()
+        lo = self.marks[0] if self.marks else 0.0
+        hi = self.marks[-1] if self.marks else 1e30
         for ln in self.lines:
             f = [x.strip() for x in ln.split(",")]
-            if len(f) < 7:
+            if len(f) < 8:
                 continue
+            try:
+                ts = datetime.datetime.strptime(f[0], "%Y/%m/%d %H:%M:%S.%f").timestamp()
+            except ValueError:
+                continue
+            if not (lo - 0.15 <= ts <= hi + 0.15):
+                continue
+            f = f[1:]
             try:
                 sm.append(float(f[0]))
                 mx = float(f[1])
@@ -252,6 +268,7 @@ def run_ours(args, rank, world, local_rank):
     ev = [[torch.cuda.Event(enable_timing=True) for _ in range(3)] for _ in range(K)]
     with ClockSampler(local_rank) as clk:
         barrier()
+        clk.mark()
         e_start = torch.cuda.Event(enable_timing=True)
         e_end = torch.cuda.Event(enable_timing=True)
         e_start.record(stream)
@@ -263,6 +280,7 @@ def run_ours(args, rank, world, local_rank):
             ev[k][2].record(stream)
         e_end.record(stream)
         torch.cuda.synchronize()
+        clk.mark()
         barrier()
     total_ms = e_start.elapsed_time(e_end)
     jac_ms = sum(ev[k][0].elapsed_time(ev[k][1]) for k in range(K))

@@ -63,6 +63,7 @@ def lib():
         L.spo_jacobi1d_f64.argtypes = [f64p, i64, i32, f64p]
         L.spo_jacobi1d_tiled.argtypes = [f32p, i64, i32, i32, i64, f32p, f32p]
         L.spo_jacobi1d_points.argtypes = [f32p, i64, i32, ctypes.POINTER(i64), i64, f32p, f32p]
+        L.spo_jacobi1d_window.argtypes = [f32p, i64, i64, i64, i32, f32p]
         L.spo_me_search.argtypes = [ctypes.c_void_p, ctypes.c_void_p, i64, i32, i32, i32,
                                     ctypes.POINTER(i32), i64, ctypes.POINTER(ctypes.c_int16),
                                     ctypes.POINTER(ctypes.c_uint32), ctypes.POINTER(ctypes.c_uint32)]
@@ -103,6 +104,14 @@ def jacobi1d_tiled(a0: np.ndarray, steps: int, time_tile: int, space_tile: int) 
     local = np.empty(2 * (space_tile + 2 * time_tile) + 8, dtype=np.float32)
     lib().spo_jacobi1d_tiled(_p(a, ctypes.c_float), a.size, int(steps), int(time_tile), int(space_tile),
                              _p(work, ctypes.c_float), _p(local, ctypes.c_float))
+    return a
+
+
+def jacobi1d_window(w: np.ndarray, g0: int, n: int, steps: int) -> np.ndarray:
+    """h steps on a window holding global cells [g0, g0+len) (edges held; see oracle.c)."""
+    a = np.array(w, dtype=np.float32, copy=True)
+    scratch = np.empty_like(a)
+    lib().spo_jacobi1d_window(_p(a, ctypes.c_float), a.size, int(g0), int(n), int(steps), _p(scratch, ctypes.c_float))
     return a
 
 

@@ -164,6 +164,29 @@ void spo_jacobi1d_points(const float* a0, int64_t n, int32_t steps, const int64_
     }
 }
 
+/* h steps of the definition on a window w[0..len) holding global cells [g0, g0+len) of a
+ * domain of n cells: global cells 0 and n-1 stay fixed, and so do the window's two edge
+ * cells (their true neighbours are outside the window, so after h steps only cells at
+ * distance >= h from a non-domain window edge are exact).  scratch: len floats. */
+void spo_jacobi1d_window(float* w, int64_t len, int64_t g0, int64_t n, int32_t steps, float* scratch) {
+    float* L0 = w;
+    float* L1 = scratch;
+    for (int32_t t = 0; t < steps; ++t) {
+        for (int64_t j = 0; j < len; ++j) {
+            int64_t g = g0 + j;
+            if (g <= 0 || g >= n - 1 || j == 0 || j == len - 1) {
+                L1[j] = L0[j];
+            } else {
+                float v = L0[j - 1] + L0[j];
+                v = v + L0[j + 1];
+                L1[j] = v * SPO_W;
+            }
+        }
+        float* tmp = L0; L0 = L1; L1 = tmp;
+    }
+    if (L0 != w) memcpy(w, L0, (size_t)len * sizeof(float));
+}
+
 /* ---------------------------------------------------------------------------------
  * Motion estimation: full search (Fig. 2 nest with WS = 16).
  * DESIGN.md readings R-M1..R-M6:

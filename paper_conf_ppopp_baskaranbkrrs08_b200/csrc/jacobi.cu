@@ -22,6 +22,7 @@
 
 #include <algorithm>
 #include <cstdint>
+#include <cstdlib>
 #include <mutex>
 
 #include "../../include/sp.h"
@@ -32,11 +33,20 @@ namespace {
 
 using namespace sp::ptx;
 
-constexpr int kK = 16;                   // packed pairs per thread
-constexpr int kWarps = 8;                // warps per CTA
-constexpr int kThreads = 32 * kWarps;    // 256
-constexpr int kStrip = 64 * kK;          // cells per warp strip (1024)
-constexpr int kStage = kWarps * kStrip;  // floats per shared-memory stage (8192 = 32 KB)
+// Kernel geometry.  K packed pairs per thread (2K cells; K/4 odd keeps the 16-byte shared
+// accesses at stride 4K bytes bank-conflict free), WARPS warps per CTA, MINB CTAs per SM
+// for the register budget.  A warp strip is 64K cells; a shared-memory stage holds
+// WARPS strips.
+template <int K_, int WARPS_, int MINB_>
+struct JCfg {
+    static constexpr int K = K_;
+    static constexpr int kWarps = WARPS_;
+    static constexpr int kMinBlocks = MINB_;
+    static constexpr int kThreads = 32 * WARPS_;
+    static constexpr int kStrip = 64 * K_;
+    static constexpr int kStage = WARPS_ * 2 * 64 * K_;  // floats of shared memory per CTA
+    static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && K_ <= 32, "K/4 must be odd, K <= 32");
+};
 constexpr int kStages = 2;
 constexpr int kMaxTimeTile = 128;
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
@@ -57,11 +67,10 @@ struct PassArgs {
     uint64_t mz;       // (-0.0f, -0.0f), opaque to ptxas (see f2_mul_nofuse)
 };
 
-// One Jacobi step on the thread's 2K cells.  kBoundary: the warp strip contains global
-// cell 0 or n-1, which must keep its value (fix_u / fix_v: bit j set = pair j's u / v
-// component is a fixed boundary cell).
-template <bool kBoundary>
-__device__ __forceinline__ void step(uint64_t (&P)[kK], int lane, uint64_t w2, uint64_t mz, uint32_t fix_u, uint32_t fix_v) {
+// One Jacobi step on the thread's 2K cells, P -> Q (out of place, so the step loop needs
+// no register copies).  The lane neighbours come from four shuffles.
+template <int kK>
+__device__ __forceinline__ void step(const uint64_t (&P)[kK], uint64_t (&Q)[kK], int lane, uint64_t w2, uint64_t mz) {
     const float ul = f2_lo(P[kK - 1]), vl = f2_hi(P[kK - 1]);
     const float uf = f2_lo(P[0]), vf = f2_hi(P[0]);
     const float a = __shfl_sync(0xffffffffu, ul, (lane + 31) & 31);  // lane-1's last u
@@ -70,88 +79,124 @@ __device__ __forceinline__ void step(uint64_t (&P)[kK], int lane, uint64_t w2, u
     const float d = __shfl_sync(0xffffffffu, vf, (lane + 1) & 31);   // lane+1's first v
     // the v strip continues the u strip: lane 0's v-left is lane 31's last u and
     // lane 31's u-right is lane 0's first v
-    uint64_t prev = f2_pack(a, lane == 0 ? a : b);
+    const uint64_t left = f2_pack(a, lane == 0 ? a : b);
     const uint64_t right = f2_pack(lane == 31 ? d : c, d);
 #pragma unroll
     for (int j = 0; j < kK; ++j) {
-        const uint64_t cur = P[j];
+        const uint64_t prv = (j > 0) ? P[j - 1] : left;
         const uint64_t nxt = (j + 1 < kK) ? P[j + 1] : right;
-        uint64_t r = f2_mul_nofuse(f2_add(f2_add(prev, cur), nxt), w2, mz);
-        if (kBoundary) {
-            if ((fix_u >> j) & 1u) r = f2_pack(f2_lo(cur), f2_hi(r));
-            if ((fix_v >> j) & 1u) r = f2_pack(f2_lo(r), f2_hi(cur));
-        }
-        P[j] = r;
-        prev = cur;
+        Q[j] = f2_mul_nofuse(f2_add(f2_add(prv, P[j]), nxt), w2, mz);
     }
 }
 
-__global__ void __launch_bounds__(kThreads, 3) jacobi1d_pass_kernel(PassArgs A) {
+// Global cells 0 and n-1 are fixed (Dirichlet): in the (rare) warp strips that contain
+// one, restore it after each step.  Bit j of f0 / fn marks pair j's component holding
+// cell 0 / cell n-1 (bits 0..31: u component, bits 32..63: v component).
+template <int kK>
+__device__ __forceinline__ void restore(uint64_t (&Q)[kK], uint64_t f0, uint64_t fn, float v0, float vn) {
+#pragma unroll
+    for (int j = 0; j < kK; ++j) {
+        float u = f2_lo(Q[j]), v = f2_hi(Q[j]);
+        if ((f0 >> j) & 1u) u = v0;
+        if ((fn >> j) & 1u) u = vn;
+        if ((f0 >> (32 + j)) & 1u) v = v0;
+        if ((fn >> (32 + j)) & 1u) v = vn;
+        Q[j] = f2_pack(u, v);
+    }
+}
+
+// h steps, ping-ponging between two register arrays.  `boundary` is warp-uniform; the
+// restore sits outside the shuffles so they stay in converged code.
+template <int kK>
+__device__ __forceinline__ void run_steps(uint64_t (&P)[kK], int h, int lane, uint64_t w2, uint64_t mz, bool boundary,
+                                          uint64_t f0, uint64_t fn, float v0, float vn) {
+    uint64_t Q[kK];
+    int k = 0;
+    for (; k + 2 <= h; k += 2) {
+        step(P, Q, lane, w2, mz);
+        if (boundary) restore(Q, f0, fn, v0, vn);
+        step(Q, P, lane, w2, mz);
+        if (boundary) restore(P, f0, fn, v0, vn);
+    }
+    if (k < h) {
+        step(P, Q, lane, w2, mz);
+        if (boundary) restore(Q, f0, fn, v0, vn);
+#pragma unroll
+        for (int j = 0; j < kK; ++j) P[j] = Q[j];
+    }
+}
+
+// One launch = one time tile (pass).  Every WARP is an independent outer-level process
+// (processes on one multiprocessor divide its scratchpad): it owns a sequence of
+// space tiles of S cells, each staged as the warp strip [x0 - H, x0 - H + 64K) in the warp's
+// private double-buffered shared-memory slice.  Per tile:
+//   move-in  (H4): 1-D TMA bulk copy global -> shared, prefetched one tile ahead;
+//   compute  (H5a): registers (K packed pairs per lane), h steps, shuffles for neighbours;
+//   move-out (H7): owned cells [x0, x0+S) registers -> shared -> 1-D TMA bulk store.
+// No CTA-wide barrier anywhere: warps drift freely, so one warp's transfers overlap the
+// other warps' arithmetic.
+template <class Cfg>
+__global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_kernel(PassArgs A) {
+    constexpr int kK = Cfg::K, kStrip = Cfg::kStrip;
     extern __shared__ __align__(128) float smem[];
-    __shared__ __align__(8) uint64_t full[kStages];
+    __shared__ __align__(8) uint64_t full[Cfg::kWarps][2];
 
-    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    float* const stage0 = smem + warp * 2 * kStrip;  // this warp's two stages
+    uint64_t* const bar = full[warp];
     const uint64_t w2 = (uint64_t(kW) << 32) | kW;
-    const int64_t G = gridDim.x;
-    const int64_t first = blockIdx.x;
-
+    const int64_t GW = (int64_t)gridDim.x * Cfg::kWarps;
+    const int64_t first = (int64_t)blockIdx.x * Cfg::kWarps + warp;
     const int64_t lo_avail = A.g0 > 0 ? A.g0 : 0;
     const int64_t hi_avail = (A.g0 + A.len < A.n) ? A.g0 + A.len : A.n;
 
-    // Footprint actually transferred for tile t: [lo, hi) with lo 16-byte aligned; the
-    // 16-byte-multiple prefix goes by TMA, a <= 3-cell ragged end by plain loads.
+    // tile t owns [x0, x0 + st); its staged footprint is [lo, hi) (clipped to the domain and to
+    // the caller's window); the 16-byte-multiple prefix goes by TMA, a <= 3-cell end by loads
     auto tile_range = [&](int64_t t, int64_t& x0, int64_t& st, int64_t& lo, int64_t& hi) {
         x0 = A.own_begin + t * A.S;
         st = A.own_end - x0 < A.S ? A.own_end - x0 : A.S;
         lo = x0 - A.H > lo_avail ? x0 - A.H : lo_avail;
         hi = x0 + st + A.H < hi_avail ? x0 + st + A.H : hi_avail;
     };
-    auto issue = [&](int64_t t, int s) {  // single thread
+    auto issue = [&](int64_t t, int s) {  // lane 0 only
         int64_t x0, st, lo, hi;
         tile_range(t, x0, st, lo, hi);
         const uint32_t bytes = (uint32_t)(((hi - lo) & ~int64_t(3)) * 4);
-        mbar_arrive_expect_tx(&full[s], bytes);
-        if (bytes) tma_load_1d(smem + s * kStage + (lo - (x0 - A.H)), A.src + (lo - A.g0), bytes, &full[s]);
+        mbar_arrive_expect_tx(&bar[s], bytes);
+        if (bytes) tma_load_1d(stage0 + s * kStrip + (lo - (x0 - A.H)), A.src + (lo - A.g0), bytes, &bar[s]);
     };
 
-    if (tid == 0) {
-        for (int s = 0; s < kStages; ++s) mbar_init(&full[s], 1);
+    if (lane == 0) {
+        mbar_init(&bar[0], 1);
+        mbar_init(&bar[1], 1);
         fence_mbar_init();
+        if (first < A.tiles) issue(first, 0);
     }
-    __syncthreads();
-    if (tid == 0) {
-        for (int s = 0; s < kStages; ++s)
-            if (first + s * G < A.tiles) issue(first + s * G, s);
-    }
+    __syncwarp();
 
     int it = 0;
-    for (int64_t t = first; t < A.tiles; t += G, ++it) {
+    for (int64_t t = first; t < A.tiles; t += GW, ++it) {
         const int s = it & 1;
-        const uint32_t parity = (it >> 1) & 1;
-        float* buf = smem + s * kStage;
+        float* const buf = stage0 + s * kStrip;
         int64_t x0, st, lo, hi;
         tile_range(t, x0, st, lo, hi);
         const int64_t base = x0 - A.H;  // buf[j] <-> global base + j
-        {   // ragged end (<= 3 cells) that the 16-byte TMA could not carry
+        {
             const int64_t tail0 = lo + ((hi - lo) & ~int64_t(3));
-            if (tid < hi - tail0) buf[tail0 - base + tid] = A.src[tail0 + tid - A.g0];
+            if (lane < hi - tail0) buf[tail0 - base + lane] = A.src[tail0 + lane - A.g0];
         }
-        if (tid == 0 && A.flog) {
-            const int64_t flb = x0 - A.h > 0 ? x0 - A.h : 0;
-            const int64_t fub = x0 + st - 1 + A.h < A.n - 1 ? x0 + st - 1 + A.h : A.n - 1;
-            A.flog[2 * t] = flb;
-            A.flog[2 * t + 1] = fub;
+        if (lane == 0 && A.flog) {
+            A.flog[2 * t] = x0 - A.h > 0 ? x0 - A.h : 0;
+            A.flog[2 * t + 1] = x0 + st - 1 + A.h < A.n - 1 ? x0 + st - 1 + A.h : A.n - 1;
         }
-        mbar_wait(&full[s], parity);
-        __syncthreads();  // ragged-end stores visible
+        mbar_wait(&bar[s], (it >> 1) & 1);
+        __syncwarp();
 
-        // ---- registers <- staged strip -------------------------------------------------
-        const int wofs = warp * A.wo;                 // strip start in buf (multiple of 4)
-        const int64_t rb = base + wofs;               // global index of strip cell 0
+        // ---- registers <- staged strip (conflict-free: stride 4K bytes, K/4 odd) ---------
         uint64_t P[kK];
         {
-            const float4* pu = reinterpret_cast<const float4*>(buf + wofs + lane * kK);
-            const float4* pv = reinterpret_cast<const float4*>(buf + wofs + 32 * kK + lane * kK);
+            const float4* pu = reinterpret_cast<const float4*>(buf + lane * kK);
+            const float4* pv = reinterpret_cast<const float4*>(buf + 32 * kK + lane * kK);
 #pragma unroll
             for (int q = 0; q < kK / 4; ++q) {
                 const float4 u = pu[q], v = pv[q];
@@ -161,72 +206,114 @@ __global__ void __launch_bounds__(kThreads, 3) jacobi1d_pass_kernel(PassArgs A) 
                 P[4 * q + 3] = f2_pack(u.w, v.w);
             }
         }
-        // ---- h steps in registers ---------------------------------------------------
-        const bool boundary = (rb <= 0 && 0 < rb + kStrip) || (rb <= A.n - 1 && A.n - 1 < rb + kStrip);
-        if (!boundary) {
-            for (int k = 0; k < A.h; ++k) step<false>(P, lane, w2, A.mz, 0u, 0u);
-        } else {
-            const int64_t cu = rb + lane * kK, cv = rb + 32 * kK + lane * kK;
-            uint32_t fix_u = 0, fix_v = 0;
-            if (cu <= 0 && 0 < cu + kK) fix_u |= 1u << (0 - cu);
-            if (cu <= A.n - 1 && A.n - 1 < cu + kK) fix_u |= 1u << (A.n - 1 - cu);
-            if (cv <= 0 && 0 < cv + kK) fix_v |= 1u << (0 - cv);
-            if (cv <= A.n - 1 && A.n - 1 < cv + kK) fix_v |= 1u << (A.n - 1 - cv);
-            for (int k = 0; k < A.h; ++k) step<true>(P, lane, w2, A.mz, fix_u, fix_v);
+        // ---- prefetch the next tile into the other stage once its store has drained ----
+        if (lane == 0 && t + GW < A.tiles) {
+            bulk_wait_read0();
+            issue(t + GW, s ^ 1);
         }
-        __syncthreads();  // every warp has finished reading this stage
-
-        // ---- owned cells -> staged buffer (move-out staging) -------------------------
+        // ---- h steps in registers ---------------------------------------------------
         {
-            // warp owns strip offsets [H, H + own_w); tile-local owned range is [H, H + st)
-            const int own_lo = A.H;
-            const int64_t rem_w = st - (int64_t)wofs;
-            const int own_hi = A.H + (int)(rem_w < A.wo ? rem_w : (int64_t)A.wo);
-            float4* qu = reinterpret_cast<float4*>(buf + wofs + lane * kK);
-            float4* qv = reinterpret_cast<float4*>(buf + wofs + 32 * kK + lane * kK);
+            const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= A.n - 1 && A.n - 1 < base + kStrip);
+            uint64_t f0 = 0, fn = 0;
+            float v0 = 0.f, vn = 0.f;
+            if (boundary) {
+                const int64_t cu = base + lane * kK, cv = base + 32 * kK + lane * kK;
+                if (cu <= 0 && 0 < cu + kK) f0 |= 1ull << (0 - cu);
+                if (cv <= 0 && 0 < cv + kK) f0 |= 1ull << (32 + (0 - cv));
+                if (cu <= A.n - 1 && A.n - 1 < cu + kK) fn |= 1ull << (A.n - 1 - cu);
+                if (cv <= A.n - 1 && A.n - 1 < cv + kK) fn |= 1ull << (32 + (A.n - 1 - cv));
+                if (0 >= base) v0 = buf[0 - base];
+                if (A.n - 1 - base < kStrip) vn = buf[A.n - 1 - base];
+            }
+            run_steps(P, A.h, lane, w2, A.mz, boundary, f0, fn, v0, vn);
+        }
+        // ---- owned cells -> staged buffer -> TMA bulk store ------------------------------
+        {
+            const int own_hi = A.H + (int)st;  // strip offsets [H, H + st) are owned
+            float4* qu = reinterpret_cast<float4*>(buf + lane * kK);
+            float4* qv = reinterpret_cast<float4*>(buf + 32 * kK + lane * kK);
 #pragma unroll
             for (int q = 0; q < kK / 4; ++q) {
                 const int ou = lane * kK + 4 * q, ov = 32 * kK + lane * kK + 4 * q;
-                if (ou >= own_lo && ou < own_hi)
+                if (ou >= A.H && ou < own_hi)
                     qu[q] = make_float4(f2_lo(P[4 * q]), f2_lo(P[4 * q + 1]), f2_lo(P[4 * q + 2]), f2_lo(P[4 * q + 3]));
-                if (ov >= own_lo && ov < own_hi)
+                if (ov >= A.H && ov < own_hi)
                     qv[q] = make_float4(f2_hi(P[4 * q]), f2_hi(P[4 * q + 1]), f2_hi(P[4 * q + 2]), f2_hi(P[4 * q + 3]));
             }
         }
-        __syncthreads();
-        // ---- coalesced 128-bit copy of the owned cells to global ----------------------
-        {
-            const float4* s4 = reinterpret_cast<const float4*>(buf + A.H);
-            float4* d4 = reinterpret_cast<float4*>(A.dst + (x0 - A.g0));
-            const int n4 = (int)(st >> 2);
-            for (int q = tid; q < n4; q += kThreads) d4[q] = s4[q];
-            const int rem = (int)(st & 3);
-            if (tid < rem) A.dst[x0 - A.g0 + 4 * n4 + tid] = buf[A.H + 4 * n4 + tid];
-        }
         fence_proxy_async_smem();
-        __syncthreads();  // stage free: refill it with tile t + 2G
-        if (tid == 0 && t + 2 * G < A.tiles) issue(t + 2 * G, s);
+        __syncwarp();
+        {
+            const int64_t n16 = st & ~int64_t(3);
+            if (lane == 0 && n16 > 0) {
+                tma_store_1d(A.dst + (x0 - A.g0), buf + A.H, (uint32_t)(n16 * 4));
+                bulk_commit();
+            }
+            if (lane < st - n16) A.dst[x0 - A.g0 + n16 + lane] = buf[A.H + n16 + lane];
+        }
     }
+    if (lane == 0) bulk_wait0();
 }
 
-struct DeviceInfo {
-    int sms = 0;
-    int occ = 0;
+// ---- host side: kernel variants (geometry sweep; SP_JACOBI_VARIANT selects one) ----------
+struct Variant {
+    int K, warps, threads, strip, stage_floats;
+    void (*kernel)(PassArgs);
+    int sms = 0, occ = 0;
     bool ok = false;
 };
 
-int device_info(DeviceInfo& out) {
+template <class Cfg>
+Variant make_variant() {
+    Variant v;
+    v.K = Cfg::K;
+    v.warps = Cfg::kWarps;
+    v.threads = Cfg::kThreads;
+    v.strip = Cfg::kStrip;
+    v.stage_floats = Cfg::kStage;
+    v.kernel = jacobi1d_pass_kernel<Cfg>;
+    return v;
+}
+
+constexpr int kNumVariants = 5;
+constexpr int kDefaultVariant = 1;
+
+Variant* variants() {
+    static Variant v[kNumVariants] = {
+        make_variant<JCfg<12, 4, 8>>(),  // 0: 24 cells/lane, 4 warps/CTA, <= 64 regs
+        make_variant<JCfg<12, 8, 4>>(),  // 1: 24 cells/lane, 8 warps/CTA
+        make_variant<JCfg<20, 4, 5>>(),  // 2: 40 cells/lane
+        make_variant<JCfg<28, 4, 4>>(),  // 3: 56 cells/lane
+        make_variant<JCfg<12, 4, 6>>(),  // 4: 24 cells/lane, <= 85 regs
+    };
+    return v;
+}
+
+int variant_index() {
+    static int idx = [] {
+        const char* e = std::getenv("SP_JACOBI_VARIANT");
+        int i = e ? std::atoi(e) : kDefaultVariant;
+        return (i >= 0 && i < kNumVariants) ? i : kDefaultVariant;
+    }();
+    return idx;
+}
+
+int smem_bytes(const Variant& v) { return v.stage_floats * (int)sizeof(float); }
+
+// occupancy of the selected variant on the current device (cached per device)
+int device_info(Variant& out) {
     static std::mutex mu;
-    static DeviceInfo cache[64];
+    static Variant cache[64][kNumVariants];
     int dev = 0;
     SP_CUDA_TRY(cudaGetDevice(&dev));
+    const int vi = variant_index();
     std::lock_guard<std::mutex> lk(mu);
-    DeviceInfo& d = cache[dev & 63];
+    Variant& d = cache[dev & 63][vi];
     if (!d.ok) {
+        d = variants()[vi];
         SP_CUDA_TRY(cudaDeviceGetAttribute(&d.sms, cudaDevAttrMultiProcessorCount, dev));
-        const int smem = kStages * kStage * (int)sizeof(float);
-        SP_CUDA_TRY(cudaFuncSetAttribute(jacobi1d_pass_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem));
-        SP_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&d.occ, jacobi1d_pass_kernel, kThreads, smem));
+        SP_CUDA_TRY(cudaFuncSetAttribute(d.kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes(d)));
+        SP_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&d.occ, d.kernel, d.threads, smem_bytes(d)));
         if (d.occ < 1) d.occ = 1;
         d.ok = true;
     }
@@ -237,28 +324,27 @@ int device_info(DeviceInfo& out) {
 inline int32_t halo_of(int32_t time_tile) { return (time_tile + 3) & ~3; }
 
 int geometry(int32_t time_tile, int32_t space_tile, int64_t& S, int32_t& wo) {
+    const Variant& v = variants()[variant_index()];
     if (time_tile < 1 || time_tile > kMaxTimeTile) return SP_ERR_INVALID_ARG;
     const int32_t H = halo_of(time_tile);
-    const int32_t wo_max = kStrip - 2 * H;  // multiple of 4
-    const int64_t S_max = (int64_t)kWarps * wo_max;
+    const int32_t S_max = v.strip - 2 * H;  // owned cells of a warp tile (multiple of 4)
+    if (S_max < 4) return SP_ERR_INVALID_ARG;
     if (space_tile == 0) {
         S = S_max;
-        wo = wo_max;
+        wo = S_max;
         return SP_OK;
     }
     if (space_tile < 4 || space_tile % 4 != 0 || space_tile > S_max) return SP_ERR_INVALID_ARG;
     S = space_tile;
-    wo = (int32_t)(((S + kWarps - 1) / kWarps + 3) & ~int64_t(3));
+    wo = space_tile;
     return SP_OK;
 }
 
-int launch_pass(const PassArgs& a0, cudaStream_t stream, const DeviceInfo& di) {
-    PassArgs a = a0;
+int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v) {
     if (a.tiles <= 0) return SP_OK;
-    const int64_t cap = (int64_t)di.sms * di.occ;
+    const int64_t cap = (int64_t)v.sms * v.occ;
     const int grid = (int)(a.tiles < cap ? a.tiles : cap);
-    const int smem = kStages * kStage * (int)sizeof(float);
-    jacobi1d_pass_kernel<<<grid, kThreads, smem, stream>>>(a);
+    v.kernel<<<grid, v.threads, smem_bytes(v), stream>>>(a);
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }
@@ -278,10 +364,11 @@ extern "C" int sp_jacobi1d_plan(int64_t n, int32_t steps, int32_t time_tile, int
     out->passes = (steps + time_tile - 1) / time_tile;
     out->space_tile = S;
     out->tiles = (n + S - 1) / S;
-    out->threads = kThreads;
-    out->smem_bytes = kStages * kStage * (int)sizeof(float);
-    out->cells_per_thread = 2 * kK;
-    DeviceInfo di;
+    const Variant& v = variants()[variant_index()];
+    out->threads = v.threads;
+    out->smem_bytes = smem_bytes(v);
+    out->cells_per_thread = 2 * v.K;
+    Variant di;
     out->grid = 0;
     if (device_info(di) == SP_OK) {
         const int64_t cap = (int64_t)di.sms * di.occ;
@@ -322,7 +409,7 @@ extern "C" int sp_jacobi1d_pass_segment(const float* src, float* dst, int64_t n_
                                         cudaMemcpyDeviceToDevice, (cudaStream_t)stream));
         return SP_OK;
     }
-    DeviceInfo di;
+    Variant di;
     if ((st = device_info(di))) return st;
     PassArgs a{src, dst, n_global, g0, len, own_begin, own_end, S, (own_end - own_begin + S - 1) / S, h, H, wo, nullptr, kNegZero2};
     return launch_pass(a, (cudaStream_t)stream, di);
@@ -337,7 +424,7 @@ extern "C" int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t s
     int st = geometry(time_tile, space_tile, S, wo);
     if (st) return st;
     if (steps == 0) return SP_OK;
-    DeviceInfo di;
+    Variant di;
     if ((st = device_info(di))) return st;
     const cudaStream_t s = (cudaStream_t)stream;
     const int32_t H = halo_of(time_tile);

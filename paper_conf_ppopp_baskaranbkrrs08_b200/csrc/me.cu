@@ -42,7 +42,7 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 constexpr int kRows = kTy + kMB - 1;  // window rows a thread sweeps (23)
 
 struct MeArgs {
-    int32_t width, frame_height, row0, range;
+    int32_t width, frame_height, row0, range, n_pairs;
     int32_t mbx, mb_row_begin, mb_rows;
     int32_t win;  // window edge = 2R + 16 (bytes per copy row, rows per copy)
     int16_t* mv;
@@ -63,162 +63,260 @@ __device__ __forceinline__ uint64_t warp_min_key(uint64_t k) {
     return ((uint64_t)mh << 32) | ml;
 }
 
-// Fast path: R in {16, 32} (x0 - R 16-byte aligned); blockDim = R*R/8.
-__global__ void __launch_bounds__(128, 3)
-me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
-    extern __shared__ __align__(128) uint8_t smem_raw[];
-    __shared__ __align__(8) uint64_t bar;
-    __shared__ uint64_t warp_keys[32];
-    // TMA tile destinations must be 128-byte aligned
-    uint8_t* smem = reinterpret_cast<uint8_t*>((reinterpret_cast<uintptr_t>(smem_raw) + 127) & ~uintptr_t(127));
+// Fast path: R in {16, 32} (x0 - R is then 16-byte aligned, as the TMA box origin must
+// be).  Persistent CTAs walk the (pair, MB row, MB column) space; the next-but-one
+// macroblock's window streams in by TMA (double-buffered) while the current one is searched.
+template <int R>
+struct MeGeom {
+    static constexpr int kWin = 2 * R + 16;              // window edge (bytes per row, rows)
+    static constexpr int kCopy = kWin * kWin;            // bytes per staged copy (multiple of 128)
+    static constexpr int kThreads = R * R / 8;           // one 4x8 candidate tile per thread
+    static constexpr int kGx = R / 8;                    // dx groups per byte phase
+    static constexpr int kPhStride = kCopy + 32;         // phase copies at 32-byte bank offsets
+    static constexpr int kOffCur = 2 * kCopy;            // cur[2] after raw[2]
+    static constexpr int kOffPh = 2 * kCopy + 512 + 32;  // copy p at kOffPh + (p-1)*kPhStride
+    static constexpr int kSmem = kOffPh + 3 * kPhStride + 128;  // + alignment slack
+    static constexpr int kTail = 4 * R + 1;
+};
 
-    const int R = A.range;
-    const int win = A.win;
-    const int copy_bytes = win * win;
-    uint8_t* cur_s = smem + 4 * copy_bytes;
-    const int tid = threadIdx.x, nthr = blockDim.x;
-    const int bx = blockIdx.x, byr = blockIdx.y, pair = blockIdx.z;
-    const int by = A.mb_row_begin + byr;  // global MB row
-    const int x0 = kMB * bx, y0 = kMB * by;
-    const int ywin = y0 - R - A.row0;  // buffer row of window row 0
+template <int R>
+__global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
+me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
+    using G = MeGeom<R>;
+    constexpr int win = G::kWin;
+    extern __shared__ __align__(128) uint8_t smem_raw[];
+    __shared__ __align__(8) uint64_t full[2];
+    __shared__ uint32_t red32[32];
+    __shared__ uint64_t red64[32];
+    // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
+    uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
+
+    const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    constexpr int nwarps = (G::kThreads + 31) / 32;
+    const int mbx = A.mbx;
+    const int64_t per_pair = (int64_t)A.mb_rows * mbx;
+    const int64_t total = per_pair * A.n_pairs;
+    const int64_t Gs = gridDim.x;
+    const int W = A.width, Hf = A.frame_height;
+    constexpr int side = 2 * R + 1;
+
+    auto issue = [&](int64_t mb, int s) {  // single thread: stage the window + cur of mb
+        const int pair = (int)(mb / per_pair);
+        const int64_t rem = mb - (int64_t)pair * per_pair;
+        const int by = A.mb_row_begin + (int)(rem / mbx), bx = (int)(rem % mbx);
+        const int x0 = kMB * bx, y0 = kMB * by;
+        mbar_arrive_expect_tx(&full[s], (uint32_t)(G::kCopy + kMB * kMB));
+        tma_load_3d(smem + s * G::kCopy, &ref_map, x0 - R, y0 - R - A.row0, pair, &full[s]);
+        tma_load_3d(smem + G::kOffCur + s * 256, &cur_map, x0, y0 - A.row0, pair, &full[s]);
+    };
 
     if (tid == 0) {
         prefetch_tmap(&ref_map);
         prefetch_tmap(&cur_map);
-        mbar_init(&bar, 1);
+        mbar_init(&full[0], 1);
+        mbar_init(&full[1], 1);
         fence_mbar_init();
-        mbar_arrive_expect_tx(&bar, (uint32_t)(copy_bytes + kMB * kMB));
-        // the TMA box origin must be 16-byte aligned in the innermost dimension, so the
-        // window is staged once at x0 - R (R % 16 == 0) and the byte phases are built below
-        tma_load_3d(smem, &ref_map, x0 - R, ywin, pair, &bar);
-        tma_load_3d(cur_s, &cur_map, x0, y0 - A.row0, pair, &bar);
     }
     __syncthreads();
-    mbar_wait(&bar, 0);
-    {   // byte-phase copies p = 1..3: word q of copy p = bytes [4q+p, 4q+p+4) of the row
-        const int v4_per_row = win / 16;
-        const int nv4 = win * v4_per_row;
-        for (int v = tid; v < nv4; v += nthr) {
-            const int r = v / v4_per_row, c = v - r * v4_per_row;
-            const uint32_t* row = reinterpret_cast<const uint32_t*>(smem + r * win);
-            const uint4 w = reinterpret_cast<const uint4*>(row)[c];
-            const uint32_t nx = (c + 1 < v4_per_row) ? row[4 * c + 4] : 0u;
+    if (tid == 0) {
+        if (blockIdx.x < total) issue(blockIdx.x, 0);
+        if (blockIdx.x + Gs < total) issue(blockIdx.x + Gs, 1);
+    }
+
+    // thread's candidate tile: dx = -R + p + 4*(4g + j), dy = -R + 8d + i
+    const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
+
+    int it = 0;
+    for (int64_t mb = blockIdx.x; mb < total; mb += Gs, ++it) {
+        const int s = it & 1;
+        const int pair = (int)(mb / per_pair);
+        const int64_t rem = mb - (int64_t)pair * per_pair;
+        const int byr = (int)(rem / mbx), bx = (int)(rem % mbx);
+        const int x0 = kMB * bx, y0 = kMB * (A.mb_row_begin + byr);
+        const uint8_t* raw = smem + s * G::kCopy;
+        mbar_wait(&full[s], (it >> 1) & 1);
+
+        {   // byte-phase copies p = 1..3: word q of copy p = bytes [4q+p, 4q+p+4) of the row
+            constexpr int v4_per_row = win / 16;
+            for (int v = tid; v < win * v4_per_row; v += G::kThreads) {
+                const int r = v / v4_per_row, c = v - r * v4_per_row;
+                const uint32_t* row = reinterpret_cast<const uint32_t*>(raw + r * win);
+                const uint4 w = reinterpret_cast<const uint4*>(row)[c];
+                const uint32_t nx = (c + 1 < v4_per_row) ? row[4 * c + 4] : 0u;
 #pragma unroll
-            for (int p = 1; p < 4; ++p) {
-                uint4 o;
-                o.x = __funnelshift_r(w.x, w.y, 8 * p);
-                o.y = __funnelshift_r(w.y, w.z, 8 * p);
-                o.z = __funnelshift_r(w.z, w.w, 8 * p);
-                o.w = __funnelshift_r(w.w, nx, 8 * p);
-                reinterpret_cast<uint4*>(smem + p * copy_bytes + r * win)[c] = o;
+                for (int q = 1; q < 4; ++q) {
+                    uint4 o;
+                    o.x = __funnelshift_r(w.x, w.y, 8 * q);
+                    o.y = __funnelshift_r(w.y, w.z, 8 * q);
+                    o.z = __funnelshift_r(w.z, w.w, 8 * q);
+                    o.w = __funnelshift_r(w.w, nx, 8 * q);
+                    reinterpret_cast<uint4*>(smem + G::kOffPh + (q - 1) * G::kPhStride + r * win)[c] = o;
+                }
             }
         }
-    }
-    __syncthreads();
+        __syncthreads();  // phase copies complete
 
-    // hoisted current block: 16 rows x 4 words
-    uint32_t C[kMB][4];
-#pragma unroll
-    for (int v = 0; v < kMB; ++v) {
-        const uint4 q = reinterpret_cast<const uint4*>(cur_s)[v];
-        C[v][0] = q.x;
-        C[v][1] = q.y;
-        C[v][2] = q.z;
-        C[v][3] = q.w;
-    }
-
-    const int ngx = R / 8;             // dx groups per phase
-    const int nmain = ngx * 4 * (R / 4);
-    uint64_t best = ~0ull;
-    const int side = 2 * R + 1;
-    const int W = A.width, Hf = A.frame_height;
-    const size_t mb_index = ((size_t)pair * A.mb_rows + byr) * A.mbx + bx;
-
-    if (tid < nmain) {
-        const int p = tid & 3;
-        const int g = (tid >> 2) % ngx;
-        const int d = tid / (4 * ngx);
+        // ---- main 2R x 2R candidates: 4 dx (one byte phase) x 8 dy per thread ----------
         uint32_t acc[kTx][kTy];
 #pragma unroll
         for (int j = 0; j < kTx; ++j)
 #pragma unroll
             for (int i = 0; i < kTy; ++i) acc[j][i] = 0;
-        const uint8_t* rowp = smem + p * copy_bytes + (kTy * d) * win + 16 * g;
+        {
+            // Candidate (j, i) compares cur row v with window row 8d + i + v.  Loop over v with
+            // a ring of the 8 window rows in use (row rho in slot rho & 7, 7 words each: the
+            // 4 dx candidates x 4 words of one byte phase); body unrolled 8x so every ring
+            // index is static, outer loop rolled to halve the code (I-cache).  Innermost
+            // order (k, i, j) makes consecutive VABSDIFF4s independent.
+            const uint8_t* base = (p == 0) ? raw : smem + G::kOffPh + (p - 1) * G::kPhStride;
+            const uint8_t* rowp = base + (kTy * d) * win + 16 * g;
+            const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+            uint32_t Rw[8][7];  // words 4g..4g+6 (j + k <= 6)
 #pragma unroll
-        for (int r = 0; r < kRows; ++r) {
-            const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + r * win);
-            const uint4 w1 = *reinterpret_cast<const uint4*>(rowp + r * win + 16);
-            const uint32_t Wd[8] = {w0.x, w0.y, w0.z, w0.w, w1.x, w1.y, w1.z, w1.w};
+            for (int rr = 0; rr < 7; ++rr) {
+                const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + rr * win);
+                const uint4 w1 = *reinterpret_cast<const uint4*>(rowp + rr * win + 16);
+                Rw[rr][0] = w0.x; Rw[rr][1] = w0.y; Rw[rr][2] = w0.z; Rw[rr][3] = w0.w;
+                Rw[rr][4] = w1.x; Rw[rr][5] = w1.y; Rw[rr][6] = w1.z;
+            }
+#pragma unroll 1
+            for (int vb = 0; vb < kMB; vb += 8) {
 #pragma unroll
-            for (int i = 0; i < kTy; ++i) {
-                const int v = r - i;
-                if (v < 0 || v >= kMB) continue;
+                for (int vv = 0; vv < 8; ++vv) {
+                    const int v = vb + vv;
+                    {
+                        const int slot = (vv + 7) & 7;
+                        const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + (v + 7) * win);
+                        const uint4 w1 = *reinterpret_cast<const uint4*>(rowp + (v + 7) * win + 16);
+                        Rw[slot][0] = w0.x; Rw[slot][1] = w0.y; Rw[slot][2] = w0.z; Rw[slot][3] = w0.w;
+                        Rw[slot][4] = w1.x; Rw[slot][5] = w1.y; Rw[slot][6] = w1.z;
+                    }
+                    const uint4 cv = cq[v];
+                    const uint32_t Cv[4] = {cv.x, cv.y, cv.z, cv.w};
 #pragma unroll
-                for (int j = 0; j < kTx; ++j) {
-                    uint32_t a = acc[j][i];
-                    a = sad4(Wd[j + 0], C[v][0], a);
-                    a = sad4(Wd[j + 1], C[v][1], a);
-                    a = sad4(Wd[j + 2], C[v][2], a);
-                    a = sad4(Wd[j + 3], C[v][3], a);
-                    acc[j][i] = a;
+                    for (int k = 0; k < 4; ++k)
+#pragma unroll
+                        for (int i = 0; i < kTy; ++i)
+#pragma unroll
+                            for (int j = 0; j < kTx; ++j)
+                                acc[j][i] = sad4(Rw[(vv + i) & 7][j + k], Cv[k], acc[j][i]);
                 }
             }
         }
-        // epilogue: validity, keys, optional surface
-        const bool interior = (x0 - R >= 0) && (x0 + 16 + R <= W) && (y0 - R >= 0) && (y0 + 16 + R <= Hf);
+        // ---- tail candidates: column dx = +R (dy in [-R, R]) and row dy = +R (dx < R) ----
+        constexpr int kTailPer = (G::kTail + G::kThreads - 1) / G::kThreads;
+        uint32_t tacc[kTailPer];
 #pragma unroll
-        for (int j = 0; j < kTx; ++j) {
-            const int dx = -R + p + 4 * (4 * g + j);
+        for (int t = 0; t < kTailPer; ++t) {
+            const int c = tid + t * G::kThreads;
+            uint32_t a = 0xffffffffu;
+            if (c < G::kTail) {
+                const int dx = (c < side) ? R : -R + (c - side);
+                const int dy = (c < side) ? -R + c : R;
+                const int pp = (dx + R) & 3, m = (dx + R) >> 2;
+                const uint8_t* cb = (pp == 0) ? raw : smem + G::kOffPh + (pp - 1) * G::kPhStride;
+                const uint32_t* rw = reinterpret_cast<const uint32_t*>(cb + (dy + R) * win) + m;
+                a = 0;
 #pragma unroll
-            for (int i = 0; i < kTy; ++i) {
-                const int dy = -R + kTy * d + i;
-                const bool valid =
-                    interior || ((x0 + dx >= 0) && (x0 + dx + 16 <= W) && (y0 + dy >= 0) && (y0 + dy + 16 <= Hf));
-                const uint64_t k = valid ? make_key(acc[j][i], dx, dy, R) : ~0ull;
-                best = k < best ? k : best;
-                if (A.surface) A.surface[mb_index * side * side + (size_t)(dy + R) * side + (dx + R)] = valid ? acc[j][i] : 0xffffffffu;
+                for (int v = 0; v < kMB; ++v) {
+                    const uint32_t* q = rw + v * (win / 4);
+                    const uint4 cv = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256)[v];
+                    a = sad4(q[0], cv.x, a);
+                    a = sad4(q[1], cv.y, a);
+                    a = sad4(q[2], cv.z, a);
+                    a = sad4(q[3], cv.w, a);
+                }
+            }
+            tacc[t] = a;
+        }
+
+        // ---- validity (restricted vectors) only matters near the frame border ----------
+        const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
+        const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
+        const bool interior = dxlo == -R && dxhi == R && dylo == -R && dyhi == R;
+        if (!interior) {
+#pragma unroll
+            for (int j = 0; j < kTx; ++j) {
+                const int dx = -R + p + 4 * (4 * g + j);
+#pragma unroll
+                for (int i = 0; i < kTy; ++i) {
+                    const int dy = -R + kTy * d + i;
+                    if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) acc[j][i] = 0xffffffffu;
+                }
+            }
+#pragma unroll
+            for (int t = 0; t < kTailPer; ++t) {
+                const int c = tid + t * G::kThreads;
+                const int dx = (c < side) ? R : -R + (c - side);
+                const int dy = (c < side) ? -R + c : R;
+                if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) tacc[t] = 0xffffffffu;
             }
         }
-    }
-    // tail candidates: column dx = +R (dy in [-R, R]) and row dy = +R (dx in [-R, R-1])
-    const int ntail = 4 * R + 1;
-    for (int c = tid; c < ntail; c += nthr) {
-        int dx, dy;
-        if (c < side) {
-            dx = R;
-            dy = -R + c;
-        } else {
-            dx = -R + (c - side);
-            dy = R;
-        }
-        const int p = (dx + R) & 3, m = (dx + R) >> 2;
-        const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + p * copy_bytes + (dy + R) * win) + m;
-        uint32_t a = 0;
+        const size_t mb_index = ((size_t)pair * A.mb_rows + byr) * mbx + bx;
+        if (A.surface) {
+            uint32_t* sf = A.surface + mb_index * side * side;
 #pragma unroll
-        for (int v = 0; v < kMB; ++v) {
-            const uint32_t* q = rw + v * (win / 4);
-            a = sad4(q[0], C[v][0], a);
-            a = sad4(q[1], C[v][1], a);
-            a = sad4(q[2], C[v][2], a);
-            a = sad4(q[3], C[v][3], a);
+            for (int j = 0; j < kTx; ++j)
+#pragma unroll
+                for (int i = 0; i < kTy; ++i)
+                    sf[(kTy * d + i) * side + (p + 4 * (4 * g + j))] = acc[j][i];
+#pragma unroll
+            for (int t = 0; t < kTailPer; ++t) {
+                const int c = tid + t * G::kThreads;
+                if (c < G::kTail) {
+                    const int dx = (c < side) ? R : -R + (c - side);
+                    const int dy = (c < side) ? -R + c : R;
+                    sf[(dy + R) * side + (dx + R)] = tacc[t];
+                }
+            }
         }
-        const bool valid = (x0 + dx >= 0) && (x0 + dx + 16 <= W) && (y0 + dy >= 0) && (y0 + dy + 16 <= Hf);
-        const uint64_t k = valid ? make_key(a, dx, dy, R) : ~0ull;
-        best = k < best ? k : best;
-        if (A.surface) A.surface[mb_index * side * side + (size_t)(dy + R) * side + (dx + R)] = valid ? a : 0xffffffffu;
-    }
-    // argmin across the CTA
-    best = warp_min_key(best);
-    const int warp = tid >> 5, lane = tid & 31, nwarps = (nthr + 31) >> 5;
-    if (lane == 0) warp_keys[warp] = best;
-    __syncthreads();
-    if (tid == 0) {
-        uint64_t b = warp_keys[0];
-        for (int w = 1; w < nwarps; ++w) b = warp_keys[w] < b ? warp_keys[w] : b;
-        const int dx = (int)(b & 127) - R, dy = (int)((b >> 7) & 127) - R;
-        A.mv[2 * mb_index] = (int16_t)dx;
-        A.mv[2 * mb_index + 1] = (int16_t)dy;
-        A.sad[mb_index] = (uint32_t)(b >> 21);
+        // ---- argmin (SAD, |dx|+|dy|, dy, dx): block min of SAD, then the tie-break key
+        //      only among candidates that reach it (invalid candidates hold 0xFFFFFFFF) ----
+        uint32_t m = 0xffffffffu;
+#pragma unroll
+        for (int j = 0; j < kTx; ++j)
+#pragma unroll
+            for (int i = 0; i < kTy; ++i) m = min(m, acc[j][i]);
+#pragma unroll
+        for (int t = 0; t < kTailPer; ++t) m = min(m, tacc[t]);
+        const uint32_t wm = __reduce_min_sync(0xffffffffu, m);
+        if (lane == 0) red32[warp] = wm;
+        __syncthreads();
+        uint32_t M = red32[0];
+#pragma unroll
+        for (int w = 1; w < nwarps; ++w) M = min(M, red32[w]);
+        uint64_t key = ~0ull;
+        if (m == M) {  // rare: only threads holding a minimal candidate
+#pragma unroll
+            for (int j = 0; j < kTx; ++j)
+#pragma unroll
+                for (int i = 0; i < kTy; ++i)
+                    if (acc[j][i] == M) {
+                        const uint64_t k = make_key(M, -R + p + 4 * (4 * g + j), -R + kTy * d + i, R);
+                        key = k < key ? k : key;
+                    }
+#pragma unroll
+            for (int t = 0; t < kTailPer; ++t) {
+                const int c = tid + t * G::kThreads;
+                if (c < G::kTail && tacc[t] == M) {
+                    const uint64_t k = make_key(M, (c < side) ? R : -R + (c - side), (c < side) ? -R + c : R, R);
+                    key = k < key ? k : key;
+                }
+            }
+        }
+        key = warp_min_key(key);
+        if (lane == 0) red64[warp] = key;
+        __syncthreads();  // also: every thread is done with raw[s], cur[s] and the phases
+        if (tid == 0) {
+            uint64_t b = red64[0];
+#pragma unroll
+            for (int w = 1; w < nwarps; ++w) b = red64[w] < b ? red64[w] : b;
+            A.mv[2 * mb_index] = (int16_t)((int)(b & 127) - R);
+            A.mv[2 * mb_index + 1] = (int16_t)((int)((b >> 7) & 127) - R);
+            A.sad[mb_index] = (uint32_t)(b >> 21);
+            fence_proxy_async_smem();
+            if (mb + 2 * Gs < total) issue(mb + 2 * Gs, s);
+        }
     }
 }
 
@@ -316,6 +414,28 @@ int make_map(CUtensorMap* m, const uint8_t* base, int32_t width, int32_t rows, i
 
 bool fast_range(int R) { return R == 16 || R == 32; }
 
+template <int R>
+int launch_fast(const CUtensorMap& rm, const CUtensorMap& cm, const MeArgs& a, int64_t total, cudaStream_t s) {
+    using G = MeGeom<R>;
+    static int grid_cap = 0;
+    static std::once_flag once;
+    static cudaError_t err = cudaSuccess;
+    std::call_once(once, [] {
+        int dev = 0, sms = 0, occ = 0;
+        err = cudaGetDevice(&dev);
+        if (err == cudaSuccess) err = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
+        if (err == cudaSuccess)
+            err = cudaFuncSetAttribute(me_sad_kernel<R>, cudaFuncAttributeMaxDynamicSharedMemorySize, G::kSmem);
+        if (err == cudaSuccess)
+            err = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, me_sad_kernel<R>, G::kThreads, G::kSmem);
+        grid_cap = sms * (occ > 0 ? occ : 1);
+    });
+    SP_CUDA_TRY(err);
+    const int grid = (int)(total < grid_cap ? total : grid_cap);
+    me_sad_kernel<R><<<grid, G::kThreads, G::kSmem, s>>>(rm, cm, a);
+    return SP_OK;
+}
+
 }  // namespace
 
 extern "C" int sp_me_ref_window(int32_t width, int32_t frame_height, int32_t range, int32_t bx, int32_t by,
@@ -352,26 +472,19 @@ extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t 
     const int rows = mb_row_end - mb_row_begin;
     if (n_pairs == 0 || rows == 0 || mbx == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
-    MeArgs a{width, frame_height, row0_global, range, mbx, mb_row_begin, rows, 2 * range + 16, mv, best_sad, surface};
-    dim3 grid(mbx, rows, n_pairs);
+    MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, mv, best_sad, surface};
     if (fast_range(range)) {
         CUtensorMap rm, cm;
         int st;
-        if ((st = make_map(&rm, ref, width, rows_in_buffer, n_pairs, pitch, n_pairs > 1 ? pair_stride : pitch * rows_in_buffer,
-                           (uint32_t)a.win, (uint32_t)a.win)))
+        const int64_t ps = n_pairs > 1 ? pair_stride : pitch * rows_in_buffer;
+        if ((st = make_map(&rm, ref, width, rows_in_buffer, n_pairs, pitch, ps, (uint32_t)a.win, (uint32_t)a.win)))
             return st;
-        if ((st = make_map(&cm, cur, width, rows_in_buffer, n_pairs, pitch, n_pairs > 1 ? pair_stride : pitch * rows_in_buffer,
-                           kMB, kMB)))
-            return st;
-        const int smem = 4 * a.win * a.win + kMB * kMB + 128;
-        static std::once_flag once;
-        static cudaError_t attr_err = cudaSuccess;
-        std::call_once(once, [] {
-            attr_err = cudaFuncSetAttribute(me_sad_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 4 * 80 * 80 + 256 + 128);
-        });
-        SP_CUDA_TRY(attr_err);
-        const int threads = ((range * range / 8) + 31) & ~31;
-        me_sad_kernel<<<grid, threads, smem, s>>>(rm, cm, a);
+        if ((st = make_map(&cm, cur, width, rows_in_buffer, n_pairs, pitch, ps, kMB, kMB))) return st;
+        a.n_pairs = n_pairs;
+        const int64_t total = (int64_t)mbx * rows * n_pairs;
+        if (range == 32) st = launch_fast<32>(rm, cm, a, total, s);
+        else st = launch_fast<16>(rm, cm, a, total, s);
+        if (st) return st;
     } else {
         const int smem = a.win * a.win + kMB * kMB;
         static std::once_flag once;
@@ -380,7 +493,7 @@ extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t 
             attr_err = cudaFuncSetAttribute(me_sad_generic_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 142 * 142 + 256);
         });
         SP_CUDA_TRY(attr_err);
-        me_sad_generic_kernel<<<grid, 256, smem, s>>>(ref, cur, pitch, rows_in_buffer, n_pairs > 1 ? pair_stride : 0, a);
+        me_sad_generic_kernel<<<dim3(mbx, rows, n_pairs), 256, smem, s>>>(ref, cur, pitch, rows_in_buffer, n_pairs > 1 ? pair_stride : 0, a);
     }
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;

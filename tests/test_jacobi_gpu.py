@@ -35,7 +35,7 @@ def test_J1_config():
     want = oracle.jacobi1d(a, 64)
     _check(_run(a, 64, 16), want)
     _check(_run(a, 64, 16, 256), want)
-    _check(_run(a, 64, 16, 1024), want)
+    _check(_run(a, 64, 16, 512), want)
 
 
 @pytest.mark.parametrize("n", [3, 4, 5, 7, 31, 32, 33, 63, 64, 65, 131, 1000, 4097])
@@ -52,7 +52,8 @@ def test_time_tiles(tt):
     a = sp_inputs.jacobi_input(20000, seed=tt)
     want = oracle.jacobi1d(a, 70)
     _check(_run(a, 70, tt), want)
-    _check(_run(a, 70, tt, 1000), want)
+    S = sp.jacobi1d_plan(20000, 70, tt, 0)["space_tile"]
+    _check(_run(a, 70, tt, max(4, (S // 3) & ~3)), want)
 
 
 def test_fixed_points_on_gpu():
@@ -96,7 +97,7 @@ def test_J3_size_sampled():
     rng = np.random.default_rng(0)
     idx = [0, 1, 2, n - 3, n - 2, n - 1]
     for t in [0, 1, 7, 1000, (n // S) - 1, n // S]:
-        for off in (-1, 0, 1, 991, 992, 993):
+        for off in (-1, 0, 1, S // 2, S - 1, S + 1):
             i = t * S + off
             if 0 <= i < n:
                 idx.append(i)
@@ -123,7 +124,7 @@ def test_loopback_partition_equals_oracle(P):
         buf[lo - (xb - H): hi - (xb - H)] = torch.from_numpy(a[lo:hi]).cuda()
         locs.append(buf)
         works.append(torch.zeros_like(buf))
-    sp.jacobi1d_timetiled_loopback(locs, works, n, [s[0] for s in slabs], [s[1] for s in slabs], steps, tt, 2048)
+    sp.jacobi1d_timetiled_loopback(locs, works, n, [s[0] for s in slabs], [s[1] for s in slabs], steps, tt, 256)
     torch.cuda.synchronize()
     got = np.concatenate([locs[r][H:H + slabs[r][1]].cpu().numpy() for r in range(P)])
     _check(got, want)

@@ -4,6 +4,7 @@
 #include <cstdio>
 #include <cstdint>
 #include <cuda_runtime.h>
+#include <cstdlib>
 
 #define CK(x) do { cudaError_t e = (x); if (e != cudaSuccess) { printf("CUDA %s @%d\n", cudaGetErrorString(e), __LINE__); return 1; } } while (0)
 
@@ -21,7 +22,7 @@ __device__ __forceinline__ unsigned long long f2mul(unsigned long long a, unsign
 }
 
 template <int KIND>
-__global__ void __launch_bounds__(256) kbench(float seedf, unsigned seedu) {
+__global__ void __launch_bounds__(256, 4) kbench(float seedf, unsigned seedu) {
   long long t0 = clock64();
   float f[CH]; unsigned u[CH]; unsigned long long p[CH];
   #pragma unroll
@@ -31,6 +32,7 @@ __global__ void __launch_bounds__(256) kbench(float seedf, unsigned seedu) {
   }
   const float w = 0.33333334f;
   const unsigned long long w2 = ((unsigned long long)__float_as_uint(w) << 32) | __float_as_uint(w);
+  const unsigned long long mzr = (unsigned long long)seedu << 63 | ((unsigned long long)seedu << 31);
   for (int it = 0; it < ITERS; ++it) {
     #pragma unroll
     for (int c = 0; c < CH; ++c) {
@@ -54,6 +56,10 @@ __global__ void __launch_bounds__(256) kbench(float seedf, unsigned seedu) {
         f[c] = __fmul_rn(__fadd_rn(__fadd_rn(f[c], f[(c + 1) % CH]), f[(c + 2) % CH]), w);
       } else if (KIND == 9) {   // Jacobi update packed f32x2 (3 FP2 ops = 6 flops)
         p[c] = f2mul(f2add(f2add(p[c], p[(c + 1) % CH]), p[(c + 2) % CH]), w2);
+      } else if (KIND == 11) {  // Jacobi packed exactly as the kernel: FADD2, FADD2, FFMA2(x, w, -0 reg)
+        unsigned long long d;
+        asm volatile("fma.rn.f32x2 %0, %1, %2, %3;" : "=l"(d) : "l"(f2add(f2add(p[c], p[(c + 1) % CH]), p[(c + 2) % CH])), "l"(w2), "l"(mzr));
+        p[c] = d;
       } else if (KIND == 10) {  // mixed: VABSDIFF4 + FADD in parallel pipes
         unsigned d; asm volatile("vabsdiff4.u32.u32.u32.add %0, %1, %2, %3;" : "=r"(d) : "r"(u[(c + 3) % CH]), "r"(seedu ^ c), "r"(u[c])); u[c] = d;
         f[c] = __fadd_rn(f[c], f[(c + 1) % CH]);
@@ -92,11 +98,11 @@ int run(const char* name, double ops_per_inner, int blocks) {
   return 0;
 }
 
-int main() {
+int main(int argc, char** argv) {
   int nsm; cudaDeviceGetAttribute(&nsm, cudaDevAttrMultiProcessorCount, 0);
   cudaDeviceProp pr; cudaGetDeviceProperties(&pr, 0);
   printf("device %s  SMs %d  smem/SM %zu  regs/SM %d  cc %d.%d\n", pr.name, nsm, pr.sharedMemPerMultiprocessor, pr.regsPerMultiprocessor, pr.major, pr.minor);
-  int blocks = nsm * 8;  // 8 x 256 threads = 64 warps/SM
+  int blocks = nsm * (argc > 1 ? atoi(argv[1]) : 4);  // one resident wave (4 x 256 threads/SM)
   run<0>("FADD r,r", 1, blocks);
   run<1>("FMUL r,imm", 1, blocks);
   run<2>("FADD2 (x2 flops)", 2, blocks);
@@ -108,5 +114,6 @@ int main() {
   run<8>("jacobi unpacked (updates)", 1, blocks);
   run<9>("jacobi f32x2 (updates)", 2, blocks);
   run<10>("vabsdiff4 bytes (+FADD mix)", 4, blocks);
+  run<11>("jacobi f32x2 as kernel (upd)", 2, blocks);
   return 0;
 }

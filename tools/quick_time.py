@@ -40,6 +40,8 @@ def main():
         ups = (n - 2) * T / (t * 1e-3)
         print(f"jacobi N=2^26 T={T} Tt={tt}: {t:.3f} ms  {ups/1e9:.1f} GUpd/s  "
               f"HBM-alg {8.0*(n)*(T/tt)/(t*1e-3)/1e9:.0f} GB/s  plan={sp.jacobi1d_plan(n, T, tt, 0)}", flush=True)
+    if '--no-me' in sys.argv:
+        return
     W, H, R, F = 1920, 1080, 32, 65
     t0 = time.time()
     fr = torch.from_numpy(sp_inputs.me_sequence(F, W, H, R)).cuda()
