@@ -67,26 +67,33 @@ struct PassArgs {
     uint64_t mz;       // (-0.0f, -0.0f), opaque to ptxas (see f2_mul_nofuse)
 };
 
-// One Jacobi step on the thread's 2K cells, P -> Q (out of place, so the step loop needs
-// no register copies).  The lane neighbours come from four shuffles.
+// Lane neighbours of a thread's 2K cells: four shuffles.  The v strip continues the u strip:
+// lane 0's v-left is lane 31's last u and lane 31's u-right is lane 0's first v.
 template <int kK>
-__device__ __forceinline__ void step(const uint64_t (&P)[kK], uint64_t (&Q)[kK], int lane, uint64_t w2, uint64_t mz) {
-    const float ul = f2_lo(P[kK - 1]), vl = f2_hi(P[kK - 1]);
-    const float uf = f2_lo(P[0]), vf = f2_hi(P[0]);
-    const float a = __shfl_sync(0xffffffffu, ul, (lane + 31) & 31);  // lane-1's last u
-    const float b = __shfl_sync(0xffffffffu, vl, (lane + 31) & 31);  // lane-1's last v
-    const float c = __shfl_sync(0xffffffffu, uf, (lane + 1) & 31);   // lane+1's first u
-    const float d = __shfl_sync(0xffffffffu, vf, (lane + 1) & 31);   // lane+1's first v
-    // the v strip continues the u strip: lane 0's v-left is lane 31's last u and
-    // lane 31's u-right is lane 0's first v
-    const uint64_t left = f2_pack(a, lane == 0 ? a : b);
-    const uint64_t right = f2_pack(lane == 31 ? d : c, d);
+__device__ __forceinline__ void neighbours(uint64_t first, uint64_t last, int lane, uint64_t& left, uint64_t& right) {
+    const float a = __shfl_sync(0xffffffffu, f2_lo(last), (lane + 31) & 31);   // lane-1's last u
+    const float b = __shfl_sync(0xffffffffu, f2_hi(last), (lane + 31) & 31);   // lane-1's last v
+    const float c = __shfl_sync(0xffffffffu, f2_lo(first), (lane + 1) & 31);   // lane+1's first u
+    const float d = __shfl_sync(0xffffffffu, f2_hi(first), (lane + 1) & 31);   // lane+1's first v
+    left = f2_pack(a, lane == 0 ? a : b);
+    right = f2_pack(lane == 31 ? d : c, d);
+}
+
+__device__ __forceinline__ uint64_t update(uint64_t l, uint64_t c, uint64_t r, uint64_t w2, uint64_t mz) {
+    return f2_mul_nofuse(f2_add(f2_add(l, c), r), w2, mz);
+}
+
+// One Jacobi step on the thread's 2K cells, P -> Q (out of place: no register copies).  The
+// two edge pairs are computed first and their shuffles for the NEXT step are issued before
+// the interior, so the shuffle latency hides under the interior arithmetic.
+template <int kK>
+__device__ __forceinline__ void step(const uint64_t (&P)[kK], uint64_t (&Q)[kK], uint64_t& left, uint64_t& right,
+                                     int lane, uint64_t w2, uint64_t mz) {
+    Q[0] = update(left, P[0], P[1], w2, mz);
+    Q[kK - 1] = update(P[kK - 2], P[kK - 1], right, w2, mz);
+    neighbours<kK>(Q[0], Q[kK - 1], lane, left, right);
 #pragma unroll
-    for (int j = 0; j < kK; ++j) {
-        const uint64_t prv = (j > 0) ? P[j - 1] : left;
-        const uint64_t nxt = (j + 1 < kK) ? P[j + 1] : right;
-        Q[j] = f2_mul_nofuse(f2_add(f2_add(prv, P[j]), nxt), w2, mz);
-    }
+    for (int j = 1; j < kK - 1; ++j) Q[j] = update(P[j - 1], P[j], P[j + 1], w2, mz);
 }
 
 // Global cells 0 and n-1 are fixed (Dirichlet): in the (rare) warp strips that contain
@@ -105,22 +112,30 @@ __device__ __forceinline__ void restore(uint64_t (&Q)[kK], uint64_t f0, uint64_t
     }
 }
 
-// h steps, ping-ponging between two register arrays.  `boundary` is warp-uniform; the
-// restore sits outside the shuffles so they stay in converged code.
-template <int kK>
-__device__ __forceinline__ void run_steps(uint64_t (&P)[kK], int h, int lane, uint64_t w2, uint64_t mz, bool boundary,
-                                          uint64_t f0, uint64_t fn, float v0, float vn) {
+// h steps, ping-ponging between two register arrays.  kBoundary (warp-uniform, chosen per
+// tile) adds the Dirichlet restore; the common path carries no boundary code at all.
+template <bool kBoundary, int kK>
+__device__ __forceinline__ void run_steps(uint64_t (&P)[kK], int h, int lane, uint64_t w2, uint64_t mz, uint64_t f0,
+                                          uint64_t fn, float v0, float vn) {
     uint64_t Q[kK];
+    uint64_t left, right;
+    neighbours<kK>(P[0], P[kK - 1], lane, left, right);
     int k = 0;
     for (; k + 2 <= h; k += 2) {
-        step(P, Q, lane, w2, mz);
-        if (boundary) restore(Q, f0, fn, v0, vn);
-        step(Q, P, lane, w2, mz);
-        if (boundary) restore(P, f0, fn, v0, vn);
+        step(P, Q, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore(Q, f0, fn, v0, vn);
+            neighbours<kK>(Q[0], Q[kK - 1], lane, left, right);
+        }
+        step(Q, P, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore(P, f0, fn, v0, vn);
+            neighbours<kK>(P[0], P[kK - 1], lane, left, right);
+        }
     }
     if (k < h) {
-        step(P, Q, lane, w2, mz);
-        if (boundary) restore(Q, f0, fn, v0, vn);
+        step(P, Q, left, right, lane, w2, mz);
+        if (kBoundary) restore(Q, f0, fn, v0, vn);
 #pragma unroll
         for (int j = 0; j < kK; ++j) P[j] = Q[j];
     }
@@ -225,7 +240,8 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
                 if (0 >= base) v0 = buf[0 - base];
                 if (A.n - 1 - base < kStrip) vn = buf[A.n - 1 - base];
             }
-            run_steps(P, A.h, lane, w2, A.mz, boundary, f0, fn, v0, vn);
+            if (boundary) run_steps<true>(P, A.h, lane, w2, A.mz, f0, fn, v0, vn);
+            else run_steps<false>(P, A.h, lane, w2, A.mz, 0ull, 0ull, 0.f, 0.f);
         }
         // ---- owned cells -> staged buffer -> TMA bulk store ------------------------------
         {
@@ -276,15 +292,15 @@ Variant make_variant() {
 }
 
 constexpr int kNumVariants = 5;
-constexpr int kDefaultVariant = 1;
+constexpr int kDefaultVariant = 0;
 
 Variant* variants() {
     static Variant v[kNumVariants] = {
-        make_variant<JCfg<12, 4, 8>>(),  // 0: 24 cells/lane, 4 warps/CTA, <= 64 regs
-        make_variant<JCfg<12, 8, 4>>(),  // 1: 24 cells/lane, 8 warps/CTA
-        make_variant<JCfg<20, 4, 5>>(),  // 2: 40 cells/lane
-        make_variant<JCfg<28, 4, 4>>(),  // 3: 56 cells/lane
-        make_variant<JCfg<12, 4, 6>>(),  // 4: 24 cells/lane, <= 85 regs
+        make_variant<JCfg<20, 8, 2>>(),  // 0: 40 cells/lane, 8 warps/CTA, <= 128 regs
+        make_variant<JCfg<12, 8, 3>>(),  // 1: 24 cells/lane, 8 warps/CTA, <= 85 regs
+        make_variant<JCfg<20, 4, 4>>(),  // 2: 40 cells/lane, <= 128 regs
+        make_variant<JCfg<28, 4, 4>>(),  // 3: 56 cells/lane, <= 128 regs
+        make_variant<JCfg<20, 2, 8>>(),  // 4: 40 cells/lane, 2 warps/CTA, <= 128 regs
     };
     return v;
 }
