@@ -260,6 +260,21 @@ int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_locals, int32_
 /* ncclAllGather of `bytes` per rank (device buffers) — used for the ME results. */
 int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream);
 
+/* =====================================================================================
+ * 5. Ablation baselines: the paper's "GPU w/o scratchpad memory"
+ *    versions (Figs. 4-5), same arithmetic and results, no on-chip staging.
+ * ===================================================================================== */
+/* Jacobi without staging or time tiling: one launch per time step, operands read from
+ * global memory.  Same contract as sp_jacobi1d_timetiled (a, work device, n >= 3). */
+int sp_jacobi1d_untiled(float* a, float* work, int64_t n, int32_t steps, void* stream);
+/* ME without staging: one CTA per macroblock, candidates read straight from global memory.
+ * Same arguments and outputs as sp_me_sad_search; pitch, bases and pair_stride need only
+ * 4-byte alignment. */
+int sp_me_sad_search_direct(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                            int32_t rows_in_buffer, int32_t row0_global, int32_t frame_height, int32_t n_pairs,
+                            int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
+                            int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream);
+
 #ifdef __cplusplus
 }
 #endif

@@ -99,6 +99,9 @@ SYMBOLS = {
     "sp_jacobi1d_timetiled_loopback": (ctypes.c_int, [ctypes.POINTER(vp), ctypes.POINTER(vp), i32, i64,
                                                       ctypes.POINTER(i64), ctypes.POINTER(i64), i32, i32, i32, vp]),
     "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
+    "sp_jacobi1d_untiled": (ctypes.c_int, [vp, vp, i64, i32, vp]),
+    "sp_me_sad_search_direct": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp,
+                                               vp, vp]),
 }
 
 
@@ -240,6 +243,15 @@ def jacobi1d_timetiled(a, steps: int, time_tile: int = 16, space_tile: int = 0, 
     return a
 
 
+def jacobi1d_untiled(a, steps: int, work=None, stream=None):
+    """N1 ablation: no staging, no time tiling (one launch per step).  In place on a[n]."""
+    import torch
+    if work is None:
+        work = torch.empty_like(a)
+    _check(lib.sp_jacobi1d_untiled(_ptr(a), _ptr(work), a.numel(), int(steps), _stream(stream)), "sp_jacobi1d_untiled")
+    return a
+
+
 def jacobi1d_pass_segment(src, dst, n_global: int, g0: int, own_begin: int, own_end: int, h: int, time_tile: int,
                           space_tile: int = 0, stream=None):
     _check(lib.sp_jacobi1d_pass_segment(_ptr(src), _ptr(dst), int(n_global), int(g0), src.numel(), int(own_begin),
@@ -307,6 +319,32 @@ def me_sad_search(ref, cur, width: int, frame_height: int, search_range: int, *,
                                 int(frame_height), int(n_pairs), int(pair_stride), 16, int(search_range),
                                 int(mb_row_begin), int(mb_row_end), _ptr(mv), _ptr(sad), _ptr(surf), _stream(stream)),
            "sp_me_sad_search")
+    return mv, sad, surf
+
+
+def me_sad_search_direct(ref, cur, width: int, frame_height: int, search_range: int, *, row0: int = 0,
+                         mb_row_begin: int = 0, mb_row_end: int | None = None, with_surface: bool = False,
+                         out=None, stream=None):
+    """N1 ablation: same as me_sad_search, candidates read straight from global memory."""
+    import torch
+    n_pairs, rows_in_buffer, _ = ref.shape
+    pitch = ref.stride(1)
+    pair_stride = ref.stride(0) if n_pairs > 1 else pitch * rows_in_buffer
+    mbx = width // 16
+    if mb_row_end is None:
+        mb_row_end = frame_height // 16
+    rows = mb_row_end - mb_row_begin
+    side = 2 * search_range + 1
+    if out is None:
+        mv = torch.empty((n_pairs, rows, mbx, 2), dtype=torch.int16, device=ref.device)
+        sad = torch.empty((n_pairs, rows, mbx), dtype=torch.int32, device=ref.device)
+        surf = torch.empty((n_pairs, rows, mbx, side * side), dtype=torch.int32, device=ref.device) if with_surface else None
+    else:
+        mv, sad, surf = out
+    _check(lib.sp_me_sad_search_direct(_ptr(ref), _ptr(cur), pitch, int(width), int(rows_in_buffer), int(row0),
+                                       int(frame_height), int(n_pairs), int(pair_stride), 16, int(search_range),
+                                       int(mb_row_begin), int(mb_row_end), _ptr(mv), _ptr(sad), _ptr(surf),
+                                       _stream(stream)), "sp_me_sad_search_direct")
     return mv, sad, surf
 
 

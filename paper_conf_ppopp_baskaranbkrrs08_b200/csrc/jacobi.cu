@@ -47,7 +47,6 @@ struct JCfg {
     static constexpr int kStage = WARPS_ * 2 * 64 * K_;  // floats of shared memory per CTA
     static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && K_ <= 32, "K/4 must be odd, K <= 32");
 };
-constexpr int kStages = 2;
 constexpr int kMaxTimeTile = 128;
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
 constexpr uint64_t kNegZero2 = 0x8000000080000000ull;

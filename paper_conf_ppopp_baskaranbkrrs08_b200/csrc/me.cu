@@ -39,7 +39,6 @@ using namespace sp::ptx;
 constexpr int kMB = 16;      // macroblock edge (WS = 16)
 constexpr int kTy = 8;       // dy candidates per thread
 constexpr int kTx = 4;       // dx candidates per thread (same byte phase, stride 4)
-constexpr int kRows = kTy + kMB - 1;  // window rows a thread sweeps (23)
 
 struct MeArgs {
     int32_t width, frame_height, row0, range, n_pairs;
@@ -74,9 +73,8 @@ struct MeGeom {
     static constexpr int kGx = R / 8;                    // dx groups per byte phase
     static constexpr int kPhStride = kCopy + 32;         // phase copies at 32-byte bank offsets
     static constexpr int kOffCur = 2 * kCopy;            // cur[2] after raw[2]
-    static constexpr int kOffPh = 2 * kCopy + 512 + 32;  // stage s, copy p at kOffPh + s*kPhSet + (p-1)*kPhStride
-    static constexpr int kPhSet = 3 * kPhStride + 32;    // keeps copy p of both stages at 32p mod 128
-    static constexpr int kSmem = kOffPh + 2 * kPhSet + 128;  // + alignment slack
+    static constexpr int kOffPh = 2 * kCopy + 512 + 32;  // copy p at kOffPh + (p-1)*kPhStride
+    static constexpr int kSmem = kOffPh + 3 * kPhStride + 128;  // + alignment slack
     static constexpr int kTail = 4 * R + 1;
 };
 
@@ -87,11 +85,13 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     constexpr int win = G::kWin;
     extern __shared__ __align__(128) uint8_t smem_raw[];
     __shared__ __align__(8) uint64_t full[2];
-    __shared__ unsigned long long keyslot[2];  // per-stage argmin key (block-wide atomicMin)
+    __shared__ uint32_t red32[32];
+    __shared__ uint64_t red64[32];
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
 
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+    constexpr int nwarps = (G::kThreads + 31) / 32;
     const int mbx = A.mbx;
     const int64_t per_pair = (int64_t)A.mb_rows * mbx;
     const int64_t total = per_pair * A.n_pairs;
@@ -115,22 +115,12 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         mbar_init(&full[0], 1);
         mbar_init(&full[1], 1);
         fence_mbar_init();
-        keyslot[0] = keyslot[1] = ~0ull;
     }
     __syncthreads();
-    if (tid == 0 && blockIdx.x < total) issue(blockIdx.x, 0);
-
-    // tid 0: publish the argmin of macroblock `mbp` (key in keyslot[sp]) and reset the slot
-    auto finalize = [&](int64_t mbp, int sp) {
-        const uint64_t b = keyslot[sp];
-        keyslot[sp] = ~0ull;
-        const int pr = (int)(mbp / per_pair);
-        const int64_t rm = mbp - (int64_t)pr * per_pair;
-        const size_t idx = ((size_t)pr * A.mb_rows + (size_t)(rm / mbx)) * mbx + (size_t)(rm % mbx);
-        A.mv[2 * idx] = (int16_t)((int)(b & 127) - R);
-        A.mv[2 * idx + 1] = (int16_t)((int)((b >> 7) & 127) - R);
-        A.sad[idx] = (uint32_t)(b >> 21);
-    };
+    if (tid == 0) {
+        if (blockIdx.x < total) issue(blockIdx.x, 0);
+        if (blockIdx.x + Gs < total) issue(blockIdx.x + Gs, 1);
+    }
 
     // thread's candidate tile: dx = -R + p + 4*(4g + j), dy = -R + 8d + i
     const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
@@ -159,18 +149,11 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     o.y = __funnelshift_r(w.y, w.z, 8 * q);
                     o.z = __funnelshift_r(w.z, w.w, 8 * q);
                     o.w = __funnelshift_r(w.w, nx, 8 * q);
-                    reinterpret_cast<uint4*>(smem + G::kOffPh + s * G::kPhSet + (q - 1) * G::kPhStride + r * win)[c] = o;
+                    reinterpret_cast<uint4*>(smem + G::kOffPh + (q - 1) * G::kPhStride + r * win)[c] = o;
                 }
             }
         }
-        __syncthreads();  // phase copies of stage s complete; every warp is done with the previous MB
-        if (tid == 0) {
-            if (it > 0) finalize(mb - Gs, s ^ 1);
-            if (mb + Gs < total) {
-                fence_proxy_async_smem();
-                issue(mb + Gs, s ^ 1);  // next MB streams in while this one is searched
-            }
-        }
+        __syncthreads();  // phase copies complete
 
         // ---- main 2R x 2R candidates: 4 dx (one byte phase) x 8 dy per thread ----------
         uint32_t acc[kTx][kTy];
@@ -184,7 +167,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             // 4 dx candidates x 4 words of one byte phase); body unrolled 8x so every ring
             // index is static, outer loop rolled to halve the code (I-cache).  Innermost
             // order (k, i, j) makes consecutive VABSDIFF4s independent.
-            const uint8_t* base = (p == 0) ? raw : smem + G::kOffPh + s * G::kPhSet + (p - 1) * G::kPhStride;
+            const uint8_t* base = (p == 0) ? raw : smem + G::kOffPh + (p - 1) * G::kPhStride;
             const uint8_t* rowp = base + (kTy * d) * win + 16 * g;
             const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
             uint32_t Rw[8][7];  // words 4g..4g+6 (j + k <= 6)
@@ -230,7 +213,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 const int dx = (c < side) ? R : -R + (c - side);
                 const int dy = (c < side) ? -R + c : R;
                 const int pp = (dx + R) & 3, m = (dx + R) >> 2;
-                const uint8_t* cb = (pp == 0) ? raw : smem + G::kOffPh + s * G::kPhSet + (pp - 1) * G::kPhStride;
+                const uint8_t* cb = (pp == 0) ? raw : smem + G::kOffPh + (pp - 1) * G::kPhStride;
                 const uint32_t* rw = reinterpret_cast<const uint32_t*>(cb + (dy + R) * win) + m;
                 a = 0;
 #pragma unroll
@@ -286,24 +269,23 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 }
             }
         }
-        // ---- argmin (SAD, |dx|+|dy|, dy, dx): warp min of SAD (tree, then CREDUX), the
-        //      tie-break key only for the warp's candidates that reach it, block-wide
-        //      atomicMin of the 64-bit keys (invalid candidates hold 0xFFFFFFFF) ----------
-        uint32_t t32[kTx * kTy];
+        // ---- argmin (SAD, |dx|+|dy|, dy, dx): block min of SAD, then the tie-break key
+        //      only among candidates that reach it (invalid candidates hold 0xFFFFFFFF) ----
+        uint32_t m = 0xffffffffu;
 #pragma unroll
         for (int j = 0; j < kTx; ++j)
 #pragma unroll
-            for (int i = 0; i < kTy; ++i) t32[j * kTy + i] = acc[j][i];
-#pragma unroll
-        for (int w = kTx * kTy / 2; w >= 1; w /= 2)
-#pragma unroll
-            for (int q = 0; q < w; ++q) t32[q] = min(t32[q], t32[q + w]);
-        uint32_t m = t32[0];
+            for (int i = 0; i < kTy; ++i) m = min(m, acc[j][i]);
 #pragma unroll
         for (int t = 0; t < kTailPer; ++t) m = min(m, tacc[t]);
-        const uint32_t M = __reduce_min_sync(0xffffffffu, m);
+        const uint32_t wm = __reduce_min_sync(0xffffffffu, m);
+        if (lane == 0) red32[warp] = wm;
+        __syncthreads();
+        uint32_t M = red32[0];
+#pragma unroll
+        for (int w = 1; w < nwarps; ++w) M = min(M, red32[w]);
         uint64_t key = ~0ull;
-        if (m == M) {  // rare: only lanes holding the warp's minimal SAD
+        if (m == M) {  // rare: only threads holding a minimal candidate
 #pragma unroll
             for (int j = 0; j < kTx; ++j)
 #pragma unroll
@@ -322,10 +304,19 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
         }
         key = warp_min_key(key);
-        if (lane == 0) atomicMin(&keyslot[s], (unsigned long long)key);
+        if (lane == 0) red64[warp] = key;
+        __syncthreads();  // also: every thread is done with raw[s], cur[s] and the phases
+        if (tid == 0) {
+            uint64_t b = red64[0];
+#pragma unroll
+            for (int w = 1; w < nwarps; ++w) b = red64[w] < b ? red64[w] : b;
+            A.mv[2 * mb_index] = (int16_t)((int)(b & 127) - R);
+            A.mv[2 * mb_index + 1] = (int16_t)((int)((b >> 7) & 127) - R);
+            A.sad[mb_index] = (uint32_t)(b >> 21);
+            fence_proxy_async_smem();
+            if (mb + 2 * Gs < total) issue(mb + 2 * Gs, s);
+        }
     }
-    __syncthreads();
-    if (tid == 0 && it > 0) finalize(blockIdx.x + (int64_t)(it - 1) * Gs, (it - 1) & 1);
 }
 
 // Generic path (any 0 <= R <= 63): window staged byte-wise with zero fill, one thread per

@@ -17,7 +17,7 @@ if what == "jacobi":
     sp.jacobi1d_timetiled(a, 4 * tt, tt, 0, work=w)  # 4 launches
 else:
     W, H, R = 1920, 1080, 32
-    fr = torch.from_numpy(sp_inputs.me_sequence(9, W, H, R)).cuda()
+    fr = torch.from_numpy(sp_inputs.me_sequence(65, W, H, R)).cuda()  # the bench launch: 64 pairs
     for _ in range(2):
         sp.me_search_sequence(fr, W, H, R)
 torch.cuda.synchronize()
