@@ -261,6 +261,43 @@ int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_locals, int32_
 int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream);
 
 /* =====================================================================================
+ * 6. Tile-size search (§4.3).  Minimise the paper's
+ *    data-movement cost over a grid of candidate tile vectors t (one list per loop):
+ *      C(t) = sum_{k in I} prod_{i<=r_k} ceil(N_i/t_i) (P S + V_in_k(t) L / P)
+ *           + sum_{k in O} prod_{i<=r_k} ceil(N_i/t_i) (P S + V_out_k(t) L / P)
+ *    subject to 0 < t_i <= N_i, sum_k M_k(t) <= M_up, prod t_i >= P.  The tile
+ *    is the box 0 <= i_l < t_l of a perfectly nested band; M_k, V_in_k, V_out_k come from
+ *    Alg. 2 (sp_plan_buffers, PER_ARRAY) on that box; r_k is the deepest loop array k's
+ *    references depend on (movement hoisted above redundant loops, §4.2).  The paper
+ *    solves the real relaxation by SQP and rounds; this evaluates the exact
+ *    objective on the grid.  Host-only.
+ * ===================================================================================== */
+typedef struct {
+    int32_t depth;          /* m: loops of the band, outermost first (<= SP_MAX_DEPTH) */
+    int32_t n_refs;
+    const int64_t* extent;  /* [m] N_i (loop trip counts) */
+    const sp_ref* refs;     /* rows [rank][m + 1] over the tile-local iterators (stmt ignored) */
+    const int32_t* n_cand;  /* [m] number of candidate sizes per loop */
+    const int64_t* cand;    /* concatenated candidate sizes (each in [1, N_i]) */
+    int64_t mup_elems;      /* M_up in elements; 0 = unlimited */
+    int32_t procs;          /* P: inner-level parallel processes per outer process */
+    int32_t reserved;       /* must be 0 */
+    double sync_cost;       /* S: synchronisation cost per process per movement */
+    double elem_cost;       /* L: cost of moving one element */
+} sp_tile_problem;
+
+typedef struct {
+    int64_t tile[SP_MAX_DEPTH]; /* argmin t */
+    double cost;                /* C(t) */
+    int64_t local_elems;        /* sum_k M_k(t) */
+    int64_t evaluated;          /* candidates evaluated (prod t_i >= P) */
+    int32_t feasible;           /* 0: no candidate met the constraints */
+    int32_t reserved;
+} sp_tile_result;
+
+int sp_tile_search(const sp_tile_problem* prob, sp_tile_result* out);
+
+/* =====================================================================================
  * 5. Ablation baselines: the paper's "GPU w/o scratchpad memory"
  *    versions (Figs. 4-5), same arithmetic and results, no on-chip staging.
  * ===================================================================================== */

@@ -79,6 +79,17 @@ class sp_jacobi_plan(ctypes.Structure):
                 ("tiles", i64), ("grid", i32), ("threads", i32), ("smem_bytes", i32), ("cells_per_thread", i32)]
 
 
+class sp_tile_problem(ctypes.Structure):
+    _fields_ = [("depth", i32), ("n_refs", i32), ("extent", ctypes.POINTER(i64)), ("refs", ctypes.POINTER(sp_ref)),
+                ("n_cand", ctypes.POINTER(i32)), ("cand", ctypes.POINTER(i64)), ("mup_elems", i64), ("procs", i32),
+                ("reserved", i32), ("sync_cost", f64), ("elem_cost", f64)]
+
+
+class sp_tile_result(ctypes.Structure):
+    _fields_ = [("tile", i64 * 8), ("cost", f64), ("local_elems", i64), ("evaluated", i64), ("feasible", i32),
+                ("reserved", i32)]
+
+
 SYMBOLS = {
     "sp_status_string": (ctypes.c_char_p, [ctypes.c_int]),
     "sp_last_cuda_error": (ctypes.c_int, []),
@@ -100,6 +111,7 @@ SYMBOLS = {
                                                       ctypes.POINTER(i64), ctypes.POINTER(i64), i32, i32, i32, vp]),
     "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
     "sp_jacobi1d_untiled": (ctypes.c_int, [vp, vp, i64, i32, vp]),
+    "sp_tile_search": (ctypes.c_int, [ctypes.POINTER(sp_tile_problem), ctypes.POINTER(sp_tile_result)]),
     "sp_me_sad_search_direct": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp,
                                                vp, vp]),
 }
@@ -213,6 +225,30 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
         out["local_rows"].append([list(local[pos + k * w: pos + (k + 1) * w]) for k in range(rk)])
         pos += rk * w
     return out
+
+
+def tile_search(extent, refs, candidates, mup_elems: int = 0, procs: int = 32, sync_cost: float = 1.0,
+                elem_cost: float = 1.0) -> dict:
+    """sp_tile_search (§4.3).  extent: [m] trip counts; refs: [{"array", "is_write", "rank",
+    "rows" [rank][m+1]}] over tile-local iterators; candidates: per loop, a list of sizes."""
+    m = len(extent)
+    ext = np.ascontiguousarray(np.asarray(extent, dtype=np.int64))
+    keep = []
+    rr = (sp_ref * len(refs))()
+    for k, r in enumerate(refs):
+        rows = np.ascontiguousarray(np.asarray(r["rows"], dtype=np.int64))
+        keep.append(rows)
+        rr[k] = sp_ref(0, int(r["array"]), int(bool(r["is_write"])), int(r["rank"]),
+                       rows.ctypes.data_as(ctypes.POINTER(i64)))
+    nc = (i32 * m)(*[len(c) for c in candidates])
+    flat = np.ascontiguousarray(np.asarray([x for c in candidates for x in c], dtype=np.int64))
+    prob = sp_tile_problem(m, len(refs), ext.ctypes.data_as(ctypes.POINTER(i64)), rr, nc,
+                           flat.ctypes.data_as(ctypes.POINTER(i64)), int(mup_elems), int(procs), 0, float(sync_cost),
+                           float(elem_cost))
+    res = sp_tile_result()
+    _check(lib.sp_tile_search(ctypes.byref(prob), ctypes.byref(res)), "sp_tile_search")
+    return {"tile": list(res.tile[:m]), "cost": res.cost, "local_elems": res.local_elems, "evaluated": res.evaluated,
+            "feasible": bool(res.feasible)}
 
 
 # ---------------------------------------------------------------------------------------

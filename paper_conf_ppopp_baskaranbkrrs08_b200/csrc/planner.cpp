@@ -587,3 +587,118 @@ extern "C" int sp_plan_buffers(const sp_block* blk, const sp_plan_opts* opts, sp
         return SP_ERR_UNSUPPORTED;  // e.g. std::bad_alloc on an enormous block
     }
 }
+
+// ---------------------------------------------------------------------------------------
+// Tile-size search (§4.3).
+// For every candidate tile vector t the tile's iteration space is the box 0 <= i_l < t_l;
+// Algorithm 2 (plan_impl, PER_ARRAY as in Figure 1) gives each array's local size M_k and
+// move volumes V_in_k / V_out_k (§3.1.3).  Array k's movement code sits under the tiling
+// loops 0..r_k, r_k = the deepest loop any of its references depends on (§4.2 hoisting), so
+// it runs prod_{i<=r_k} ceil(N_i / t_i) times.  The paper relaxes t to reals and uses SQP
+// (P:L788-794); here the objective is evaluated exactly on the caller's candidate grid.
+// ---------------------------------------------------------------------------------------
+namespace {
+
+int tile_search_impl(const sp_tile_problem* pb, sp_tile_result* out) {
+    if (!pb || !out) return SP_ERR_INVALID_ARG;
+    const int m = pb->depth, nr = pb->n_refs;
+    if (m < 1 || m > SP_MAX_DEPTH || nr < 1 || !pb->extent || !pb->refs || !pb->n_cand || !pb->cand || pb->procs < 1 ||
+        pb->mup_elems < 0 || pb->reserved != 0)
+        return SP_ERR_INVALID_ARG;
+    std::vector<std::vector<i64>> cand(m);
+    size_t off = 0;
+    for (int l = 0; l < m; ++l) {
+        if (pb->n_cand[l] < 1 || pb->extent[l] < 1) return SP_ERR_INVALID_ARG;
+        for (int q = 0; q < pb->n_cand[l]; ++q) {
+            const i64 t = pb->cand[off + q];
+            if (t < 1 || t > pb->extent[l]) return SP_ERR_INVALID_ARG;  // 0 < t_i <= N_i
+            cand[l].push_back(t);
+        }
+        off += pb->n_cand[l];
+    }
+    // r_k per array id: deepest loop with a nonzero coefficient in any of its refs
+    std::vector<int> arrays;
+    for (int r = 0; r < nr; ++r) arrays.push_back(pb->refs[r].array);
+    std::sort(arrays.begin(), arrays.end());
+    arrays.erase(std::unique(arrays.begin(), arrays.end()), arrays.end());
+    std::vector<int> rk(arrays.size(), -1);
+    for (int r = 0; r < nr; ++r) {
+        const sp_ref& R = pb->refs[r];
+        if (R.rank < 1 || R.rank > SP_MAX_RANK || !R.rows) return SP_ERR_INVALID_ARG;
+        const size_t a = std::lower_bound(arrays.begin(), arrays.end(), R.array) - arrays.begin();
+        for (int k = 0; k < R.rank; ++k)
+            for (int l = 0; l < m; ++l)
+                if (R.rows[(size_t)k * (m + 1) + l] != 0 && l > rk[a]) rk[a] = l;
+    }
+    std::vector<sp_ref> refs(pb->refs, pb->refs + nr);
+    for (auto& R : refs) R.stmt = 0;
+    std::vector<i64> rows(2 * (size_t)m * (m + 1), 0);
+    sp_domain dom{m, 2 * m, rows.data()};
+    sp_block blk{0, 1, nr, 0, nullptr, &dom, refs.data()};
+    sp_plan_opts opts{SP_PLAN_PER_ARRAY, 0, 0.30, 0, 0};
+    std::vector<sp_buffer> bufs(arrays.size());
+    std::vector<size_t> idx(m, 0);
+    std::memset(out, 0, sizeof(*out));
+    out->cost = 0.0;
+    bool have = false;
+    i64 evaluated = 0;
+    for (;;) {
+        i64 t[SP_MAX_DEPTH];
+        i128 prod = 1;
+        for (int l = 0; l < m; ++l) {
+            t[l] = cand[l][idx[l]];
+            prod *= t[l];
+        }
+        if (prod >= pb->procs) {  // t_1 x ... x t_m >= P
+            for (int l = 0; l < m; ++l) {  // box 0 <= i_l <= t_l - 1
+                i64* r0 = &rows[(size_t)(2 * l) * (m + 1)];
+                i64* r1 = &rows[(size_t)(2 * l + 1) * (m + 1)];
+                std::fill(r0, r0 + m + 1, 0);
+                std::fill(r1, r1 + m + 1, 0);
+                r0[l] = 1;
+                r1[l] = -1;
+                r1[m] = t[l] - 1;
+            }
+            int32_t nb = 0;
+            const int st = plan_impl(&blk, &opts, bufs.data(), (int32_t)bufs.size(), &nb, nullptr, nullptr);
+            if (st) return st;
+            ++evaluated;
+            i128 mem = 0;
+            double cost = 0.0;
+            for (int b = 0; b < nb; ++b) {
+                mem += bufs[b].size;
+                const size_t a = std::lower_bound(arrays.begin(), arrays.end(), bufs[b].array) - arrays.begin();
+                double moves = 1.0;
+                for (int l = 0; l <= rk[a]; ++l) moves *= (double)((pb->extent[l] + t[l] - 1) / t[l]);
+                const double P = (double)pb->procs;
+                if (bufs[b].in_count > 0) cost += moves * (P * pb->sync_cost + (double)bufs[b].v_in_ub * pb->elem_cost / P);
+                if (bufs[b].out_count > 0)
+                    cost += moves * (P * pb->sync_cost + (double)bufs[b].v_out_ub * pb->elem_cost / P);
+            }
+            if ((pb->mup_elems == 0 || mem <= pb->mup_elems) && (!have || cost < out->cost)) {
+                have = true;
+                out->cost = cost;
+                out->local_elems = (i64)mem;
+                for (int l = 0; l < m; ++l) out->tile[l] = t[l];
+            }
+        }
+        int l = m - 1;
+        while (l >= 0 && ++idx[l] == cand[l].size()) idx[l--] = 0;
+        if (l < 0) break;
+    }
+    out->evaluated = evaluated;
+    out->feasible = have ? 1 : 0;
+    return SP_OK;
+}
+
+}  // namespace
+
+extern "C" int sp_tile_search(const sp_tile_problem* prob, sp_tile_result* out) {
+    try {
+        return tile_search_impl(prob, out);
+    } catch (const PlanError& e) {
+        return e.code;
+    } catch (...) {
+        return SP_ERR_UNSUPPORTED;
+    }
+}
