@@ -47,6 +47,15 @@ def me_valid_sads(width, height, r, pairs):
     return tot * pairs
 
 
+def bench_config(world, tt):
+    h = (tt + 3) & ~3
+    return {"workload": f"J3: Jacobi fp32 N=2^26 cells/GPU, T={JAC_T}, time tile {tt} (halo {h}) + "
+                        f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs/GPU",
+            "jacobi_global_n": JAC_N_LOCAL * world, "time_tile": tt, "me_pairs_global": ME_PAIRS * world,
+            "l2": "inputs larger than L2 (256 MiB Jacobi state per GPU, 135 MB frame batch); no flush",
+            "parallelism": f"weak scaling over {world} GPU(s); Jacobi halo exchange per time tile"}
+
+
 def peaks():
     p = {"hbm_gbs": 6650.0, "sm_max_mhz": 1965.0, "source": "fallback (B200_PROFILING.md)"}
     try:
@@ -186,8 +195,8 @@ def run_reference(args, rank, world):
         "impl": "reference", "metric": METRIC, "value": val, "unit": "GPoint-updates/s", "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": tot / max(1, args.steps) * 1e3,
         "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
-        "config": {"workload": "J3 (Jacobi fp32 N=2^26, T=1024) + M4 (ME 1920x1080 +-32 uint8)",
-                   "note": "oracle timed on bounded samples of the workload (see cpu_baseline.sample)"},
+        "config": dict(bench_config(world, args.time_tile),
+                       note="oracle timed on bounded samples of the workload (see cpu_baseline.sample)"),
         "me": {"value": statistics.median(ms) / 1e9, "unit": "GSAD/s"},
         "cpu_baseline": {"value": val, "unit": "GPoint-updates/s", "cores": last["cores"], "kind": "oracle",
                          "sample": last["sample"], "me_value": statistics.median(ms) / 1e9, "me_unit": "GSAD/s"},
@@ -384,13 +393,9 @@ def run_ours(args, rank, world, local_rank):
         "metric": METRIC, "value": round(jac_val, 2), "unit": "GPoint-updates/s", "n_gpus": world, "steps": K,
         "warmup": args.warmup, "ms_per_step": round(total_ms / K, 4), "higher_is_better": True, "scaling": "weak",
         "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
-        "config": {"workload": f"J3: Jacobi fp32 N=2^26 cells/GPU, T={JAC_T}, time tile {tt} (halo {H}) + "
-                               f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs/GPU",
-                   "jacobi_global_n": n_global, "time_tile": tt, "space_tile": plan["space_tile"],
-                   "me_pairs_global": ME_PAIRS * world,
-                   "l2": "inputs larger than L2 (256 MiB Jacobi state per GPU, 135 MB frame batch); no flush",
-                   "parallelism": f"weak scaling over {world} GPU(s); Jacobi halo exchange per time tile"},
-        "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4)},
+        "config": bench_config(world, tt),
+        "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4),
+                   "space_tile": plan["space_tile"], "passes_per_step": plan["passes"]},
         "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
                "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},
         "roofline": dominant, "roofline_jacobi": roof_jac,

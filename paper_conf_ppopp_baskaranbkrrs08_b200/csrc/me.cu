@@ -86,6 +86,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     extern __shared__ __align__(128) uint8_t smem_raw[];
     __shared__ __align__(8) uint64_t full[2];
     __shared__ uint32_t red32[32];
+    __shared__ unsigned int lsum;  // SAD of the leftover tail candidate (dx = R-1, dy = R)
     __shared__ uint64_t red64[32];
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
@@ -153,6 +154,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 }
             }
         }
+        if (tid == 0) lsum = 0u;
         __syncthreads();  // phase copies complete
 
         // ---- main 2R x 2R candidates: 4 dx (one byte phase) x 8 dy per thread ----------
@@ -203,13 +205,16 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
         }
         // ---- tail candidates: column dx = +R (dy in [-R, R]) and row dy = +R (dx < R) ----
-        constexpr int kTailPer = (G::kTail + G::kThreads - 1) / G::kThreads;
+        // 4R of the 4R+1 tail candidates spread evenly over the threads; the last one
+        // (dx = R-1, dy = R) is split one 4-pixel word per lane across the warps so that
+        // no warp carries extra work into the reduction barrier
+        constexpr int kTailPer = (G::kTail - 1 + G::kThreads - 1) / G::kThreads;
         uint32_t tacc[kTailPer];
 #pragma unroll
         for (int t = 0; t < kTailPer; ++t) {
             const int c = tid + t * G::kThreads;
             uint32_t a = 0xffffffffu;
-            if (c < G::kTail) {
+            if (c < G::kTail - 1) {
                 const int dx = (c < side) ? R : -R + (c - side);
                 const int dy = (c < side) ? -R + c : R;
                 const int pp = (dx + R) & 3, m = (dx + R) >> 2;
@@ -227,6 +232,21 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 }
             }
             tacc[t] = a;
+        }
+        {   // leftover: byte phase 3, word R/2 - 1, window rows 2R .. 2R+15
+            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + G::kOffPh + 2 * G::kPhStride + (2 * R) * win) +
+                                 (R / 2 - 1);
+            const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+            uint32_t part = 0;
+#pragma unroll
+            for (int o = tid; o < 64; o += G::kThreads) {
+                const int v = o >> 2, k = o & 3;
+                const uint4 cv = cq4[v];
+                const uint32_t cw = k == 0 ? cv.x : k == 1 ? cv.y : k == 2 ? cv.z : cv.w;
+                part = sad4(rw[v * (win / 4) + k], cw, part);
+            }
+            const uint32_t wsum = __reduce_add_sync(0xffffffffu, part);
+            if (lane == 0 && warp * 32 < 64) atomicAdd(&lsum, wsum);
         }
 
         // ---- validity (restricted vectors) only matters near the frame border ----------
@@ -262,7 +282,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
 #pragma unroll
             for (int t = 0; t < kTailPer; ++t) {
                 const int c = tid + t * G::kThreads;
-                if (c < G::kTail) {
+                if (c < G::kTail - 1) {
                     const int dx = (c < side) ? R : -R + (c - side);
                     const int dy = (c < side) ? -R + c : R;
                     sf[(dy + R) * side + (dx + R)] = tacc[t];
@@ -284,6 +304,9 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         uint32_t M = red32[0];
 #pragma unroll
         for (int w = 1; w < nwarps; ++w) M = min(M, red32[w]);
+        const bool lvalid = (x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf);  // dx = R-1 >= 0, dy = R >= 0
+        const uint32_t lsad = lsum;
+        if (lvalid) M = min(M, lsad);
         uint64_t key = ~0ull;
         if (m == M) {  // rare: only threads holding a minimal candidate
 #pragma unroll
@@ -297,12 +320,18 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
 #pragma unroll
             for (int t = 0; t < kTailPer; ++t) {
                 const int c = tid + t * G::kThreads;
-                if (c < G::kTail && tacc[t] == M) {
+                if (c < G::kTail - 1 && tacc[t] == M) {
                     const uint64_t k = make_key(M, (c < side) ? R : -R + (c - side), (c < side) ? -R + c : R, R);
                     key = k < key ? k : key;
                 }
             }
         }
+        if (tid == 0 && lvalid && lsad == M) {
+            const uint64_t k = make_key(M, R - 1, R, R);
+            key = k < key ? k : key;
+        }
+        if (tid == 0 && A.surface)
+            A.surface[mb_index * side * side + (size_t)(2 * R) * side + (2 * R - 1)] = lvalid ? lsad : 0xffffffffu;
         key = warp_min_key(key);
         if (lane == 0) red64[warp] = key;
         __syncthreads();  // also: every thread is done with raw[s], cur[s] and the phases

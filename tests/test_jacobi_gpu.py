@@ -141,3 +141,27 @@ def test_host_api_end_to_end():
     a = sp_inputs.jacobi_input(100003, seed=9)
     got = sp.jacobi1d(a, 40, 16).numpy()
     _check(got, oracle.jacobi1d(a, 40))
+
+
+def test_dist_path_single_rank_nccl():
+    """The NCCL layer of the multi-GPU path (dlopen, unique id, communicator, distributed pass
+    loop) on the one GPU this box has: a single rank owning the whole domain."""
+    n, steps, tt = 20011, 70, 16
+    H = sp.halo_of(tt)
+    a = sp_inputs.jacobi_input(n, seed=21)
+    comm = sp.Comm(sp.get_unique_id(), 1, 0, torch.cuda.current_device())
+    try:
+        buf = torch.zeros(n + 2 * H, dtype=torch.float32, device="cuda")
+        buf[H:H + n] = torch.from_numpy(a).cuda()
+        work = torch.zeros_like(buf)
+        comm.jacobi1d_timetiled_dist(buf, work, n, 0, n, steps, tt)
+        torch.cuda.synchronize()
+        _check(buf[H:H + n].cpu().numpy(), oracle.jacobi1d(a, steps))
+        # all-gather of one rank is a copy
+        src = torch.arange(100, dtype=torch.int32, device="cuda")
+        dst = torch.zeros_like(src)
+        comm.allgather(src, dst)
+        torch.cuda.synchronize()
+        assert torch.equal(src, dst)
+    finally:
+        comm.destroy()
