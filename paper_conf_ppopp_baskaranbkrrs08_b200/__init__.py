@@ -39,7 +39,7 @@ __all__ = [
 ]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_HERE, "libsp.so")
+LIB_PATH = os.environ.get("SP_LIB") or os.path.join(_HERE, "libsp.so")
 
 PER_ARRAY = 0
 COMPONENTS = 1

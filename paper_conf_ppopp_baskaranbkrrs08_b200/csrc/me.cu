@@ -85,9 +85,9 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     constexpr int win = G::kWin;
     extern __shared__ __align__(128) uint8_t smem_raw[];
     __shared__ __align__(8) uint64_t full[2];
-    __shared__ uint32_t red32[32];
-    __shared__ unsigned int lsum;  // SAD of the leftover tail candidate (dx = R-1, dy = R)
-    __shared__ uint64_t red64[32];
+    __shared__ uint32_t red32[32];       // per-warp minimal SAD of the current MB
+    __shared__ unsigned int lsum[2];     // per-stage SAD of the leftover tail candidate (dx = R-1, dy = R)
+    __shared__ uint64_t red64[2][32];    // per-stage per-warp best key (published at the next MB)
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
 
@@ -116,8 +116,23 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         mbar_init(&full[0], 1);
         mbar_init(&full[1], 1);
         fence_mbar_init();
+        lsum[0] = lsum[1] = 0u;
     }
     __syncthreads();
+    // Publish macroblock mbp's argmin from the per-warp keys of stage sp (the last warp does
+    // it right after the next macroblock's barrier, when every warp has written its key).
+    auto finalize = [&](int64_t mbp, int sp) {
+        uint64_t b = red64[sp][0];
+#pragma unroll
+        for (int w = 1; w < nwarps; ++w) b = red64[sp][w] < b ? red64[sp][w] : b;
+        lsum[sp] = 0u;
+        const int pr = (int)(mbp / per_pair);
+        const int64_t rm = mbp - (int64_t)pr * per_pair;
+        const size_t idx = ((size_t)pr * A.mb_rows + (size_t)(rm / mbx)) * mbx + (size_t)(rm % mbx);
+        A.mv[2 * idx] = (int16_t)((int)(b & 127) - R);
+        A.mv[2 * idx + 1] = (int16_t)((int)((b >> 7) & 127) - R);
+        A.sad[idx] = (uint32_t)(b >> 21);
+    };
     if (tid == 0) {
         if (blockIdx.x < total) issue(blockIdx.x, 0);
         if (blockIdx.x + Gs < total) issue(blockIdx.x + Gs, 1);
@@ -154,8 +169,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 }
             }
         }
-        if (tid == 0) lsum = 0u;
-        __syncthreads();  // phase copies complete
+        __syncthreads();  // phase copies complete; every warp has finished the previous MB
+        if (tid == nwarps * 32 - 32 && it > 0) finalize(mb - Gs, s ^ 1);
 
         // ---- main 2R x 2R candidates: 4 dx (one byte phase) x 8 dy per thread ----------
         uint32_t acc[kTx][kTy];
@@ -220,16 +235,30 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 const int pp = (dx + R) & 3, m = (dx + R) >> 2;
                 const uint8_t* cb = (pp == 0) ? raw : smem + G::kOffPh + (pp - 1) * G::kPhStride;
                 const uint32_t* rw = reinterpret_cast<const uint32_t*>(cb + (dy + R) * win) + m;
-                a = 0;
+                uint32_t a0 = 0, a1 = 0, a2 = 0, a3 = 0;  // four independent chains (latency)
+                const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+                if (c < side) {  // column dx = +R: phase 0, word R/2 (16-byte aligned): LDS.128
 #pragma unroll
-                for (int v = 0; v < kMB; ++v) {
-                    const uint32_t* q = rw + v * (win / 4);
-                    const uint4 cv = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256)[v];
-                    a = sad4(q[0], cv.x, a);
-                    a = sad4(q[1], cv.y, a);
-                    a = sad4(q[2], cv.z, a);
-                    a = sad4(q[3], cv.w, a);
+                    for (int v = 0; v < kMB; ++v) {
+                        const uint4 q = *reinterpret_cast<const uint4*>(rw + v * (win / 4));
+                        const uint4 cv = cq[v];
+                        a0 = sad4(q.x, cv.x, a0);
+                        a1 = sad4(q.y, cv.y, a1);
+                        a2 = sad4(q.z, cv.z, a2);
+                        a3 = sad4(q.w, cv.w, a3);
+                    }
+                } else {
+#pragma unroll
+                    for (int v = 0; v < kMB; ++v) {
+                        const uint32_t* q = rw + v * (win / 4);
+                        const uint4 cv = cq[v];
+                        a0 = sad4(q[0], cv.x, a0);
+                        a1 = sad4(q[1], cv.y, a1);
+                        a2 = sad4(q[2], cv.z, a2);
+                        a3 = sad4(q[3], cv.w, a3);
+                    }
                 }
+                a = (a0 + a1) + (a2 + a3);
             }
             tacc[t] = a;
         }
@@ -246,7 +275,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 part = sad4(rw[v * (win / 4) + k], cw, part);
             }
             const uint32_t wsum = __reduce_add_sync(0xffffffffu, part);
-            if (lane == 0 && warp * 32 < 64) atomicAdd(&lsum, wsum);
+            if (lane == 0 && warp * 32 < 64) atomicAdd(&lsum[s], wsum);
         }
 
         // ---- validity (restricted vectors) only matters near the frame border ----------
@@ -300,12 +329,16 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         for (int t = 0; t < kTailPer; ++t) m = min(m, tacc[t]);
         const uint32_t wm = __reduce_min_sync(0xffffffffu, m);
         if (lane == 0) red32[warp] = wm;
-        __syncthreads();
+        __syncthreads();  // every warp is done with raw[s], cur[s] and the phase copies
+        if (tid == 0 && mb + 2 * Gs < total) {
+            fence_proxy_async_smem();
+            issue(mb + 2 * Gs, s);
+        }
         uint32_t M = red32[0];
 #pragma unroll
         for (int w = 1; w < nwarps; ++w) M = min(M, red32[w]);
         const bool lvalid = (x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf);  // dx = R-1 >= 0, dy = R >= 0
-        const uint32_t lsad = lsum;
+        const uint32_t lsad = lsum[s];
         if (lvalid) M = min(M, lsad);
         uint64_t key = ~0ull;
         if (m == M) {  // rare: only threads holding a minimal candidate
@@ -333,19 +366,10 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         if (tid == 0 && A.surface)
             A.surface[mb_index * side * side + (size_t)(2 * R) * side + (2 * R - 1)] = lvalid ? lsad : 0xffffffffu;
         key = warp_min_key(key);
-        if (lane == 0) red64[warp] = key;
-        __syncthreads();  // also: every thread is done with raw[s], cur[s] and the phases
-        if (tid == 0) {
-            uint64_t b = red64[0];
-#pragma unroll
-            for (int w = 1; w < nwarps; ++w) b = red64[w] < b ? red64[w] : b;
-            A.mv[2 * mb_index] = (int16_t)((int)(b & 127) - R);
-            A.mv[2 * mb_index + 1] = (int16_t)((int)((b >> 7) & 127) - R);
-            A.sad[mb_index] = (uint32_t)(b >> 21);
-            fence_proxy_async_smem();
-            if (mb + 2 * Gs < total) issue(mb + 2 * Gs, s);
-        }
+        if (lane == 0) red64[s][warp] = key;
     }
+    __syncthreads();
+    if (tid == 0 && it > 0) finalize(blockIdx.x + (int64_t)(it - 1) * Gs, (it - 1) & 1);
 }
 
 // Generic path (any 0 <= R <= 63): window staged byte-wise with zero fill, one thread per
