@@ -37,7 +37,10 @@ namespace {
 using namespace sp::ptx;
 
 constexpr int kMB = 16;      // macroblock edge (WS = 16)
-constexpr int kTy = 8;       // dy candidates per thread
+#ifndef SP_ME_TY
+#define SP_ME_TY 8
+#endif
+constexpr int kTy = SP_ME_TY;  // dy candidates per thread (8, or 4 for twice the threads)
 constexpr int kTx = 4;       // dx candidates per thread (same byte phase, stride 4)
 
 struct MeArgs {
@@ -69,7 +72,8 @@ template <int R>
 struct MeGeom {
     static constexpr int kWin = 2 * R + 16;              // window edge (bytes per row, rows)
     static constexpr int kCopy = kWin * kWin;            // bytes per staged copy (multiple of 128)
-    static constexpr int kThreads = R * R / 8;           // one 4x8 candidate tile per thread
+    static constexpr int kThreads = R * R / kTy;         // one 4 x kTy candidate tile per thread
+    static constexpr int kSplit = kThreads / (4 * R) > 1 ? kThreads / (4 * R) : 1;  // threads per tail candidate
     static constexpr int kGx = R / 8;                    // dx groups per byte phase
     static constexpr int kPhStride = kCopy + 32;         // phase copies at 32-byte bank offsets
     static constexpr int kOffCur = 2 * kCopy;            // cur[2] after raw[2]
@@ -79,7 +83,7 @@ struct MeGeom {
 };
 
 template <int R>
-__global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
+__global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? (kTy == 8 ? 4 : 3) : (kTy == 8 ? 16 : 8)))
 me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
     using G = MeGeom<R>;
     constexpr int win = G::kWin;
@@ -187,23 +191,23 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             const uint8_t* base = (p == 0) ? raw : smem + G::kOffPh + (p - 1) * G::kPhStride;
             const uint8_t* rowp = base + (kTy * d) * win + 16 * g;
             const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
-            uint32_t Rw[8][7];  // words 4g..4g+6 (j + k <= 6)
+            uint32_t Rw[kTy][7];  // words 4g..4g+6 (j + k <= 6)
 #pragma unroll
-            for (int rr = 0; rr < 7; ++rr) {
+            for (int rr = 0; rr < kTy - 1; ++rr) {
                 const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + rr * win);
                 const uint4 w1 = *reinterpret_cast<const uint4*>(rowp + rr * win + 16);
                 Rw[rr][0] = w0.x; Rw[rr][1] = w0.y; Rw[rr][2] = w0.z; Rw[rr][3] = w0.w;
                 Rw[rr][4] = w1.x; Rw[rr][5] = w1.y; Rw[rr][6] = w1.z;
             }
 #pragma unroll 1
-            for (int vb = 0; vb < kMB; vb += 8) {
+            for (int vb = 0; vb < kMB; vb += kTy) {
 #pragma unroll
-                for (int vv = 0; vv < 8; ++vv) {
+                for (int vv = 0; vv < kTy; ++vv) {
                     const int v = vb + vv;
                     {
-                        const int slot = (vv + 7) & 7;
-                        const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + (v + 7) * win);
-                        const uint4 w1 = *reinterpret_cast<const uint4*>(rowp + (v + 7) * win + 16);
+                        const int slot = (vv + kTy - 1) % kTy;
+                        const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + (v + kTy - 1) * win);
+                        const uint4 w1 = *reinterpret_cast<const uint4*>(rowp + (v + kTy - 1) * win + 16);
                         Rw[slot][0] = w0.x; Rw[slot][1] = w0.y; Rw[slot][2] = w0.z; Rw[slot][3] = w0.w;
                         Rw[slot][4] = w1.x; Rw[slot][5] = w1.y; Rw[slot][6] = w1.z;
                     }
@@ -215,7 +219,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                         for (int i = 0; i < kTy; ++i)
 #pragma unroll
                             for (int j = 0; j < kTx; ++j)
-                                acc[j][i] = sad4(Rw[(vv + i) & 7][j + k], Cv[k], acc[j][i]);
+                                acc[j][i] = sad4(Rw[(vv + i) % kTy][j + k], Cv[k], acc[j][i]);
                 }
             }
         }
@@ -223,23 +227,28 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // 4R of the 4R+1 tail candidates spread evenly over the threads; the last one
         // (dx = R-1, dy = R) is split one 4-pixel word per lane across the warps so that
         // no warp carries extra work into the reduction barrier
-        constexpr int kTailPer = (G::kTail - 1 + G::kThreads - 1) / G::kThreads;
+        // (with kSplit > 1 threads per candidate, each sums kMB/kSplit rows, combined by shuffle)
+        constexpr int KS = G::kSplit;
+        constexpr int kTRows = kMB / KS;
+        constexpr int kTailThreads = G::kThreads / KS;
+        constexpr int kTailPer = (G::kTail - 1 + kTailThreads - 1) / kTailThreads;
+        const int tc = tid / KS, th = tid % KS;
         uint32_t tacc[kTailPer];
 #pragma unroll
         for (int t = 0; t < kTailPer; ++t) {
-            const int c = tid + t * G::kThreads;
-            uint32_t a = 0xffffffffu;
+            const int c = tc + t * kTailThreads;
+            uint32_t a = 0;
             if (c < G::kTail - 1) {
                 const int dx = (c < side) ? R : -R + (c - side);
                 const int dy = (c < side) ? -R + c : R;
                 const int pp = (dx + R) & 3, m = (dx + R) >> 2;
                 const uint8_t* cb = (pp == 0) ? raw : smem + G::kOffPh + (pp - 1) * G::kPhStride;
-                const uint32_t* rw = reinterpret_cast<const uint32_t*>(cb + (dy + R) * win) + m;
+                const uint32_t* rw = reinterpret_cast<const uint32_t*>(cb + (dy + R + th * kTRows) * win) + m;
                 uint32_t a0 = 0, a1 = 0, a2 = 0, a3 = 0;  // four independent chains (latency)
-                const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+                const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256) + th * kTRows;
                 if (c < side) {  // column dx = +R: phase 0, word R/2 (16-byte aligned): LDS.128
 #pragma unroll
-                    for (int v = 0; v < kMB; ++v) {
+                    for (int v = 0; v < kTRows; ++v) {
                         const uint4 q = *reinterpret_cast<const uint4*>(rw + v * (win / 4));
                         const uint4 cv = cq[v];
                         a0 = sad4(q.x, cv.x, a0);
@@ -249,7 +258,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     }
                 } else {
 #pragma unroll
-                    for (int v = 0; v < kMB; ++v) {
+                    for (int v = 0; v < kTRows; ++v) {
                         const uint32_t* q = rw + v * (win / 4);
                         const uint4 cv = cq[v];
                         a0 = sad4(q[0], cv.x, a0);
@@ -260,7 +269,9 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 }
                 a = (a0 + a1) + (a2 + a3);
             }
-            tacc[t] = a;
+#pragma unroll
+            for (int o = 1; o < KS; o <<= 1) a += __shfl_xor_sync(0xffffffffu, a, o);
+            tacc[t] = (c < G::kTail - 1 && th == 0) ? a : 0xffffffffu;
         }
         {   // leftover: byte phase 3, word R/2 - 1, window rows 2R .. 2R+15
             const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + G::kOffPh + 2 * G::kPhStride + (2 * R) * win) +
@@ -294,7 +305,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
 #pragma unroll
             for (int t = 0; t < kTailPer; ++t) {
-                const int c = tid + t * G::kThreads;
+                const int c = tc + t * kTailThreads;
                 const int dx = (c < side) ? R : -R + (c - side);
                 const int dy = (c < side) ? -R + c : R;
                 if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) tacc[t] = 0xffffffffu;
@@ -310,8 +321,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     sf[(kTy * d + i) * side + (p + 4 * (4 * g + j))] = acc[j][i];
 #pragma unroll
             for (int t = 0; t < kTailPer; ++t) {
-                const int c = tid + t * G::kThreads;
-                if (c < G::kTail - 1) {
+                const int c = tc + t * kTailThreads;
+                if (c < G::kTail - 1 && th == 0) {
                     const int dx = (c < side) ? R : -R + (c - side);
                     const int dy = (c < side) ? -R + c : R;
                     sf[(dy + R) * side + (dx + R)] = tacc[t];
@@ -352,7 +363,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     }
 #pragma unroll
             for (int t = 0; t < kTailPer; ++t) {
-                const int c = tid + t * G::kThreads;
+                const int c = tc + t * kTailThreads;
                 if (c < G::kTail - 1 && tacc[t] == M) {
                     const uint64_t k = make_key(M, (c < side) ? R : -R + (c - side), (c < side) ? -R + c : R, R);
                     key = k < key ? k : key;
