@@ -6,8 +6,8 @@ One step = one pass of the whole hot path over one ba
   * ME (BASELINE config 4): full-search SAD motion estimation of a 64-pair batch of
     1920x1080 uint8 frames, +-32, 16x16 macroblocks, per GPU.
 Multi-GPU (torchrun, one process per GPU): weak scaling.  Jacobi's global domain is the
-concatenation of the ranks' slabs with a halo exchange (NCCL send/recv inside libsp) once
-per time tile; ME ranks search their own 64-pair shard of a 64*N-pair batch (no data-path
+concatenation of the ranks' slabs with a halo exchange once per time tile, fused into the
+pass kernel as peer-memory stores (default) or as NCCL send/recv (--halo nccl); ME ranks search their own 64-pair shard of a 64*N-pair batch (no data-path
 collective).  `value` = Jacobi point-updates of all ranks / max-over-ranks device time;
 ME's throughput is reported in the `me` object with its own roofline.
 
@@ -53,7 +53,8 @@ def bench_config(world, tt):
                         f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs/GPU",
             "jacobi_global_n": JAC_N_LOCAL * world, "time_tile": tt, "me_pairs_global": ME_PAIRS * world,
             "l2": "inputs larger than L2 (256 MiB Jacobi state per GPU, 135 MB frame batch); no flush",
-            "parallelism": f"weak scaling over {world} GPU(s); Jacobi halo exchange per time tile"}
+            "parallelism": f"weak scaling over {world} GPU(s); Jacobi halo exchange per time tile "
+                           "(fused peer-memory stores inside the pass kernel)"}
 
 
 def peaks():
@@ -228,10 +229,17 @@ def run_ours(args, rank, world, local_rank):
     n_global = n_local * world
     x_begin = rank * n_local
     comm = None
+    slab = None
     if world == 1:
         a_host = sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED)
         a = torch.from_numpy(a_host).to(dev)
         work = torch.empty_like(a)
+    elif args.halo == "peer":
+        # fused halo exchange: the pass kernels store halos into the neighbours' buffers
+        slab = sp.PeerSlab(n_global, x_begin, n_local, tt)
+        slab.a[H:H + n_local] = torch.from_numpy(
+            sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED, begin=x_begin)).to(dev)
+        a, work = slab.a, slab.work
     else:
         lo, hi = max(0, x_begin - H), min(n_global, x_begin + n_local + H)
         a = torch.zeros(n_local + 2 * H, dtype=torch.float32, device=dev)
@@ -244,15 +252,20 @@ def run_ours(args, rank, world, local_rank):
         dist.broadcast(uid, 0)
         comm = sp.Comm(bytes(uid.cpu().numpy().tobytes()), world, rank, local_rank)
 
-    def jacobi_step():
-        if comm is None:
-            sp.jacobi1d_timetiled(a, JAC_T, tt, 0, work=work)
+    def jacobi_run(steps):
+        if slab is not None:
+            slab.run(steps)
+        elif comm is not None:
+            comm.jacobi1d_timetiled_dist(a, work, n_global, x_begin, n_local, steps, tt, 0)
         else:
-            comm.jacobi1d_timetiled_dist(a, work, n_global, x_begin, n_local, JAC_T, tt, 0)
+            sp.jacobi1d_timetiled(a, steps, tt, 0, work=work)
+
+    def jacobi_step():
+        jacobi_run(JAC_T)
 
     # ---- ME batch: this rank's 64 pairs = frames [64 r, 64 r + 65) of the sequence
     f0 = ME_PAIRS * rank
-    frames_host = np.stack([sp_inputs.me_frame(f0 + f, ME_W, ME_H, ME_R) for f in range(ME_PAIRS + 1)])
+    frames_host = np.ascontiguousarray(np.stack([sp_inputs.me_frame(f0 + f, ME_W, ME_H, ME_R) for f in range(ME_PAIRS + 1)]))
     frames = torch.from_numpy(frames_host).to(dev)
     mbx, mby = ME_W // 16, ME_H // 16
     me_out = (torch.empty((ME_PAIRS, mby, mbx, 2), dtype=torch.int16, device=dev),
@@ -298,7 +311,7 @@ def run_ours(args, rank, world, local_rank):
     def max_over_ranks(x):
         if world == 1:
             return x
-        t = torch.tensor([x], dtype=torch.float64, device=dev)
+        t = torch.tensor([x], dtype=torch.float64, device="cpu" if dist.get_backend() == "gloo" else dev)
         dist.all_reduce(t, op=dist.ReduceOp.MAX)
         return float(t.item())
 
@@ -315,10 +328,7 @@ def run_ours(args, rank, world, local_rank):
     torch.cuda.synchronize()
     e0.record(stream)
     for _ in range(reps):
-        if comm is None:
-            sp.jacobi1d_timetiled(a, 2 * tt, tt, 0, work=work)  # 2 full-height launches
-        else:
-            comm.jacobi1d_timetiled_dist(a, work, n_global, x_begin, n_local, 2 * tt, tt, 0)
+        jacobi_run(2 * tt)  # 2 full-height launches
     e1.record(stream)
     torch.cuda.synchronize()
     jac_launch_ms = e0.elapsed_time(e1) / (2 * reps)
@@ -388,7 +398,7 @@ def run_ours(args, rank, world, local_rank):
         cpu = {"value": s["jacobi_ups"] / 1e9, "unit": "GPoint-updates/s", "cores": s["cores"], "kind": "oracle",
                "sample": s["sample"], "me_value": s["me_sads"] / 1e9, "me_unit": "GSAD/s"}
 
-    launches_per_step = plan["passes"] + 1  # Jacobi passes + one ME launch
+    launches_per_step = plan["passes"] + 1 + (1 if slab is not None else 0)  # passes + ME (+ peer done signal)
     line = {
         "metric": METRIC, "value": round(jac_val, 2), "unit": "GPoint-updates/s", "n_gpus": world, "steps": K,
         "warmup": args.warmup, "ms_per_step": round(total_ms / K, 4), "higher_is_better": True, "scaling": "weak",
@@ -405,6 +415,8 @@ def run_ours(args, rank, world, local_rank):
         print(json.dumps(line), flush=True)
     if comm is not None:
         comm.destroy()
+    if slab is not None:
+        slab.close()
     return 0
 
 
@@ -416,17 +428,27 @@ def main():
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
     ap.add_argument("--time-tile", type=int, default=32)
     ap.add_argument("--no-cpu-baseline", action="store_true")
+    ap.add_argument("--halo", choices=["peer", "nccl"], default="peer",
+                    help="multi-GPU Jacobi halo exchange: fused peer stores in the pass kernel, or NCCL send/recv")
     args = ap.parse_args()
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local_rank = int(os.environ.get("LOCAL_RANK", "0"))
+    # test hook: SP_BENCH_SHARE_GPU=1 runs every rank on cuda:0 with a gloo process group, to
+    # exercise the multi-rank path on a one-GPU box (timings are then meaningless)
+    share = os.environ.get("SP_BENCH_SHARE_GPU") == "1"
+    if share:
+        local_rank = 0
     if args.impl == "reference":
         return run_reference(args, rank, world)
     if world > 1:
         import torch
         import torch.distributed as dist
         torch.cuda.set_device(local_rank)
-        dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
+        if share:
+            dist.init_process_group("gloo")
+        else:
+            dist.init_process_group("nccl", device_id=torch.device("cuda", local_rank))
     try:
         return run_ours(args, rank, world, local_rank)
     finally:

@@ -257,6 +257,39 @@ int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_locals, int32_
                                    const int64_t* x_begins, const int64_t* n_locals, int32_t steps,
                                    int32_t time_tile, int32_t space_tile, void* stream);
 
+/* Fused variant: the halo exchange runs inside the pass kernel over peer memory (NVLink P2P
+ * or CUDA-IPC mapped pointers) instead of a separate NCCL step.  At the start of pass p the
+ * kernel stores this rank's first / last H owned cells straight into the neighbours'
+ * current buffers and raises their epoch flags (release, system scope); only the tiles whose
+ * footprint reaches into a halo wait (acquire) for this rank's own flags; interior tiles
+ * never wait, so the exchange overlaps the interior work tile by tile.  Every rank uses
+ * a_local in even and work_local in odd passes (layout as in sp_jacobi1d_timetiled_dist).
+ * Flags are monotone epochs: this call uses epoch0+1 .. epoch0+passes; callers advance
+ * epoch0 by the pass count between calls (flags start at 0).  flags[2] / flags[3] receive the
+ * left / right neighbour's "done with the call" epoch; the first push of a call waits for
+ * them (the push targets a buffer the neighbour may still read in its previous call). */
+typedef struct {
+    float* left_bufs[2];       /* left neighbour's a_local / work_local (mapped), NULL if none */
+    float* right_bufs[2];      /* right neighbour's a_local / work_local (mapped) */
+    int64_t left_n_local;      /* left neighbour's owned cell count */
+    int64_t right_n_local;
+    unsigned long long* left_flags;   /* left neighbour's flags[4] (mapped) */
+    unsigned long long* right_flags;  /* right neighbour's flags[4] (mapped) */
+    unsigned long long* my_flags;     /* own flags[4]: [0] left-halo epoch, [1] right-halo epoch,
+                                         [2] left neighbour done, [3] right neighbour done */
+    uint64_t epoch0;
+} sp_peer_links;
+int sp_jacobi1d_timetiled_peer(const sp_peer_links* links, float* a_local, float* work_local, int64_t n_global,
+                               int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
+                               int32_t space_tile, void* stream);
+
+/* Exportable device allocations and CUDA-IPC handles (64 bytes) for the peer path. */
+int sp_device_alloc(void** ptr, int64_t bytes); /* cudaMalloc + zero fill */
+int sp_device_free(void* ptr);
+int sp_ipc_get_handle(const void* ptr, uint8_t out_handle[64]);
+int sp_ipc_open_handle(const uint8_t handle[64], void** ptr);
+int sp_ipc_close_handle(void* ptr);
+
 /* ncclAllGather of `bytes` per rank (device buffers) — used for the ME results. */
 int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream);
 

@@ -79,6 +79,11 @@ class sp_jacobi_plan(ctypes.Structure):
                 ("tiles", i64), ("grid", i32), ("threads", i32), ("smem_bytes", i32), ("cells_per_thread", i32)]
 
 
+class sp_peer_links(ctypes.Structure):
+    _fields_ = [("left_bufs", vp * 2), ("right_bufs", vp * 2), ("left_n_local", i64), ("right_n_local", i64),
+                ("left_flags", vp), ("right_flags", vp), ("my_flags", vp), ("epoch0", ctypes.c_uint64)]
+
+
 class sp_tile_problem(ctypes.Structure):
     _fields_ = [("depth", i32), ("n_refs", i32), ("extent", ctypes.POINTER(i64)), ("refs", ctypes.POINTER(sp_ref)),
                 ("n_cand", ctypes.POINTER(i32)), ("cand", ctypes.POINTER(i64)), ("mup_elems", i64), ("procs", i32),
@@ -112,6 +117,13 @@ SYMBOLS = {
     "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
     "sp_jacobi1d_untiled": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_tile_search": (ctypes.c_int, [ctypes.POINTER(sp_tile_problem), ctypes.POINTER(sp_tile_result)]),
+    "sp_jacobi1d_timetiled_peer": (ctypes.c_int, [ctypes.POINTER(sp_peer_links), vp, vp, i64, i64, i64, i32, i32, i32,
+                                                  vp]),
+    "sp_device_alloc": (ctypes.c_int, [ctypes.POINTER(vp), i64]),
+    "sp_device_free": (ctypes.c_int, [vp]),
+    "sp_ipc_get_handle": (ctypes.c_int, [vp, ctypes.POINTER(ctypes.c_uint8)]),
+    "sp_ipc_open_handle": (ctypes.c_int, [ctypes.POINTER(ctypes.c_uint8), ctypes.POINTER(vp)]),
+    "sp_ipc_close_handle": (ctypes.c_int, [vp]),
     "sp_me_sad_search_direct": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp,
                                                vp, vp]),
 }
@@ -445,3 +457,92 @@ class Comm:
     def allgather(self, send, recv, stream=None):
         nbytes = send.numel() * send.element_size()
         _check(lib.sp_allgather(self.handle, _ptr(send), _ptr(recv), nbytes, _stream(stream)), "sp_allgather")
+
+
+# ---------------------------------------------------------------------------------------
+# Fused peer-memory halo exchange (sp_jacobi1d_timetiled_peer)
+# ---------------------------------------------------------------------------------------
+class _DevView:
+    """__cuda_array_interface__ view of a libsp device allocation (for torch.as_tensor)."""
+
+    def __init__(self, ptr: int, n: int, typestr: str):
+        self.__cuda_array_interface__ = {"shape": (n,), "typestr": typestr, "data": (ptr, False), "version": 3}
+
+
+class PeerSlab:
+    """One rank's slab of the distributed Jacobi domain for the fused peer-memory path.
+
+    a / work / flags are CUDA-IPC-exportable allocations owned by libsp; the handles are
+    exchanged with the neighbours through torch.distributed (any backend) and mapped, so the
+    pass kernel stores halos straight into the neighbours' buffers (NVLink peer writes between
+    GPUs; the same code runs between processes sharing one GPU).  `a` is a torch view of the
+    rank's [x_begin - H, x_end + H) buffer."""
+
+    def __init__(self, n_global: int, x_begin: int, n_local: int, time_tile: int, space_tile: int = 0):
+        import torch
+        import torch.distributed as dist
+        self.n_global, self.x_begin, self.n_local = int(n_global), int(x_begin), int(n_local)
+        self.time_tile, self.space_tile = int(time_tile), int(space_tile)
+        self.H = halo_of(time_tile)
+        cells = self.n_local + 2 * self.H
+        self._own = []
+        ptrs = []
+        for nbytes in (4 * cells, 4 * cells, 64):
+            p = vp()
+            _check(lib.sp_device_alloc(ctypes.byref(p), nbytes), "sp_device_alloc")
+            self._own.append(p.value)
+            ptrs.append(p.value)
+        self.a_ptr, self.w_ptr, self.f_ptr = ptrs
+        handles = []
+        for p in ptrs:
+            h = (ctypes.c_uint8 * 64)()
+            _check(lib.sp_ipc_get_handle(vp(p), h), "sp_ipc_get_handle")
+            handles.append(bytes(h))
+        rank, world = dist.get_rank(), dist.get_world_size()
+        info = [None] * world
+        dist.all_gather_object(info, {"handles": handles, "n_local": self.n_local, "x_begin": self.x_begin})
+        self._mapped = []
+
+        def open_all(r):
+            out = []
+            for hb in info[r]["handles"]:
+                q = vp()
+                _check(lib.sp_ipc_open_handle((ctypes.c_uint8 * 64)(*hb), ctypes.byref(q)), "sp_ipc_open_handle")
+                self._mapped.append(q.value)
+                out.append(q.value)
+            return out
+        L = sp_peer_links()
+        if self.x_begin > 0:
+            la, lw, lf = open_all(rank - 1)
+            L.left_bufs[0], L.left_bufs[1], L.left_flags = la, lw, lf
+            L.left_n_local = info[rank - 1]["n_local"]
+        if self.x_begin + self.n_local < self.n_global:
+            ra, rw, rf = open_all(rank + 1)
+            L.right_bufs[0], L.right_bufs[1], L.right_flags = ra, rw, rf
+            L.right_n_local = info[rank + 1]["n_local"]
+        L.my_flags = self.f_ptr
+        L.epoch0 = 0
+        self.links = L
+        self.a = torch.as_tensor(_DevView(self.a_ptr, cells, "<f4"), device="cuda")
+        self.work = torch.as_tensor(_DevView(self.w_ptr, cells, "<f4"), device="cuda")
+        dist.barrier()
+
+    def run(self, steps: int, stream=None):
+        """sp_jacobi1d_timetiled_peer over this slab; advances the epoch base."""
+        _check(lib.sp_jacobi1d_timetiled_peer(ctypes.byref(self.links), vp(self.a_ptr), vp(self.w_ptr),
+                                              self.n_global, self.x_begin, self.n_local, int(steps), self.time_tile,
+                                              self.space_tile, _stream(stream)), "sp_jacobi1d_timetiled_peer")
+        self.links.epoch0 += (int(steps) + self.time_tile - 1) // self.time_tile
+
+    def close(self):
+        import torch
+        import torch.distributed as dist
+        torch.cuda.synchronize()
+        dist.barrier()
+        for p in self._mapped:
+            lib.sp_ipc_close_handle(vp(p))
+        self._mapped = []
+        dist.barrier()
+        for p in self._own:
+            lib.sp_device_free(vp(p))
+        self._own = []

@@ -23,6 +23,7 @@
 #include <algorithm>
 #include <cstdint>
 #include <cstdlib>
+#include <cstring>
 #include <mutex>
 
 #include "../../include/sp.h"
@@ -64,7 +65,34 @@ struct PassArgs {
     int32_t wo;        // owned cells per warp (multiple of 4)
     int64_t* flog;     // nullable: [tiles][2] footprint of this pass
     uint64_t mz;       // (-0.0f, -0.0f), opaque to ptxas (see f2_mul_nofuse)
+    // Fused peer-memory halo exchange (sp_jacobi1d_timetiled_peer); all null otherwise.
+    // At kernel start block 0 / warp 0 stores this rank's first / last H owned cells straight
+    // into the neighbours' current buffers (NVLink peer or IPC-mapped pointers) and raises
+    // their epoch flags (release, system scope); a tile whose footprint reaches into a halo
+    // waits for this rank's own flag (acquire) before its TMA move-in.  Interior tiles never wait.
+    float* push_left;                     // left neighbour's right-halo cells
+    float* push_right;                    // right neighbour's left-halo cells
+    unsigned long long* signal_left;      // left neighbour's right-halo flag
+    unsigned long long* signal_right;     // right neighbour's left-halo flag
+    const unsigned long long* wait_left;  // own left-halo flag
+    const unsigned long long* wait_right; // own right-halo flag
+    unsigned long long epoch;
+    // first pass of a call only: before pushing, wait until the neighbours have finished the
+    // previous call (their "done" epochs >= epoch - 1), since the push targets a buffer they
+    // may still be reading in their last pass of that call
+    const unsigned long long* done_left;
+    const unsigned long long* done_right;
 };
+
+// Spin (acquire, system scope) until *flag >= e.  A peer that never arrives (crashed rank,
+// mismatched calls) traps after ~20 s instead of hanging the device.
+__device__ __forceinline__ void wait_epoch(const unsigned long long* flag, unsigned long long e) {
+    const long long t0 = clock64();
+    while (ld_acquire_sys(flag) < e) {
+        __nanosleep(64);
+        if (clock64() - t0 > (40ll << 30)) __trap();
+    }
+}
 
 // Lane neighbours of a thread's 2K cells: four shuffles.  The v strip continues the u strip:
 // lane 0's v-left is lane 31's last u and lane 31's u-right is lane 0's first v.
@@ -175,11 +203,37 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     auto issue = [&](int64_t t, int s) {  // lane 0 only
         int64_t x0, st, lo, hi;
         tile_range(t, x0, st, lo, hi);
+        if (A.wait_left && lo < A.own_begin) {   // halo from the left neighbour (peer store)
+            wait_epoch(A.wait_left, A.epoch);
+            fence_proxy_async_global();
+        }
+        if (A.wait_right && hi > A.own_end) {
+            wait_epoch(A.wait_right, A.epoch);
+            fence_proxy_async_global();
+        }
         const uint32_t bytes = (uint32_t)(((hi - lo) & ~int64_t(3)) * 4);
         mbar_arrive_expect_tx(&bar[s], bytes);
         if (bytes) tma_load_1d(stage0 + s * kStrip + (lo - (x0 - A.H)), A.src + (lo - A.g0), bytes, &bar[s]);
     };
 
+    if (blockIdx.x == 0 && warp == 0 && (A.push_left || A.push_right)) {
+        // fused halo exchange: owned edge cells -> neighbours' halos, then their flags
+        if (lane == 0) {
+            if (A.done_left) wait_epoch(A.done_left, A.epoch - 1);
+            if (A.done_right) wait_epoch(A.done_right, A.epoch - 1);
+        }
+        __syncwarp();
+        for (int i = lane; i < A.H; i += 32) {
+            if (A.push_left) A.push_left[i] = A.src[A.own_begin + i - A.g0];
+            if (A.push_right) A.push_right[i] = A.src[A.own_end - A.H + i - A.g0];
+        }
+        __threadfence_system();
+        __syncwarp();
+        if (lane == 0) {
+            if (A.signal_left) st_release_sys(A.signal_left, A.epoch);
+            if (A.signal_right) st_release_sys(A.signal_right, A.epoch);
+        }
+    }
     if (lane == 0) {
         mbar_init(&bar[0], 1);
         mbar_init(&bar[1], 1);
@@ -426,7 +480,8 @@ extern "C" int sp_jacobi1d_pass_segment(const float* src, float* dst, int64_t n_
     }
     Variant di;
     if ((st = device_info(di))) return st;
-    PassArgs a{src, dst, n_global, g0, len, own_begin, own_end, S, (own_end - own_begin + S - 1) / S, h, H, wo, nullptr, kNegZero2};
+    PassArgs a{src, dst, n_global, g0, len, own_begin, own_end, S, (own_end - own_begin + S - 1) / S, h, H, wo, nullptr, kNegZero2,
+                nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, 0ull, nullptr, nullptr};
     return launch_pass(a, (cudaStream_t)stream, di);
 }
 
@@ -450,12 +505,109 @@ extern "C" int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t s
     for (int32_t done = 0; done < steps; done += time_tile, ++pass) {
         const int32_t h = steps - done < time_tile ? steps - done : time_tile;
         PassArgs p{cur, nxt, n, 0, n, 0, n, S, tiles, h, H, wo,
-                   footprint_log ? footprint_log + (int64_t)pass * tiles * 2 : nullptr, kNegZero2};
+                   footprint_log ? footprint_log + (int64_t)pass * tiles * 2 : nullptr, kNegZero2,
+                   nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, 0ull, nullptr, nullptr};
         if ((st = launch_pass(p, s, di))) return st;
         float* t = cur;
         cur = nxt;
         nxt = t;
     }
     if (cur != a) SP_CUDA_TRY(cudaMemcpyAsync(a, cur, (size_t)n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    return SP_OK;
+}
+
+__global__ void peer_done_kernel(unsigned long long* left_done, unsigned long long* right_done, unsigned long long e) {
+    __threadfence_system();
+    if (left_done) st_release_sys(left_done, e);
+    if (right_done) st_release_sys(right_done, e);
+}
+
+// Multi-GPU time-tiled Jacobi with the halo exchange fused into the pass kernel over peer
+// memory (see PassArgs).  Buffer parity is global: every rank uses a_local in even passes
+// and work_local in odd passes, so the neighbours' buffers are addressed by pass parity.
+extern "C" int sp_jacobi1d_timetiled_peer(const sp_peer_links* L, float* a_local, float* work_local, int64_t n_global,
+                                          int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
+                                          int32_t space_tile, void* stream) {
+    if (!L || !a_local || !work_local || a_local == work_local || n_global < 3 || x_begin < 0 || n_local < 1 ||
+        x_begin + n_local > n_global || steps < 0 || (x_begin & 3) || !L->my_flags)
+        return SP_ERR_INVALID_ARG;
+    if ((reinterpret_cast<uintptr_t>(a_local) & 15) || (reinterpret_cast<uintptr_t>(work_local) & 15))
+        return SP_ERR_INVALID_ARG;
+    const bool has_left = x_begin > 0, has_right = x_begin + n_local < n_global;
+    if ((has_left && (!L->left_bufs[0] || !L->left_bufs[1] || !L->left_flags)) ||
+        (has_right && (!L->right_bufs[0] || !L->right_bufs[1] || !L->right_flags)))
+        return SP_ERR_INVALID_ARG;
+    int64_t S;
+    int32_t wo;
+    int st = geometry(time_tile, space_tile, S, wo);
+    if (st) return st;
+    const int32_t H = halo_of(time_tile);
+    if ((has_left || has_right) && n_local < H) return SP_ERR_INVALID_ARG;
+    if (steps == 0) return SP_OK;
+    Variant di;
+    if ((st = device_info(di))) return st;
+    const cudaStream_t s = (cudaStream_t)stream;
+    const int64_t g0 = x_begin - H, len = n_local + 2 * H;
+    float* bufs[2] = {a_local, work_local};
+    int pass = 0;
+    for (int32_t done = 0; done < steps; done += time_tile, ++pass) {
+        const int32_t h = steps - done < time_tile ? steps - done : time_tile;
+        const int q = pass & 1;
+        PassArgs p{bufs[q], bufs[q ^ 1], n_global, g0, len, x_begin, x_begin + n_local, S,
+                   (n_local + S - 1) / S, h, H, wo, nullptr, kNegZero2,
+                   has_left ? L->left_bufs[q] + L->left_n_local + H : nullptr,
+                   has_right ? L->right_bufs[q] : nullptr,
+                   has_left ? L->left_flags + 1 : nullptr,
+                   has_right ? L->right_flags + 0 : nullptr,
+                   has_left ? L->my_flags + 0 : nullptr,
+                   has_right ? L->my_flags + 1 : nullptr,
+                   (unsigned long long)(L->epoch0 + (uint64_t)pass + 1),
+                   (pass == 0 && has_left) ? L->my_flags + 2 : nullptr,
+                   (pass == 0 && has_right) ? L->my_flags + 3 : nullptr};
+        if ((st = launch_pass(p, s, di))) return st;
+    }
+    if (pass & 1)
+        SP_CUDA_TRY(cudaMemcpyAsync(a_local + H, work_local + H, (size_t)n_local * sizeof(float),
+                                    cudaMemcpyDeviceToDevice, s));
+    // tell the neighbours this rank is done with every buffer of this call
+    peer_done_kernel<<<1, 1, 0, s>>>(has_left ? L->left_flags + 3 : nullptr, has_right ? L->right_flags + 2 : nullptr,
+                                     (unsigned long long)(L->epoch0 + (uint64_t)pass));
+    SP_CUDA_TRY(cudaGetLastError());
+    return SP_OK;
+}
+
+extern "C" int sp_device_alloc(void** ptr, int64_t bytes) {
+    if (!ptr || bytes < 1) return SP_ERR_INVALID_ARG;
+    SP_CUDA_TRY(cudaMalloc(ptr, (size_t)bytes));
+    SP_CUDA_TRY(cudaMemset(*ptr, 0, (size_t)bytes));
+    return SP_OK;
+}
+
+extern "C" int sp_device_free(void* ptr) {
+    if (!ptr) return SP_ERR_INVALID_ARG;
+    SP_CUDA_TRY(cudaFree(ptr));
+    return SP_OK;
+}
+
+extern "C" int sp_ipc_get_handle(const void* ptr, uint8_t out[64]) {
+    if (!ptr || !out) return SP_ERR_INVALID_ARG;
+    cudaIpcMemHandle_t h;
+    SP_CUDA_TRY(cudaIpcGetMemHandle(&h, const_cast<void*>(ptr)));
+    static_assert(sizeof(h) == 64, "cudaIpcMemHandle_t is 64 bytes");
+    std::memcpy(out, &h, 64);
+    return SP_OK;
+}
+
+extern "C" int sp_ipc_open_handle(const uint8_t handle[64], void** ptr) {
+    if (!handle || !ptr) return SP_ERR_INVALID_ARG;
+    cudaIpcMemHandle_t h;
+    std::memcpy(&h, handle, 64);
+    SP_CUDA_TRY(cudaIpcOpenMemHandle(ptr, h, cudaIpcMemLazyEnablePeerAccess));
+    return SP_OK;
+}
+
+extern "C" int sp_ipc_close_handle(void* ptr) {
+    if (!ptr) return SP_ERR_INVALID_ARG;
+    SP_CUDA_TRY(cudaIpcCloseMemHandle(ptr));
     return SP_OK;
 }

@@ -169,7 +169,7 @@ def me_frame(f: int, width: int, height: int, search_range: int, seed: int = ME_
         e = (_hash2(seed, 1000 + f, np.broadcast_to(xs, v.shape), np.broadcast_to(ys, v.shape))
              % np.uint64(5)).astype(np.int64) - 2
         v = np.clip(v + e, 0, 255)
-    return v.astype(np.uint8)
+    return np.ascontiguousarray(v, dtype=np.uint8)
 
 
 def me_sequence(n_frames: int, width: int, height: int, search_range: int, seed: int = ME_BENCH_SEED,
