@@ -219,6 +219,22 @@ int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int3
                      int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
                      int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream);
 
+/* Unrestricted motion vectors (reading R-M7): candidates may point
+ * outside the frame; out-of-frame reference pixels take the value of the nearest frame pixel
+ * (edge extension, as in MPEG-4 / H.264 unrestricted MVs), so all (2R+1)^2 candidates are
+ * valid.  ref_padded / cur_padded point at frames edge-extended by `pad` >= R pixels on every
+ * side (sp_me_pad_frames), row pitch `pitch` (multiple of 16, >= width + 2 pad), pair p at
+ * + p*pair_stride; for R in {16, 32} pad must be a multiple of 16.  Outputs as for
+ * sp_me_sad_search over all floor(height/16) macroblock rows. */
+int sp_me_sad_search_unrestricted(const uint8_t* ref_padded, const uint8_t* cur_padded, int64_t pitch, int32_t width,
+                                  int32_t height, int32_t pad, int32_t n_pairs, int64_t pair_stride, int32_t block,
+                                  int32_t range, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream);
+/* Edge-extend n_frames frames (width x height, row pitch src_pitch, frame stride
+ * src_frame_stride) by `pad` pixels on each side into dst (dst_pitch >= width + 2 pad). */
+int sp_me_pad_frames(const uint8_t* src, int64_t src_pitch, int64_t src_frame_stride, int32_t width, int32_t height,
+                     int32_t n_frames, int32_t pad, uint8_t* dst, int64_t dst_pitch, int64_t dst_frame_stride,
+                     void* stream);
+
 /* Reference window the ME kernel stages for macroblock (bx, by): the Alg. 2 bounding box
  * of ref[y0+dy+v][x0+dx+u] over valid candidates, = [y0-R, y0+15+R] x [x0-R, x0+15+R]
  * clipped to the frame (lb/ub as (row, col)).  Host-only. */

@@ -67,6 +67,7 @@ def lib():
         L.spo_me_search.argtypes = [ctypes.c_void_p, ctypes.c_void_p, i64, i32, i32, i32,
                                     ctypes.POINTER(i32), i64, ctypes.POINTER(ctypes.c_int16),
                                     ctypes.POINTER(ctypes.c_uint32), ctypes.POINTER(ctypes.c_uint32)]
+        L.spo_me_search_unrestricted.argtypes = L.spo_me_search.argtypes
         _lib = L
     return _lib
 
@@ -126,7 +127,7 @@ def jacobi1d_points(a0: np.ndarray, steps: int, idx) -> np.ndarray:
 
 
 def me_search(ref: np.ndarray, cur: np.ndarray, width: int, height: int, search_range: int,
-              mbs=None, with_surface: bool = False):
+              mbs=None, with_surface: bool = False, unrestricted: bool = False):
     """Exhaustive SAD search of one (ref, cur) pair.  ref/cur: [height, pitch] uint8.
     Returns (mv [n,2] int16 (dx,dy), sad [n] uint32, surface [n,(2R+1)^2] or None)."""
     ref = np.ascontiguousarray(ref, dtype=np.uint8)
@@ -142,7 +143,8 @@ def me_search(ref: np.ndarray, cur: np.ndarray, width: int, height: int, search_
     sad = np.zeros(n, dtype=np.uint32)
     side = 2 * search_range + 1
     surf = np.zeros((n, side * side), dtype=np.uint32) if with_surface else None
-    lib().spo_me_search(ref.ctypes.data, cur.ctypes.data, pitch, int(width), int(height), int(search_range),
-                        _p(mbs, ctypes.c_int32), n, _p(mv, ctypes.c_int16), _p(sad, ctypes.c_uint32),
-                        _p(surf, ctypes.c_uint32) if surf is not None else None)
+    fn = lib().spo_me_search_unrestricted if unrestricted else lib().spo_me_search
+    fn(ref.ctypes.data, cur.ctypes.data, pitch, int(width), int(height), int(search_range),
+       _p(mbs, ctypes.c_int32), n, _p(mv, ctypes.c_int16), _p(sad, ctypes.c_uint32),
+       _p(surf, ctypes.c_uint32) if surf is not None else None)
     return mv, sad, surf

@@ -256,3 +256,53 @@ void spo_me_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
         sad[q] = best_sad;
     }
 }
+
+/* Unrestricted-MV full search (reading R-M7): every candidate (dx, dy) in
+ * [-R, R]^2 is valid; reference pixels outside the frame take the value of the nearest
+ * frame pixel (edge extension: coordinates clamped to [0, W-1] x [0, H-1]).  Same outputs
+ * and tie-break as spo_me_search. */
+static int spo_clampi(int v, int lo, int hi) { return v < lo ? lo : (v > hi ? hi : v); }
+
+void spo_me_search_unrestricted(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width, int32_t height,
+                                int32_t range, const int32_t* mbs, int64_t n_mbs, int16_t* mv, uint32_t* sad,
+                                uint32_t* surface) {
+    const int B = 16;
+    const int mbx = width / B;
+    const int side = 2 * range + 1;
+#pragma omp parallel for schedule(dynamic, 4)
+    for (int64_t q = 0; q < n_mbs; ++q) {
+        int x0 = B * (mbs[q] % mbx), y0 = B * (mbs[q] / mbx);
+        int found = 0, best_dx = 0, best_dy = 0;
+        uint32_t best_sad = 0;
+        for (int dy = -range; dy <= range; ++dy) {
+            for (int dx = -range; dx <= range; ++dx) {
+                uint32_t s = 0;
+                for (int v = 0; v < B; ++v) {
+                    const uint8_t* c = cur + (int64_t)(y0 + v) * pitch + x0;
+                    const uint8_t* r = ref + (int64_t)spo_clampi(y0 + dy + v, 0, height - 1) * pitch;
+                    for (int u = 0; u < B; ++u)
+                        s += (uint32_t)spo_iabs((int)c[u] - (int)r[spo_clampi(x0 + dx + u, 0, width - 1)]);
+                }
+                int better;
+                if (!found) better = 1;
+                else if (s != best_sad) better = s < best_sad;
+                else {
+                    int l1 = spo_iabs(dx) + spo_iabs(dy), bl1 = spo_iabs(best_dx) + spo_iabs(best_dy);
+                    if (l1 != bl1) better = l1 < bl1;
+                    else if (dy != best_dy) better = dy < best_dy;
+                    else better = dx < best_dx;
+                }
+                if (better) {
+                    found = 1;
+                    best_sad = s;
+                    best_dx = dx;
+                    best_dy = dy;
+                }
+                if (surface) surface[q * (int64_t)side * side + (int64_t)(dy + range) * side + (dx + range)] = s;
+            }
+        }
+        mv[2 * q] = (int16_t)best_dx;
+        mv[2 * q + 1] = (int16_t)best_dy;
+        sad[q] = best_sad;
+    }
+}

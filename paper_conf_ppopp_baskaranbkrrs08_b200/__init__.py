@@ -117,6 +117,8 @@ SYMBOLS = {
     "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
     "sp_jacobi1d_untiled": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_tile_search": (ctypes.c_int, [ctypes.POINTER(sp_tile_problem), ctypes.POINTER(sp_tile_result)]),
+    "sp_me_sad_search_unrestricted": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i64, i32, i32, vp, vp, vp, vp]),
+    "sp_me_pad_frames": (ctypes.c_int, [vp, i64, i64, i32, i32, i32, i32, vp, i64, i64, vp]),
     "sp_jacobi1d_timetiled_peer": (ctypes.c_int, [ctypes.POINTER(sp_peer_links), vp, vp, i64, i64, i64, i32, i32, i32,
                                                   vp]),
     "sp_device_alloc": (ctypes.c_int, [ctypes.POINTER(vp), i64]),
@@ -393,6 +395,38 @@ def me_sad_search_direct(ref, cur, width: int, frame_height: int, search_range: 
                                        int(frame_height), int(n_pairs), int(pair_stride), 16, int(search_range),
                                        int(mb_row_begin), int(mb_row_end), _ptr(mv), _ptr(sad), _ptr(surf),
                                        _stream(stream)), "sp_me_sad_search_direct")
+    return mv, sad, surf
+
+
+def me_pad_frames(frames, width: int, height: int, pad: int, stream=None):
+    """Edge-extend a CUDA uint8 sequence [F, H, pitch] by `pad` pixels (sp_me_pad_frames);
+    returns [F, H + 2 pad, P] with P = width + 2 pad rounded up to 16."""
+    import torch
+    F = frames.shape[0]
+    P = (width + 2 * pad + 15) // 16 * 16
+    out = torch.empty((F, height + 2 * pad, P), dtype=torch.uint8, device=frames.device)
+    _check(lib.sp_me_pad_frames(_ptr(frames), frames.stride(1), frames.stride(0), int(width), int(height), F, int(pad),
+                                _ptr(out), out.stride(1), out.stride(0), _stream(stream)), "sp_me_pad_frames")
+    return out
+
+
+def me_search_sequence_unrestricted(frames, width: int, height: int, search_range: int, with_surface: bool = False,
+                                    stream=None):
+    """Unrestricted-MV search (edge-extended reference) of the consecutive pairs of a CUDA
+    uint8 sequence [F, H, pitch]: pads by max(R, 16) rounded to 16, then searches."""
+    import torch
+    pad = max(16, (int(search_range) + 15) // 16 * 16)
+    padded = me_pad_frames(frames, width, height, pad, stream)
+    ref, cur = padded[:-1], padded[1:]
+    n_pairs = ref.shape[0]
+    mbx, mby = width // 16, height // 16
+    side = 2 * search_range + 1
+    mv = torch.empty((n_pairs, mby, mbx, 2), dtype=torch.int16, device=frames.device)
+    sad = torch.empty((n_pairs, mby, mbx), dtype=torch.int32, device=frames.device)
+    surf = torch.empty((n_pairs, mby, mbx, side * side), dtype=torch.int32, device=frames.device) if with_surface else None
+    _check(lib.sp_me_sad_search_unrestricted(_ptr(ref), _ptr(cur), ref.stride(1), int(width), int(height), pad, n_pairs,
+                                             ref.stride(0), 16, int(search_range), _ptr(mv), _ptr(sad), _ptr(surf),
+                                             _stream(stream)), "sp_me_sad_search_unrestricted")
     return mv, sad, surf
 
 

@@ -47,6 +47,8 @@ struct MeArgs {
     int32_t width, frame_height, row0, range, n_pairs;
     int32_t mbx, mb_row_begin, mb_rows;
     int32_t win;  // window edge = 2R + 16 (bytes per copy row, rows per copy)
+    int32_t pad;           // frames are edge-extended by `pad` pixels (unrestricted mode), else 0
+    int32_t unrestricted;  // 1: every candidate is valid (MVs may point outside the frame)
     int16_t* mv;
     uint32_t* sad;
     uint32_t* surface;
@@ -110,8 +112,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const int by = A.mb_row_begin + (int)(rem / mbx), bx = (int)(rem % mbx);
         const int x0 = kMB * bx, y0 = kMB * by;
         mbar_arrive_expect_tx(&full[s], (uint32_t)(G::kCopy + kMB * kMB));
-        tma_load_3d(smem + s * G::kCopy, &ref_map, x0 - R, y0 - R - A.row0, pair, &full[s]);
-        tma_load_3d(smem + G::kOffCur + s * 256, &cur_map, x0, y0 - A.row0, pair, &full[s]);
+        tma_load_3d(smem + s * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, pair, &full[s]);
+        tma_load_3d(smem + G::kOffCur + s * 256, &cur_map, x0 + A.pad, y0 - A.row0 + A.pad, pair, &full[s]);
     };
 
     if (tid == 0) {
@@ -292,7 +294,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // ---- validity (restricted vectors) only matters near the frame border ----------
         const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
         const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
-        const bool interior = dxlo == -R && dxhi == R && dylo == -R && dyhi == R;
+        const bool interior = A.unrestricted || (dxlo == -R && dxhi == R && dylo == -R && dyhi == R);
         if (!interior) {
 #pragma unroll
             for (int j = 0; j < kTx; ++j) {
@@ -348,7 +350,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         uint32_t M = red32[0];
 #pragma unroll
         for (int w = 1; w < nwarps; ++w) M = min(M, red32[w]);
-        const bool lvalid = (x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf);  // dx = R-1 >= 0, dy = R >= 0
+        const bool lvalid = A.unrestricted || ((x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf));  // dx = R-1, dy = R
         const uint32_t lsad = lsum[s];
         if (lvalid) M = min(M, lsad);
         uint64_t key = ~0ull;
@@ -401,12 +403,13 @@ __global__ void __launch_bounds__(256) me_sad_generic_kernel(const uint8_t* __re
     const uint8_t* cp = cur + (int64_t)pair * pair_stride;
     for (int q = tid; q < win * win; q += nthr) {
         const int wy = q / win, wx = q % win;
-        const int gy = y0 - R + wy - A.row0, gx = x0 - R + wx;
+        const int gy = y0 - R + wy - A.row0 + A.pad, gx = x0 - R + wx + A.pad;
         uint8_t v = 0;
-        if (gy >= 0 && gy < rows_in_buffer && gx >= 0 && gx < A.width) v = rp[(int64_t)gy * pitch + gx];
+        if (gy >= 0 && gy < rows_in_buffer && gx >= 0 && gx < A.width + 2 * A.pad) v = rp[(int64_t)gy * pitch + gx];
         win_s[q] = v;
     }
-    for (int q = tid; q < kMB * kMB; q += nthr) cur_s[q] = cp[(int64_t)(y0 - A.row0 + q / kMB) * pitch + x0 + q % kMB];
+    for (int q = tid; q < kMB * kMB; q += nthr)
+        cur_s[q] = cp[(int64_t)(y0 - A.row0 + A.pad + q / kMB) * pitch + x0 + A.pad + q % kMB];
     __syncthreads();
     const int side = 2 * R + 1;
     const size_t mb_index = ((size_t)pair * A.mb_rows + byr) * A.mbx + bx;
@@ -419,7 +422,8 @@ __global__ void __launch_bounds__(256) me_sad_generic_kernel(const uint8_t* __re
                 const int x = cur_s[v * kMB + u], y = win_s[(dy + R + v) * win + (dx + R + u)];
                 a += (uint32_t)(x > y ? x - y : y - x);
             }
-        const bool valid = (x0 + dx >= 0) && (x0 + dx + 16 <= A.width) && (y0 + dy >= 0) && (y0 + dy + 16 <= A.frame_height);
+        const bool valid = A.unrestricted ||
+                           ((x0 + dx >= 0) && (x0 + dx + 16 <= A.width) && (y0 + dy >= 0) && (y0 + dy + 16 <= A.frame_height));
         const uint64_t k = valid ? make_key(a, dx, dy, R) : ~0ull;
         best = k < best ? k : best;
         if (A.surface) A.surface[mb_index * side * side + c] = valid ? a : 0xffffffffu;
@@ -514,15 +518,16 @@ extern "C" int sp_me_ref_window(int32_t width, int32_t frame_height, int32_t ran
     return SP_OK;
 }
 
-extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
-                                int32_t rows_in_buffer, int32_t row0_global, int32_t frame_height, int32_t n_pairs,
-                                int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
-                                int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream) {
+namespace {
+int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width, int32_t rows_in_buffer,
+                   int32_t row0_global, int32_t frame_height, int32_t n_pairs, int64_t pair_stride, int32_t block,
+                   int32_t range, int32_t mb_row_begin, int32_t mb_row_end, int16_t* mv, uint32_t* best_sad,
+                   uint32_t* surface, void* stream, int32_t pad) {
     if (block != kMB) return SP_ERR_UNSUPPORTED;
     if (!ref || !cur || !mv || !best_sad) return SP_ERR_INVALID_ARG;
     if (range < 0 || range > 63 || width < kMB || frame_height < kMB || n_pairs < 0 || rows_in_buffer < 1)
         return SP_ERR_INVALID_ARG;
-    if (pitch < width || (pitch & 15) || (pair_stride & 15) || (reinterpret_cast<uintptr_t>(ref) & 15) ||
+    if (pitch < width + 2 * pad || (pitch & 15) || (pair_stride & 15) || (reinterpret_cast<uintptr_t>(ref) & 15) ||
         (reinterpret_cast<uintptr_t>(cur) & 15))
         return SP_ERR_INVALID_ARG;
     if (n_pairs > 1 && pair_stride < pitch * rows_in_buffer) return SP_ERR_INVALID_ARG;
@@ -535,14 +540,15 @@ extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t 
     const int rows = mb_row_end - mb_row_begin;
     if (n_pairs == 0 || rows == 0 || mbx == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
-    MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, mv, best_sad, surface};
+    MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, pad,
+             pad > 0 ? 1 : 0, mv, best_sad, surface};
     if (fast_range(range)) {
         CUtensorMap rm, cm;
         int st;
         const int64_t ps = n_pairs > 1 ? pair_stride : pitch * rows_in_buffer;
-        if ((st = make_map(&rm, ref, width, rows_in_buffer, n_pairs, pitch, ps, (uint32_t)a.win, (uint32_t)a.win)))
+        if ((st = make_map(&rm, ref, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, (uint32_t)a.win, (uint32_t)a.win)))
             return st;
-        if ((st = make_map(&cm, cur, width, rows_in_buffer, n_pairs, pitch, ps, kMB, kMB))) return st;
+        if ((st = make_map(&cm, cur, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, kMB, kMB))) return st;
         a.n_pairs = n_pairs;
         const int64_t total = (int64_t)mbx * rows * n_pairs;
         if (range == 32) st = launch_fast<32>(rm, cm, a, total, s);
@@ -558,6 +564,56 @@ extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t 
         SP_CUDA_TRY(attr_err);
         me_sad_generic_kernel<<<dim3(mbx, rows, n_pairs), 256, smem, s>>>(ref, cur, pitch, rows_in_buffer, n_pairs > 1 ? pair_stride : 0, a);
     }
+    SP_CUDA_TRY(cudaGetLastError());
+    return SP_OK;
+}
+
+}  // namespace
+
+extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                                int32_t rows_in_buffer, int32_t row0_global, int32_t frame_height, int32_t n_pairs,
+                                int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
+                                int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream) {
+    return me_search_impl(ref, cur, pitch, width, rows_in_buffer, row0_global, frame_height, n_pairs, pair_stride,
+                          block, range, mb_row_begin, mb_row_end, mv, best_sad, surface, stream, 0);
+}
+
+extern "C" int sp_me_sad_search_unrestricted(const uint8_t* ref_padded, const uint8_t* cur_padded, int64_t pitch,
+                                             int32_t width, int32_t height, int32_t pad, int32_t n_pairs,
+                                             int64_t pair_stride, int32_t block, int32_t range, int16_t* mv,
+                                             uint32_t* best_sad, uint32_t* surface, void* stream) {
+    if (range < 0 || pad < range || (fast_range(range) && (pad % 16)) || pad < 1) return SP_ERR_INVALID_ARG;
+    return me_search_impl(ref_padded, cur_padded, pitch, width, height + 2 * pad, 0, height, n_pairs, pair_stride,
+                          block, range, 0, height / kMB, mv, best_sad, surface, stream, pad);
+}
+
+namespace {
+__global__ void pad_frames_kernel(const uint8_t* __restrict__ src, int64_t spitch, int64_t sstride, int32_t width,
+                                  int32_t height, int32_t pad, uint8_t* __restrict__ dst, int64_t dpitch,
+                                  int64_t dstride) {
+    const int f = blockIdx.z;
+    const int W2 = width + 2 * pad, H2 = height + 2 * pad;
+    for (int y = blockIdx.y * blockDim.y + threadIdx.y; y < H2; y += gridDim.y * blockDim.y) {
+        const int sy = min(max(y - pad, 0), height - 1);
+        const uint8_t* srow = src + (int64_t)f * sstride + (int64_t)sy * spitch;
+        uint8_t* drow = dst + (int64_t)f * dstride + (int64_t)y * dpitch;
+        for (int x = blockIdx.x * blockDim.x + threadIdx.x; x < W2; x += gridDim.x * blockDim.x)
+            drow[x] = srow[min(max(x - pad, 0), width - 1)];
+    }
+}
+}  // namespace
+
+extern "C" int sp_me_pad_frames(const uint8_t* src, int64_t src_pitch, int64_t src_frame_stride, int32_t width,
+                                int32_t height, int32_t n_frames, int32_t pad, uint8_t* dst, int64_t dst_pitch,
+                                int64_t dst_frame_stride, void* stream) {
+    if (!src || !dst || width < 1 || height < 1 || n_frames < 0 || pad < 0 || src_pitch < width ||
+        dst_pitch < width + 2 * pad || (n_frames > 1 && (src_frame_stride < src_pitch * height ||
+                                                         dst_frame_stride < dst_pitch * (height + 2 * pad))))
+        return SP_ERR_INVALID_ARG;
+    if (n_frames == 0) return SP_OK;
+    dim3 block(128, 4), grid((width + 2 * pad + 127) / 128, 64, n_frames);
+    pad_frames_kernel<<<grid, block, 0, (cudaStream_t)stream>>>(src, src_pitch, src_frame_stride, width, height, pad,
+                                                               dst, dst_pitch, dst_frame_stride);
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }

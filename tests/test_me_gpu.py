@@ -109,3 +109,25 @@ def test_host_api_end_to_end():
     omv, osad, _ = _oracle_pair(fr, 2, W, H, R, surface=False)
     assert np.array_equal(mv[2].numpy().reshape(-1, 2), omv)
     assert np.array_equal(sad[2].numpy().view(np.uint32).reshape(-1), osad)
+
+
+@pytest.mark.parametrize("W,H,R", [(64, 48, 5), (352, 288, 16), (130, 70, 32), (64, 64, 32)])
+def test_unrestricted_equals_oracle(W, H, R):
+    fr = sp_inputs.me_sequence(3, W, H, max(R, 2), seed=12, pitch=_pitch(W))
+    d = torch.from_numpy(fr).cuda()
+    mv, sad, surf = sp.me_search_sequence_unrestricted(d, W, H, R, with_surface=True)
+    torch.cuda.synchronize()
+    for p in range(2):
+        omv, osad, osurf = oracle.me_search(fr[p], fr[p + 1], W, H, R, with_surface=True, unrestricted=True)
+        assert np.array_equal(mv[p].cpu().numpy().reshape(-1, 2), omv)
+        assert np.array_equal(sad[p].cpu().numpy().view(np.uint32).reshape(-1), osad)
+        assert np.array_equal(surf[p].cpu().numpy().view(np.uint32).reshape(osurf.shape), osurf)
+
+
+def test_pad_frames_edge_extension():
+    W, H, pad = 50, 30, 16
+    fr = sp_inputs.me_uniform_frames(2, W, H, seed=4, pitch=64)
+    out = sp.me_pad_frames(torch.from_numpy(fr).cuda(), W, H, pad).cpu().numpy()
+    for f in range(2):
+        want = np.pad(fr[f, :, :W], pad, mode="edge")
+        assert np.array_equal(out[f, :, :W + 2 * pad], want)

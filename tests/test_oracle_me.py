@@ -112,3 +112,46 @@ def test_generator_sequence_counter_based():
     mv, sad, _ = oracle.me_search(fr[1], fr[2], 352, 288, 16)
     sad = sad.reshape(18, 22)[2:-2, 2:-2]
     assert np.median(sad) < 256 * 4
+
+
+# ---- unrestricted motion vectors (N4, reading R-M7) ------------------------------------
+def _brute_unrestricted(ref, cur, W, H, R):
+    """Independent twin: numpy edge padding (np.pad mode='edge') + broadcast SADs."""
+    P = R + 16
+    rp = np.pad(ref[:, :W].astype(np.int64), P, mode="edge")
+    mvs, sads = [], []
+    for by in range(H // 16):
+        for bx in range(W // 16):
+            x0, y0 = 16 * bx, 16 * by
+            c = cur[y0:y0 + 16, x0:x0 + 16].astype(np.int64)
+            best = None
+            for dy in range(-R, R + 1):
+                for dx in range(-R, R + 1):
+                    r = rp[P + y0 + dy:P + y0 + dy + 16, P + x0 + dx:P + x0 + dx + 16]
+                    k = (int(np.abs(c - r).sum()), abs(dx) + abs(dy), dy, dx)
+                    best = k if best is None or k < best else best
+            mvs.append((best[3], best[2]))
+            sads.append(best[0])
+    return np.array(mvs), np.array(sads)
+
+
+@pytest.mark.parametrize("W,H,R", [(48, 32, 4), (40, 36, 3), (64, 48, 8)])
+def test_unrestricted_matches_numpy_edge_padding(W, H, R):
+    fr = sp_inputs.me_sequence(2, W, H, max(R, 2), seed=6)
+    mv, sad, _ = oracle.me_search(fr[0], fr[1], W, H, R, unrestricted=True)
+    bmv, bsad = _brute_unrestricted(fr[0], fr[1], W, H, R)
+    assert np.array_equal(mv, bmv) and np.array_equal(sad, bsad)
+
+
+def test_unrestricted_reduces_to_restricted_inside():
+    # interior macroblocks (every candidate inside the frame) give identical results
+    W, H, R = 96, 96, 8
+    fr = sp_inputs.me_sequence(2, W, H, R, seed=8)
+    mv_u, sad_u, _ = oracle.me_search(fr[0], fr[1], W, H, R, unrestricted=True)
+    mv_r, sad_r, _ = oracle.me_search(fr[0], fr[1], W, H, R)
+    for k in range((W // 16) * (H // 16)):
+        bx, by = k % (W // 16), k // (W // 16)
+        if 16 * bx - R >= 0 and 16 * bx + 16 + R <= W and 16 * by - R >= 0 and 16 * by + 16 + R <= H:
+            assert tuple(mv_u[k]) == tuple(mv_r[k]) and sad_u[k] == sad_r[k]
+    # and the unrestricted optimum is never worse
+    assert np.all(sad_u <= sad_r)
