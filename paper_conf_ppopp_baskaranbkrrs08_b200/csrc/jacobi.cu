@@ -292,6 +292,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
                 if (cv <= A.n - 1 && A.n - 1 < cv + kK) fn |= 1ull << (32 + (A.n - 1 - cv));
                 if (0 >= base) v0 = buf[0 - base];
                 if (A.n - 1 - base < kStrip) vn = buf[A.n - 1 - base];
+                __syncwarp();  // these cells belong to other lanes, which overwrite them below
             }
             if (boundary) run_steps<true>(P, A.h, lane, w2, A.mz, f0, fn, v0, vn);
             else run_steps<false>(P, A.h, lane, w2, A.mz, 0ull, 0ull, 0.f, 0.f);

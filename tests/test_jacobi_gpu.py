@@ -56,6 +56,21 @@ def test_time_tiles(tt):
     _check(_run(a, 70, tt, max(4, (S // 3) & ~3)), want)
 
 
+@pytest.mark.parametrize("n,steps,tt,S", [(4099, 37, 16, 256), (4099, 3, 1, 4), (100003, 96, 32, 0), (5, 3, 1, 4)])
+def test_every_cell_written_by_tma_stores(n, steps, tt, S):
+    """Odd pass count: the result is copied back from the work buffer, which the kernel
+    writes only through TMA bulk stores (+ the ragged tail).  Poison work with NaN first;
+    a cell the pass failed to write would surface as NaN (compute-sanitizer's initcheck
+    does not track bulk-async stores, so this test is the evidence it cannot give)."""
+    a0 = sp_inputs.jacobi_input(n, seed=n + steps)
+    d = torch.from_numpy(a0.copy()).cuda()
+    w = torch.full_like(d, float("nan"))
+    sp.jacobi1d_timetiled(d, steps, tt, S, work=w)
+    torch.cuda.synchronize()
+    assert -(-steps // tt) % 2 == 1
+    _check(d.cpu().numpy(), oracle.jacobi1d(a0, steps))
+
+
 def test_fixed_points_on_gpu():
     r = sp_inputs.jacobi_ramp(100000)
     assert np.array_equal(_run(r, 64, 16), r)

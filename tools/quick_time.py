@@ -30,7 +30,8 @@ def main():
     a0 = torch.from_numpy(sp_inputs.jacobi_input(n)).cuda()
     a = a0.clone()
     w = torch.empty_like(a)
-    for tt in [int(x) for x in (sys.argv[1].split(",") if len(sys.argv) > 1 else ["16", "32"])]:
+    pos = [x for x in sys.argv[1:] if not x.startswith("--")]
+    for tt in [int(x) for x in (pos[0].split(",") if pos else ["16", "32"])]:
         def run():
             a.copy_(a0)
             sp.jacobi1d_timetiled(a, T, tt, 0, work=w)

@@ -1,0 +1,36 @@
+"""Small invocations of every device entry point, for compute-sanitizer runs (T6)."""
+import sys
+
+import torch
+
+sys.path.insert(0, ".")
+import paper_conf_ppopp_baskaranbkrrs08_b200 as sp  # noqa: E402
+import sp_inputs  # noqa: E402
+
+
+def mark(what):
+    torch.cuda.synchronize()
+    print(f"[sanitize] {what}", file=sys.stderr, flush=True)
+
+
+a = torch.from_numpy(sp_inputs.jacobi_input(4099, seed=1)).cuda()
+mark("sp.jacobi1d_timetiled")
+sp.jacobi1d_timetiled(a, 37, 16, 256)
+mark("sp.jacobi1d_timetiled")
+sp.jacobi1d_timetiled(a, 20, 5, 0)
+mark("sp.jacobi1d_untiled")
+sp.jacobi1d_untiled(a, 3)
+fr = torch.from_numpy(sp_inputs.me_sequence(3, 352, 288, 16)).cuda()
+mark("sp.me_search_sequence")
+sp.me_search_sequence(fr, 352, 288, 16, with_surface=True)
+fr2 = torch.from_numpy(sp_inputs.me_sequence(2, 130, 70, 32, pitch=144)).cuda()
+mark("sp.me_search_sequence")
+sp.me_search_sequence(fr2, 130, 70, 32)
+mark("sp.me_search_sequence")
+sp.me_search_sequence(fr2, 130, 70, 5)
+mark("sp.me_search_sequence_unrestricted")
+sp.me_search_sequence_unrestricted(fr2, 130, 70, 32)
+mark("sp.me_sad_search_direct")
+sp.me_sad_search_direct(fr2[:-1], fr2[1:], 130, 70, 8)
+torch.cuda.synchronize()
+print("sanitize target done")
