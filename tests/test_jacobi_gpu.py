@@ -122,6 +122,50 @@ def test_J3_size_sampled():
     _check(got[idx], want)
 
 
+def test_J5_full_size_sampled():
+    """BASELINE config 5 at its full size on one GPU: N = 2^30, T = 4096, Tt = 16 (8 GiB of
+    a + work), first as one domain, then through the multi-GPU pass loop with the P = 8 slab
+    decomposition (loopback transport: the same slabs, halos and segment kernel the 8-GPU
+    run uses).  Parity on sampled cells by light-cone windows of width 2T + 1 = 8193
+    (SURVEY §8(d) J5): every slab boundary +- {0, 1, Tt - 1, Tt, Tt + 1}, the domain edges,
+    and 64 random cells."""
+    from paper_conf_ppopp_baskaranbkrrs08_b200.partition import jacobi_slabs
+    n, steps, tt, P = 1 << 30, 4096, 16, 8
+    H = sp.halo_of(tt)
+    a = sp_inputs.jacobi_input(n, seed=2008)
+    slabs = jacobi_slabs(n, P, H)
+    idx = [0, 1, 2, n - 3, n - 2, n - 1]
+    for xb, _ in slabs[1:]:
+        for off in (0, 1, tt - 1, tt, tt + 1):
+            idx += [xb - off, xb + off]
+    idx += np.random.default_rng(5).integers(0, n, 64).tolist()
+    idx = np.unique(np.array(idx, dtype=np.int64))
+    want = oracle.jacobi1d_points(a, steps, idx)
+    d0 = torch.from_numpy(a).cuda()
+    del a
+    tidx = torch.from_numpy(idx).cuda()
+    d = d0.clone()
+    sp.jacobi1d_timetiled(d, steps, tt)
+    torch.cuda.synchronize()
+    _check(d[tidx].cpu().numpy(), want)
+    del d
+    locs, works = [], []
+    for xb, nl in slabs:
+        buf = torch.zeros(nl + 2 * H, dtype=torch.float32, device="cuda")
+        lo, hi = max(0, xb - H), min(n, xb + nl + H)
+        buf[lo - (xb - H): hi - (xb - H)] = d0[lo:hi]
+        locs.append(buf)
+        works.append(torch.zeros_like(buf))
+    del d0
+    sp.jacobi1d_timetiled_loopback(locs, works, n, [s[0] for s in slabs], [s[1] for s in slabs], steps, tt)
+    torch.cuda.synchronize()
+    got = []
+    for i in idx.tolist():
+        r = max(k for k in range(P) if slabs[k][0] <= i)
+        got.append(locs[r][H + i - slabs[r][0]].item())
+    _check(np.array(got, dtype=np.float32), want)
+
+
 @pytest.mark.parametrize("P", [2, 3, 4])
 def test_loopback_partition_equals_oracle(P):
     """The multi-GPU pass loop (slabs + halo exchange + segment kernel) with the
