@@ -37,11 +37,25 @@ namespace {
 using namespace sp::ptx;
 
 constexpr int kMB = 16;      // macroblock edge (WS = 16)
-#ifndef SP_ME_TY
-#define SP_ME_TY 8
-#endif
-constexpr int kTy = SP_ME_TY;  // dy candidates per thread (8, or 4 for twice the threads)
+constexpr int kTy = 8;       // dy candidates per thread
 constexpr int kTx = 4;       // dx candidates per thread (same byte phase, stride 4)
+
+#ifndef SP_ME_EXP
+#define SP_ME_EXP 0
+#endif
+#if SP_ME_EXP & 16  // development instrumentation: per-section cycle counts per warp
+__device__ unsigned long long g_me_prof[8];
+#define PMARK(k)                                              \
+    do {                                                      \
+        const unsigned t_ = (unsigned)clock();                \
+        if (lane == 0) prof_s[warp][k] += t_ - t_prev;        \
+        t_prev = t_;                                          \
+    } while (0)
+#else
+#define PMARK(k) \
+    do {         \
+    } while (0)
+#endif
 
 struct MeArgs {
     int32_t width, frame_height, row0, range, n_pairs;
@@ -68,52 +82,90 @@ __device__ __forceinline__ uint64_t warp_min_key(uint64_t k) {
 }
 
 // Fast path: R in {16, 32} (x0 - R is then 16-byte aligned, as the TMA box origin must
-// be).  Persistent CTAs walk the (pair, MB row, MB column) space; the next-but-one
-// macroblock's window streams in by TMA (double-buffered) while the current one is searched.
+// be).  Persistent CTAs walk the (pair, MB row, MB column) space; the next macroblock's
+// window streams in by TMA (double-buffered) while the current one is searched, and the
+// byte-phase copies are double-buffered too, so ONE CTA barrier per macroblock suffices.
 template <int R>
 struct MeGeom {
     static constexpr int kWin = 2 * R + 16;              // window edge (bytes per row, rows)
     static constexpr int kCopy = kWin * kWin;            // bytes per staged copy (multiple of 128)
     static constexpr int kThreads = R * R / kTy;         // one 4 x kTy candidate tile per thread
-    static constexpr int kSplit = kThreads / (4 * R) > 1 ? kThreads / (4 * R) : 1;  // threads per tail candidate
     static constexpr int kGx = R / 8;                    // dx groups per byte phase
+    static constexpr int kTail = 4 * R + 1;              // candidates outside the 2R x 2R tiling
+    static constexpr int kTailPer = 4 * R / kThreads;    // tail candidates per thread (the last one is split)
     static constexpr int kPhStride = kCopy + 32;         // phase copies at 32-byte bank offsets
     static constexpr int kOffCur = 2 * kCopy;            // cur[2] after raw[2]
-    static constexpr int kOffPh = 2 * kCopy + 512 + 32;  // copy p at kOffPh + (p-1)*kPhStride
-    static constexpr int kSmem = kOffPh + 3 * kPhStride + 128;  // + alignment slack
-    static constexpr int kTail = 4 * R + 1;
+    static constexpr int kOffPh = 2 * kCopy + 512 + 32;  // copy p of stage s at kOffPh + (3s + p-1)*kPhStride
+    static constexpr int kSmem = kOffPh + 6 * kPhStride + 128;  // + alignment slack
+    static_assert(kTailPer * kThreads == 4 * R, "tail candidates must spread evenly");
 };
 
+// 32-bit argmin key: lexicographic (SAD, |dx|+|dy|, dy, dx) in one unsigned compare.
+// Given |dx|+|dy| and dy, |dx| is fixed, so the sign of dx is the only dx information
+// left: key = SAD << 15 | l1 << 8 | (dy + R) << 1 | (dx > 0)   (SAD <= 65280, R <= 32).
+// Invalid candidates carry SAD = kInvalidSad, which keeps them above every valid key.
+constexpr uint32_t kInvalidSad = 0x1FFFFu;
+__device__ __forceinline__ uint32_t tie_bits(int dx, int dy, int R) {
+    return ((uint32_t)(abs(dx) + abs(dy)) << 8) | ((uint32_t)(dy + R) << 1) | (dx > 0 ? 1u : 0u);
+}
+
 template <int R>
-__global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? (kTy == 8 ? 4 : 3) : (kTy == 8 ? 16 : 8)))
+__global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
 me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
     using G = MeGeom<R>;
     constexpr int win = G::kWin;
+    constexpr int side = 2 * R + 1;
+    constexpr int nwarps = (G::kThreads + 31) / 32;
     extern __shared__ __align__(128) uint8_t smem_raw[];
     __shared__ __align__(8) uint64_t full[2];
-    __shared__ uint32_t red32[32];       // per-warp minimal SAD of the current MB
-    __shared__ unsigned int lsum[2];     // per-stage SAD of the leftover tail candidate (dx = R-1, dy = R)
-    __shared__ uint64_t red64[2][32];    // per-stage per-warp best key (published at the next MB)
+    __shared__ uint32_t red32[2][nwarps];  // per-stage per-warp minimal key
+    __shared__ unsigned int lsum[2];       // per-stage SAD of the split tail candidate (dx = R-1, dy = R)
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
 
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
-    constexpr int nwarps = (G::kThreads + 31) / 32;
-    const int mbx = A.mbx;
-    const int64_t per_pair = (int64_t)A.mb_rows * mbx;
-    const int64_t total = per_pair * A.n_pairs;
-    const int64_t Gs = gridDim.x;
+    const uint32_t mbx = (uint32_t)A.mbx;
+    const uint32_t per_pair = (uint32_t)A.mb_rows * mbx;
+    const uint32_t total = per_pair * (uint32_t)A.n_pairs;  // host guarantees < 2^31
+    const uint32_t Gs = gridDim.x;
     const int W = A.width, Hf = A.frame_height;
-    constexpr int side = 2 * R + 1;
-
-    auto issue = [&](int64_t mb, int s) {  // single thread: stage the window + cur of mb
-        const int pair = (int)(mb / per_pair);
-        const int64_t rem = mb - (int64_t)pair * per_pair;
-        const int by = A.mb_row_begin + (int)(rem / mbx), bx = (int)(rem % mbx);
-        const int x0 = kMB * bx, y0 = kMB * by;
-        mbar_arrive_expect_tx(&full[s], (uint32_t)(G::kCopy + kMB * kMB));
-        tma_load_3d(smem + s * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, pair, &full[s]);
-        tma_load_3d(smem + G::kOffCur + s * 256, &cur_map, x0 + A.pad, y0 - A.row0 + A.pad, pair, &full[s]);
+    auto phase_copy = [&](int st, int ph) -> uint8_t* {  // byte phase ph of stage st (ph = 0: raw)
+        return ph == 0 ? smem + st * G::kCopy : smem + G::kOffPh + (3 * st + ph - 1) * G::kPhStride;
+    };
+    struct Pos {
+        int pair, byr, bx;
+    };
+    auto locate = [&](uint32_t mb) -> Pos {
+        const uint32_t pair = mb / per_pair, rem = mb - pair * per_pair;
+        const uint32_t byr = rem / mbx;
+        return Pos{(int)pair, (int)byr, (int)(rem - byr * mbx)};
+    };
+    auto issue = [&](uint32_t mb, int st) {  // single thread: stage the window + cur of mb
+        const Pos q = locate(mb);
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
+        mbar_arrive_expect_tx(&full[st], (uint32_t)(G::kCopy + kMB * kMB));
+        tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair, &full[st]);
+        tma_load_3d(smem + G::kOffCur + st * 256, &cur_map, x0 + A.pad, y0 - A.row0 + A.pad, q.pair, &full[st]);
+    };
+    // Publish macroblock mbp's argmin (stage sp) once every warp has posted its key: the
+    // per-warp minima and the split tail candidate's SAD.
+    auto finalize = [&](uint32_t mbp, int sp) {
+        uint32_t b = red32[sp][0];
+#pragma unroll
+        for (int w = 1; w < nwarps; ++w) b = min(b, red32[sp][w]);
+        const uint32_t lsad = lsum[sp];
+        lsum[sp] = 0u;
+        const Pos q = locate(mbp);
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
+        const bool lvalid = A.unrestricted || ((x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf));  // dx = R-1, dy = R
+        if (lvalid) b = min(b, (lsad << 15) | tie_bits(R - 1, R, R));
+        const size_t idx = ((size_t)q.pair * A.mb_rows + q.byr) * mbx + q.bx;
+        const int dy = (int)((b >> 1) & 127) - R;
+        const int adx = (int)((b >> 8) & 127) - abs(dy);
+        A.mv[2 * idx] = (int16_t)((b & 1) ? adx : -adx);
+        A.mv[2 * idx + 1] = (int16_t)dy;
+        A.sad[idx] = b >> 15;
+        if (A.surface) A.surface[idx * side * side + (size_t)(2 * R) * side + (2 * R - 1)] = lvalid ? lsad : 0xffffffffu;
     };
 
     if (tid == 0) {
@@ -123,41 +175,27 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         mbar_init(&full[1], 1);
         fence_mbar_init();
         lsum[0] = lsum[1] = 0u;
+        if (blockIdx.x < total) issue(blockIdx.x, 0);
     }
     __syncthreads();
-    // Publish macroblock mbp's argmin from the per-warp keys of stage sp (the last warp does
-    // it right after the next macroblock's barrier, when every warp has written its key).
-    auto finalize = [&](int64_t mbp, int sp) {
-        uint64_t b = red64[sp][0];
-#pragma unroll
-        for (int w = 1; w < nwarps; ++w) b = red64[sp][w] < b ? red64[sp][w] : b;
-        lsum[sp] = 0u;
-        const int pr = (int)(mbp / per_pair);
-        const int64_t rm = mbp - (int64_t)pr * per_pair;
-        const size_t idx = ((size_t)pr * A.mb_rows + (size_t)(rm / mbx)) * mbx + (size_t)(rm % mbx);
-        A.mv[2 * idx] = (int16_t)((int)(b & 127) - R);
-        A.mv[2 * idx + 1] = (int16_t)((int)((b >> 7) & 127) - R);
-        A.sad[idx] = (uint32_t)(b >> 21);
-    };
-    if (tid == 0) {
-        if (blockIdx.x < total) issue(blockIdx.x, 0);
-        if (blockIdx.x + Gs < total) issue(blockIdx.x + Gs, 1);
-    }
 
     // thread's candidate tile: dx = -R + p + 4*(4g + j), dy = -R + 8d + i
     const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
-
+#if SP_ME_EXP & 16
+    __shared__ unsigned prof_s[nwarps][8];
+    if (lane == 0)
+        for (int k = 0; k < 8; ++k) prof_s[warp][k] = 0;
+    unsigned t_prev = (unsigned)clock();
+#endif
     int it = 0;
-    for (int64_t mb = blockIdx.x; mb < total; mb += Gs, ++it) {
+    for (uint32_t mb = blockIdx.x; mb < total; mb += Gs, ++it) {
         const int s = it & 1;
-        const int pair = (int)(mb / per_pair);
-        const int64_t rem = mb - (int64_t)pair * per_pair;
-        const int byr = (int)(rem / mbx), bx = (int)(rem % mbx);
-        const int x0 = kMB * bx, y0 = kMB * (A.mb_row_begin + byr);
+        const Pos q = locate(mb);
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         const uint8_t* raw = smem + s * G::kCopy;
         mbar_wait(&full[s], (it >> 1) & 1);
-
-        {   // byte-phase copies p = 1..3: word q of copy p = bytes [4q+p, 4q+p+4) of the row
+        PMARK(0);
+        if (!(SP_ME_EXP & 1)) {  // byte-phase copies p = 1..3: word q of copy p = bytes [4q+p, 4q+p+4) of the row
             constexpr int v4_per_row = win / 16;
             for (int v = tid; v < win * v4_per_row; v += G::kThreads) {
                 const int r = v / v4_per_row, c = v - r * v4_per_row;
@@ -165,33 +203,51 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 const uint4 w = reinterpret_cast<const uint4*>(row)[c];
                 const uint32_t nx = (c + 1 < v4_per_row) ? row[4 * c + 4] : 0u;
 #pragma unroll
-                for (int q = 1; q < 4; ++q) {
+                for (int ph = 1; ph < 4; ++ph) {
                     uint4 o;
-                    o.x = __funnelshift_r(w.x, w.y, 8 * q);
-                    o.y = __funnelshift_r(w.y, w.z, 8 * q);
-                    o.z = __funnelshift_r(w.z, w.w, 8 * q);
-                    o.w = __funnelshift_r(w.w, nx, 8 * q);
-                    reinterpret_cast<uint4*>(smem + G::kOffPh + (q - 1) * G::kPhStride + r * win)[c] = o;
+                    o.x = __funnelshift_r(w.x, w.y, 8 * ph);
+                    o.y = __funnelshift_r(w.y, w.z, 8 * ph);
+                    o.z = __funnelshift_r(w.z, w.w, 8 * ph);
+                    o.w = __funnelshift_r(w.w, nx, 8 * ph);
+                    reinterpret_cast<uint4*>(phase_copy(s, ph) + r * win)[c] = o;
                 }
             }
         }
-        __syncthreads();  // phase copies complete; every warp has finished the previous MB
-        if (tid == nwarps * 32 - 32 && it > 0) finalize(mb - Gs, s ^ 1);
+        PMARK(1);
+        // the only CTA barrier per macroblock: phase copies of stage s complete; every warp
+        // is done with stage s^1 (previous macroblock) and has posted its key for it
+        __syncthreads();
+        if (tid == 0 && mb + Gs < total) {
+            fence_proxy_async_smem();
+            issue(mb + Gs, s ^ 1);
+        }
+        if (tid == G::kThreads - 32 && it > 0) finalize(mb - Gs, s ^ 1);
+        PMARK(2);
 
-        // ---- main 2R x 2R candidates: 4 dx (one byte phase) x 8 dy per thread ----------
+        // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
+        //      thread's tail candidates (column dx = +R, row dy = +R), all in one row loop ----
         uint32_t acc[kTx][kTy];
 #pragma unroll
         for (int j = 0; j < kTx; ++j)
 #pragma unroll
             for (int i = 0; i < kTy; ++i) acc[j][i] = 0;
+        uint32_t ta[G::kTailPer];
+        const uint8_t* tp[G::kTailPer];
+#pragma unroll
+        for (int t = 0; t < G::kTailPer; ++t) {
+            const int c = tid + t * G::kThreads;  // c < 4R
+            const int dxt = (c < side) ? R : -R + (c - side);
+            const int dyt = (c < side) ? -R + c : R;
+            tp[t] = phase_copy(s, (dxt + R) & 3) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
+            ta[t] = 0;
+        }
         {
             // Candidate (j, i) compares cur row v with window row 8d + i + v.  Loop over v with
             // a ring of the 8 window rows in use (row rho in slot rho & 7, 7 words each: the
             // 4 dx candidates x 4 words of one byte phase); body unrolled 8x so every ring
             // index is static, outer loop rolled to halve the code (I-cache).  Innermost
             // order (k, i, j) makes consecutive VABSDIFF4s independent.
-            const uint8_t* base = (p == 0) ? raw : smem + G::kOffPh + (p - 1) * G::kPhStride;
-            const uint8_t* rowp = base + (kTy * d) * win + 16 * g;
+            const uint8_t* rowp = phase_copy(s, p) + (kTy * d) * win + 16 * g;
             const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
             uint32_t Rw[kTy][7];  // words 4g..4g+6 (j + k <= 6)
 #pragma unroll
@@ -202,10 +258,10 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 Rw[rr][4] = w1.x; Rw[rr][5] = w1.y; Rw[rr][6] = w1.z;
             }
 #pragma unroll 1
-            for (int vb = 0; vb < kMB; vb += kTy) {
+            for (int vb = 0; vb < ((SP_ME_EXP & 8) ? 4 * kMB : kMB); vb += kTy) {
 #pragma unroll
                 for (int vv = 0; vv < kTy; ++vv) {
-                    const int v = vb + vv;
+                    const int v = ((SP_ME_EXP & 8) ? (vb & (kMB - 1)) : vb) + vv;
                     {
                         const int slot = (vv + kTy - 1) % kTy;
                         const uint4 w0 = *reinterpret_cast<const uint4*>(rowp + (v + kTy - 1) * win);
@@ -215,6 +271,14 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     }
                     const uint4 cv = cq[v];
                     const uint32_t Cv[4] = {cv.x, cv.y, cv.z, cv.w};
+                    if (!(SP_ME_EXP & 2)) {
+#pragma unroll
+                        for (int t = 0; t < G::kTailPer; ++t) {
+                            const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
+#pragma unroll
+                            for (int k = 0; k < 4; ++k) ta[t] = sad4(tq[k], Cv[k], ta[t]);
+                        }
+                    }
 #pragma unroll
                     for (int k = 0; k < 4; ++k)
 #pragma unroll
@@ -225,59 +289,10 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 }
             }
         }
-        // ---- tail candidates: column dx = +R (dy in [-R, R]) and row dy = +R (dx < R) ----
-        // 4R of the 4R+1 tail candidates spread evenly over the threads; the last one
-        // (dx = R-1, dy = R) is split one 4-pixel word per lane across the warps so that
-        // no warp carries extra work into the reduction barrier
-        // (with kSplit > 1 threads per candidate, each sums kMB/kSplit rows, combined by shuffle)
-        constexpr int KS = G::kSplit;
-        constexpr int kTRows = kMB / KS;
-        constexpr int kTailThreads = G::kThreads / KS;
-        constexpr int kTailPer = (G::kTail - 1 + kTailThreads - 1) / kTailThreads;
-        const int tc = tid / KS, th = tid % KS;
-        uint32_t tacc[kTailPer];
-#pragma unroll
-        for (int t = 0; t < kTailPer; ++t) {
-            const int c = tc + t * kTailThreads;
-            uint32_t a = 0;
-            if (c < G::kTail - 1) {
-                const int dx = (c < side) ? R : -R + (c - side);
-                const int dy = (c < side) ? -R + c : R;
-                const int pp = (dx + R) & 3, m = (dx + R) >> 2;
-                const uint8_t* cb = (pp == 0) ? raw : smem + G::kOffPh + (pp - 1) * G::kPhStride;
-                const uint32_t* rw = reinterpret_cast<const uint32_t*>(cb + (dy + R + th * kTRows) * win) + m;
-                uint32_t a0 = 0, a1 = 0, a2 = 0, a3 = 0;  // four independent chains (latency)
-                const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256) + th * kTRows;
-                if (c < side) {  // column dx = +R: phase 0, word R/2 (16-byte aligned): LDS.128
-#pragma unroll
-                    for (int v = 0; v < kTRows; ++v) {
-                        const uint4 q = *reinterpret_cast<const uint4*>(rw + v * (win / 4));
-                        const uint4 cv = cq[v];
-                        a0 = sad4(q.x, cv.x, a0);
-                        a1 = sad4(q.y, cv.y, a1);
-                        a2 = sad4(q.z, cv.z, a2);
-                        a3 = sad4(q.w, cv.w, a3);
-                    }
-                } else {
-#pragma unroll
-                    for (int v = 0; v < kTRows; ++v) {
-                        const uint32_t* q = rw + v * (win / 4);
-                        const uint4 cv = cq[v];
-                        a0 = sad4(q[0], cv.x, a0);
-                        a1 = sad4(q[1], cv.y, a1);
-                        a2 = sad4(q[2], cv.z, a2);
-                        a3 = sad4(q[3], cv.w, a3);
-                    }
-                }
-                a = (a0 + a1) + (a2 + a3);
-            }
-#pragma unroll
-            for (int o = 1; o < KS; o <<= 1) a += __shfl_xor_sync(0xffffffffu, a, o);
-            tacc[t] = (c < G::kTail - 1 && th == 0) ? a : 0xffffffffu;
-        }
-        {   // leftover: byte phase 3, word R/2 - 1, window rows 2R .. 2R+15
-            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + G::kOffPh + 2 * G::kPhStride + (2 * R) * win) +
-                                 (R / 2 - 1);
+        PMARK(3);
+        {   // split tail candidate (dx = R-1, dy = R): byte phase 3, word R/2 - 1, window rows
+            // 2R .. 2R+15, one (row, word) piece per thread, summed per warp into lsum[s]
+            const uint32_t* rw = reinterpret_cast<const uint32_t*>(phase_copy(s, 3) + (2 * R) * win) + (R / 2 - 1);
             const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
             uint32_t part = 0;
 #pragma unroll
@@ -290,6 +305,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             const uint32_t wsum = __reduce_add_sync(0xffffffffu, part);
             if (lane == 0 && warp * 32 < 64) atomicAdd(&lsum[s], wsum);
         }
+        PMARK(4);
 
         // ---- validity (restricted vectors) only matters near the frame border ----------
         const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
@@ -302,87 +318,64 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
 #pragma unroll
                 for (int i = 0; i < kTy; ++i) {
                     const int dy = -R + kTy * d + i;
-                    if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) acc[j][i] = 0xffffffffu;
+                    if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) acc[j][i] = kInvalidSad;
                 }
             }
 #pragma unroll
-            for (int t = 0; t < kTailPer; ++t) {
-                const int c = tc + t * kTailThreads;
+            for (int t = 0; t < G::kTailPer; ++t) {
+                const int c = tid + t * G::kThreads;
                 const int dx = (c < side) ? R : -R + (c - side);
                 const int dy = (c < side) ? -R + c : R;
-                if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) tacc[t] = 0xffffffffu;
+                if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) ta[t] = kInvalidSad;
             }
         }
-        const size_t mb_index = ((size_t)pair * A.mb_rows + byr) * mbx + bx;
         if (A.surface) {
-            uint32_t* sf = A.surface + mb_index * side * side;
+            uint32_t* sf = A.surface + (((size_t)q.pair * A.mb_rows + q.byr) * mbx + q.bx) * side * side;
 #pragma unroll
             for (int j = 0; j < kTx; ++j)
 #pragma unroll
                 for (int i = 0; i < kTy; ++i)
-                    sf[(kTy * d + i) * side + (p + 4 * (4 * g + j))] = acc[j][i];
+                    sf[(kTy * d + i) * side + (p + 4 * (4 * g + j))] = acc[j][i] == kInvalidSad ? 0xffffffffu : acc[j][i];
 #pragma unroll
-            for (int t = 0; t < kTailPer; ++t) {
-                const int c = tc + t * kTailThreads;
-                if (c < G::kTail - 1 && th == 0) {
-                    const int dx = (c < side) ? R : -R + (c - side);
-                    const int dy = (c < side) ? -R + c : R;
-                    sf[(dy + R) * side + (dx + R)] = tacc[t];
-                }
+            for (int t = 0; t < G::kTailPer; ++t) {
+                const int c = tid + t * G::kThreads;
+                const int dx = (c < side) ? R : -R + (c - side);
+                const int dy = (c < side) ? -R + c : R;
+                sf[(dy + R) * side + (dx + R)] = ta[t] == kInvalidSad ? 0xffffffffu : ta[t];
             }
         }
-        // ---- argmin (SAD, |dx|+|dy|, dy, dx): block min of SAD, then the tie-break key
-        //      only among candidates that reach it (invalid candidates hold 0xFFFFFFFF) ----
-        uint32_t m = 0xffffffffu;
+        // ---- argmin: min over this thread's keys, key(j, i) = acc << 15 | A_j + B_i with
+        //      A_j = |dx_j| << 8 | (dx_j > 0) and B_i = |dy_i| << 8 | (dy_i + R) << 1
+        //      (no carries between the fields), then one CREDUX per warp ----
+        uint32_t key = 0xffffffffu;
 #pragma unroll
-        for (int j = 0; j < kTx; ++j)
+        for (int i = 0; i < kTy; ++i) {
+            const int dy = -R + kTy * d + i;
+            uint32_t ki = 0xffffffffu;
 #pragma unroll
-            for (int i = 0; i < kTy; ++i) m = min(m, acc[j][i]);
-#pragma unroll
-        for (int t = 0; t < kTailPer; ++t) m = min(m, tacc[t]);
-        const uint32_t wm = __reduce_min_sync(0xffffffffu, m);
-        if (lane == 0) red32[warp] = wm;
-        __syncthreads();  // every warp is done with raw[s], cur[s] and the phase copies
-        if (tid == 0 && mb + 2 * Gs < total) {
-            fence_proxy_async_smem();
-            issue(mb + 2 * Gs, s);
-        }
-        uint32_t M = red32[0];
-#pragma unroll
-        for (int w = 1; w < nwarps; ++w) M = min(M, red32[w]);
-        const bool lvalid = A.unrestricted || ((x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf));  // dx = R-1, dy = R
-        const uint32_t lsad = lsum[s];
-        if (lvalid) M = min(M, lsad);
-        uint64_t key = ~0ull;
-        if (m == M) {  // rare: only threads holding a minimal candidate
-#pragma unroll
-            for (int j = 0; j < kTx; ++j)
-#pragma unroll
-                for (int i = 0; i < kTy; ++i)
-                    if (acc[j][i] == M) {
-                        const uint64_t k = make_key(M, -R + p + 4 * (4 * g + j), -R + kTy * d + i, R);
-                        key = k < key ? k : key;
-                    }
-#pragma unroll
-            for (int t = 0; t < kTailPer; ++t) {
-                const int c = tc + t * kTailThreads;
-                if (c < G::kTail - 1 && tacc[t] == M) {
-                    const uint64_t k = make_key(M, (c < side) ? R : -R + (c - side), (c < side) ? -R + c : R, R);
-                    key = k < key ? k : key;
-                }
+            for (int j = 0; j < kTx; ++j) {
+                const int dx = -R + p + 4 * (4 * g + j);
+                ki = min(ki, (acc[j][i] << 15) + (((uint32_t)abs(dx) << 8) | (dx > 0 ? 1u : 0u)));
             }
+            key = min(key, ki + (((uint32_t)abs(dy) << 8) | ((uint32_t)(dy + R) << 1)));
         }
-        if (tid == 0 && lvalid && lsad == M) {
-            const uint64_t k = make_key(M, R - 1, R, R);
-            key = k < key ? k : key;
+#pragma unroll
+        for (int t = 0; t < G::kTailPer; ++t) {
+            const int c = tid + t * G::kThreads;
+            const int dx = (c < side) ? R : -R + (c - side);
+            const int dy = (c < side) ? -R + c : R;
+            key = min(key, (ta[t] << 15) | tie_bits(dx, dy, R));
         }
-        if (tid == 0 && A.surface)
-            A.surface[mb_index * side * side + (size_t)(2 * R) * side + (2 * R - 1)] = lvalid ? lsad : 0xffffffffu;
-        key = warp_min_key(key);
-        if (lane == 0) red64[s][warp] = key;
+        key = __reduce_min_sync(0xffffffffu, key);
+        if (lane == 0) red32[s][warp] = key;
+        PMARK(7);
     }
+#if SP_ME_EXP & 16
+    if (lane == 0)
+        for (int k = 0; k < 8; ++k) atomicAdd(&g_me_prof[k], (unsigned long long)prof_s[warp][k]);
+#endif
     __syncthreads();
-    if (tid == 0 && it > 0) finalize(blockIdx.x + (int64_t)(it - 1) * Gs, (it - 1) & 1);
+    if (tid == G::kThreads - 32 && it > 0) finalize(blockIdx.x + (uint32_t)(it - 1) * Gs, (it - 1) & 1);
 }
 
 // Generic path (any 0 <= R <= 63): window staged byte-wise with zero fill, one thread per
@@ -551,6 +544,7 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
         if ((st = make_map(&cm, cur, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, kMB, kMB))) return st;
         a.n_pairs = n_pairs;
         const int64_t total = (int64_t)mbx * rows * n_pairs;
+        if (total >= (int64_t(1) << 31)) return SP_ERR_UNSUPPORTED;  // 32-bit macroblock indices in the kernel
         if (range == 32) st = launch_fast<32>(rm, cm, a, total, s);
         else st = launch_fast<16>(rm, cm, a, total, s);
         if (st) return st;
@@ -617,3 +611,13 @@ extern "C" int sp_me_pad_frames(const uint8_t* src, int64_t src_pitch, int64_t s
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }
+
+#if SP_ME_EXP & 16
+// development instrumentation only (tools/me_sections.py): read and reset the section counters
+extern "C" int sp_me_prof_read(unsigned long long* out) {
+    SP_CUDA_TRY(cudaMemcpyFromSymbol(out, g_me_prof, sizeof(unsigned long long) * 8));
+    static const unsigned long long zero[8] = {0, 0, 0, 0, 0, 0, 0, 0};
+    SP_CUDA_TRY(cudaMemcpyToSymbol(g_me_prof, zero, sizeof(zero)));
+    return SP_OK;
+}
+#endif

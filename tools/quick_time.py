@@ -31,7 +31,7 @@ def main():
     a = a0.clone()
     w = torch.empty_like(a)
     pos = [x for x in sys.argv[1:] if not x.startswith("--")]
-    for tt in [int(x) for x in (pos[0].split(",") if pos else ["16", "32"])]:
+    for tt in ([] if "--me-only" in sys.argv else [int(x) for x in (pos[0].split(",") if pos else ["16", "32"])]):
         def run():
             a.copy_(a0)
             sp.jacobi1d_timetiled(a, T, tt, 0, work=w)
