@@ -82,21 +82,23 @@ __device__ __forceinline__ uint64_t warp_min_key(uint64_t k) {
 }
 
 // Fast path: R in {16, 32} (x0 - R is then 16-byte aligned, as the TMA box origin must
-// be).  Persistent CTAs walk the (pair, MB row, MB column) space; the next macroblock's
-// window streams in by TMA (double-buffered) while the current one is searched, and the
-// byte-phase copies are double-buffered too, so ONE CTA barrier per macroblock suffices.
+// be).  Persistent CTAs walk the (pair, MB row, MB column) space with a two-stage pipeline:
+// the next macroblock's window and current block stream in by TMA while the current one
+// is searched.  Byte-phase copies are double-buffered, so ONE CTA barrier per macroblock
+// suffices; the argmin of a macroblock is published by one warp after the next barrier.
 template <int R>
 struct MeGeom {
     static constexpr int kWin = 2 * R + 16;              // window edge (bytes per row, rows)
     static constexpr int kCopy = kWin * kWin;            // bytes per staged copy (multiple of 128)
     static constexpr int kThreads = R * R / kTy;         // one 4 x kTy candidate tile per thread
+    static constexpr int kWarps = kThreads / 32;         // 4 (R = 32) or 1 (R = 16)
     static constexpr int kGx = R / 8;                    // dx groups per byte phase
-    static constexpr int kTail = 4 * R + 1;              // candidates outside the 2R x 2R tiling
-    static constexpr int kTailPer = 4 * R / kThreads;    // tail candidates per thread (the last one is split)
-    static constexpr int kPhStride = kCopy + 32;         // phase copies at 32-byte bank offsets
+    static constexpr int kTailPer = 4 * R / kThreads;    // tail candidates per thread (+ the corner, split)
     static constexpr int kOffCur = 2 * kCopy;            // cur[2] after raw[2]
-    static constexpr int kOffPh = 2 * kCopy + 512 + 32;  // copy p of stage s at kOffPh + (3s + p-1)*kPhStride
-    static constexpr int kSmem = kOffPh + 6 * kPhStride + 128;  // + alignment slack
+    static constexpr int kOffPh = 2 * kCopy + 512;       // phase copies (128-byte aligned)
+    static constexpr int kSmem = kOffPh + 6 * kCopy + 3 * 32 + 128;  // + bank offsets + alignment slack
+    static_assert(kCopy % 128 == 0, "copies must keep 128-byte alignment");
+    static_assert(kWarps == 1 || kWarps == 4, "tail mapping assumes 1 or 4 warps");
     static_assert(kTailPer * kThreads == 4 * R, "tail candidates must spread evenly");
 };
 
@@ -109,17 +111,31 @@ __device__ __forceinline__ uint32_t tie_bits(int dx, int dy, int R) {
     return ((uint32_t)(abs(dx) + abs(dy)) << 8) | ((uint32_t)(dy + R) << 1) | (dx > 0 ? 1u : 0u);
 }
 
+// Tail candidate t of thread (warp, lane): the candidates outside the 2R x 2R register
+// tiling — column dx = +R (dy < R) and row dy = +R (dx < R); the corner (R, R) is split
+// over warp 0.  Column and row tails sit in different warps (or different t), so the
+// load path is warp-uniform: a column tail reads 16 aligned bytes (LDS.128, rows 20 words
+// apart: conflict-free per quarter warp), a row tail four words of consecutive dx.
+template <int R>
+__device__ __forceinline__ bool tail_candidate(int warp, int lane, int t, int& dx, int& dy) {
+    const bool col = MeGeom<R>::kWarps == 4 ? warp < 2 : t == 0;
+    const int k = MeGeom<R>::kWarps == 4 ? 32 * (warp & 1) + lane : lane;
+    dx = col ? R : -R + k;
+    dy = col ? -R + k : R;
+    return col;
+}
+
 template <int R>
 __global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
 me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
     using G = MeGeom<R>;
     constexpr int win = G::kWin;
     constexpr int side = 2 * R + 1;
-    constexpr int nwarps = (G::kThreads + 31) / 32;
+    constexpr int nwarps = G::kWarps;
     extern __shared__ __align__(128) uint8_t smem_raw[];
     __shared__ __align__(8) uint64_t full[2];
     __shared__ uint32_t red32[2][nwarps];  // per-stage per-warp minimal key
-    __shared__ unsigned int lsum[2];       // per-stage SAD of the split tail candidate (dx = R-1, dy = R)
+    __shared__ uint32_t lsum[2];           // per-stage SAD of the corner candidate (R, R)
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
 
@@ -129,8 +145,10 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     const uint32_t total = per_pair * (uint32_t)A.n_pairs;  // host guarantees < 2^31
     const uint32_t Gs = gridDim.x;
     const int W = A.width, Hf = A.frame_height;
-    auto phase_copy = [&](int st, int ph) -> uint8_t* {  // byte phase ph of stage st (ph = 0: raw)
-        return ph == 0 ? smem + st * G::kCopy : smem + G::kOffPh + (3 * st + ph - 1) * G::kPhStride;
+    // byte phase ph of stage st (ph = 0: the TMA'd window).  Copy ph starts 32*ph bytes past
+    // a 128-byte boundary, so the four phases a quarter warp reads hit distinct banks.
+    auto phase_copy = [&](int st, int ph) -> uint8_t* {
+        return ph == 0 ? smem + st * G::kCopy : smem + G::kOffPh + (3 * st + ph - 1) * G::kCopy + 32 * ph;
     };
     struct Pos {
         int pair, byr, bx;
@@ -147,25 +165,23 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair, &full[st]);
         tma_load_3d(smem + G::kOffCur + st * 256, &cur_map, x0 + A.pad, y0 - A.row0 + A.pad, q.pair, &full[st]);
     };
-    // Publish macroblock mbp's argmin (stage sp) once every warp has posted its key: the
-    // per-warp minima and the split tail candidate's SAD.
+    // publish macroblock mbp's argmin from stage sp (every warp's key + the corner candidate)
     auto finalize = [&](uint32_t mbp, int sp) {
         uint32_t b = red32[sp][0];
 #pragma unroll
         for (int w = 1; w < nwarps; ++w) b = min(b, red32[sp][w]);
         const uint32_t lsad = lsum[sp];
-        lsum[sp] = 0u;
         const Pos q = locate(mbp);
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
-        const bool lvalid = A.unrestricted || ((x0 + R - 1 + 16 <= W) && (y0 + R + 16 <= Hf));  // dx = R-1, dy = R
-        if (lvalid) b = min(b, (lsad << 15) | tie_bits(R - 1, R, R));
+        const bool lvalid = A.unrestricted || ((x0 + R + 16 <= W) && (y0 + R + 16 <= Hf));
+        if (lvalid) b = min(b, (lsad << 15) | tie_bits(R, R, R));
         const size_t idx = ((size_t)q.pair * A.mb_rows + q.byr) * mbx + q.bx;
         const int dy = (int)((b >> 1) & 127) - R;
         const int adx = (int)((b >> 8) & 127) - abs(dy);
         A.mv[2 * idx] = (int16_t)((b & 1) ? adx : -adx);
         A.mv[2 * idx + 1] = (int16_t)dy;
         A.sad[idx] = b >> 15;
-        if (A.surface) A.surface[idx * side * side + (size_t)(2 * R) * side + (2 * R - 1)] = lvalid ? lsad : 0xffffffffu;
+        if (A.surface) A.surface[idx * side * side + (size_t)side * side - 1] = lvalid ? lsad : 0xffffffffu;
     };
 
     if (tid == 0) {
@@ -174,12 +190,12 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         mbar_init(&full[0], 1);
         mbar_init(&full[1], 1);
         fence_mbar_init();
-        lsum[0] = lsum[1] = 0u;
         if (blockIdx.x < total) issue(blockIdx.x, 0);
     }
     __syncthreads();
 
-    // thread's candidate tile: dx = -R + p + 4*(4g + j), dy = -R + 8d + i
+    // thread's candidate tile: dx = -R + p + 4*(4g + j), dy = -R + 8d + i (a quarter warp
+    // spans the four byte phases: conflict-free LDS.128)
     const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
 #if SP_ME_EXP & 16
     __shared__ unsigned prof_s[nwarps][8];
@@ -192,24 +208,32 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const int s = it & 1;
         const Pos q = locate(mb);
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
-        const uint8_t* raw = smem + s * G::kCopy;
         mbar_wait(&full[s], (it >> 1) & 1);
         PMARK(0);
-        if (!(SP_ME_EXP & 1)) {  // byte-phase copies p = 1..3: word q of copy p = bytes [4q+p, 4q+p+4) of the row
+        {   // byte-phase copies (word q of copy p = bytes [4q+p, 4q+p+4) of the row):
+            // (row, phase) units spread over the CTA, one window row loaded per unit
             constexpr int v4_per_row = win / 16;
-            for (int v = tid; v < win * v4_per_row; v += G::kThreads) {
-                const int r = v / v4_per_row, c = v - r * v4_per_row;
-                const uint32_t* row = reinterpret_cast<const uint32_t*>(raw + r * win);
-                const uint4 w = reinterpret_cast<const uint4*>(row)[c];
-                const uint32_t nx = (c + 1 < v4_per_row) ? row[4 * c + 4] : 0u;
+            const uint8_t* raw = smem + s * G::kCopy;
 #pragma unroll
-                for (int ph = 1; ph < 4; ++ph) {
-                    uint4 o;
-                    o.x = __funnelshift_r(w.x, w.y, 8 * ph);
-                    o.y = __funnelshift_r(w.y, w.z, 8 * ph);
-                    o.z = __funnelshift_r(w.z, w.w, 8 * ph);
-                    o.w = __funnelshift_r(w.w, nx, 8 * ph);
-                    reinterpret_cast<uint4*>(phase_copy(s, ph) + r * win)[c] = o;
+            for (int k = 0; k < (3 * win + G::kThreads - 1) / G::kThreads; ++k) {
+                const int u = tid + k * G::kThreads;
+                if (u < 3 * win) {
+                    const int ph = 1 + u / win, r = u - (ph - 1) * win;
+                    const uint4* rowv = reinterpret_cast<const uint4*>(raw + r * win);
+                    uint4 wv[v4_per_row];
+#pragma unroll
+                    for (int c = 0; c < v4_per_row; ++c) wv[c] = rowv[c];
+                    uint4* out = reinterpret_cast<uint4*>(phase_copy(s, ph) + r * win);
+#pragma unroll
+                    for (int c = 0; c < v4_per_row; ++c) {
+                        const uint32_t nx = c + 1 < v4_per_row ? wv[c + 1].x : 0u;
+                        uint4 o;
+                        o.x = __funnelshift_r(wv[c].x, wv[c].y, 8 * ph);
+                        o.y = __funnelshift_r(wv[c].y, wv[c].z, 8 * ph);
+                        o.z = __funnelshift_r(wv[c].z, wv[c].w, 8 * ph);
+                        o.w = __funnelshift_r(wv[c].w, nx, 8 * ph);
+                        out[c] = o;
+                    }
                 }
             }
         }
@@ -225,7 +249,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         PMARK(2);
 
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
-        //      thread's tail candidates (column dx = +R, row dy = +R), all in one row loop ----
+        //      thread's tail candidates, all in one row loop ----
         uint32_t acc[kTx][kTy];
 #pragma unroll
         for (int j = 0; j < kTx; ++j)
@@ -233,11 +257,11 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             for (int i = 0; i < kTy; ++i) acc[j][i] = 0;
         uint32_t ta[G::kTailPer];
         const uint8_t* tp[G::kTailPer];
+        bool tcol[G::kTailPer];
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) {
-            const int c = tid + t * G::kThreads;  // c < 4R
-            const int dxt = (c < side) ? R : -R + (c - side);
-            const int dyt = (c < side) ? -R + c : R;
+            int dxt, dyt;
+            tcol[t] = tail_candidate<R>(warp, lane, t, dxt, dyt);
             tp[t] = phase_copy(s, (dxt + R) & 3) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
             ta[t] = 0;
         }
@@ -274,9 +298,16 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     if (!(SP_ME_EXP & 2)) {
 #pragma unroll
                         for (int t = 0; t < G::kTailPer; ++t) {
-                            const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
+                            uint32_t tw[4];
+                            if (tcol[t]) {  // warp-uniform
+                                const uint4 w = *reinterpret_cast<const uint4*>(tp[t] + v * win);
+                                tw[0] = w.x; tw[1] = w.y; tw[2] = w.z; tw[3] = w.w;
+                            } else {
+                                const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
+                                tw[0] = tq[0]; tw[1] = tq[1]; tw[2] = tq[2]; tw[3] = tq[3];
+                            }
 #pragma unroll
-                            for (int k = 0; k < 4; ++k) ta[t] = sad4(tq[k], Cv[k], ta[t]);
+                            for (int k = 0; k < 4; ++k) ta[t] = sad4(tw[k], Cv[k], ta[t]);
                         }
                     }
 #pragma unroll
@@ -290,20 +321,19 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
         }
         PMARK(3);
-        {   // split tail candidate (dx = R-1, dy = R): byte phase 3, word R/2 - 1, window rows
-            // 2R .. 2R+15, one (row, word) piece per thread, summed per warp into lsum[s]
-            const uint32_t* rw = reinterpret_cast<const uint32_t*>(phase_copy(s, 3) + (2 * R) * win) + (R / 2 - 1);
+        if (warp == 0) {  // the corner candidate (R, R): 64 (row, word) pieces over warp 0
+            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + s * G::kCopy + (2 * R) * win) + R / 2;
             const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
             uint32_t part = 0;
 #pragma unroll
-            for (int o = tid; o < 64; o += G::kThreads) {
+            for (int o = lane; o < 64; o += 32) {
                 const int v = o >> 2, k = o & 3;
                 const uint4 cv = cq4[v];
                 const uint32_t cw = k == 0 ? cv.x : k == 1 ? cv.y : k == 2 ? cv.z : cv.w;
                 part = sad4(rw[v * (win / 4) + k], cw, part);
             }
-            const uint32_t wsum = __reduce_add_sync(0xffffffffu, part);
-            if (lane == 0 && warp * 32 < 64) atomicAdd(&lsum[s], wsum);
+            const uint32_t tot = __reduce_add_sync(0xffffffffu, part);
+            if (lane == 0) lsum[s] = tot;
         }
         PMARK(4);
 
@@ -323,9 +353,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
 #pragma unroll
             for (int t = 0; t < G::kTailPer; ++t) {
-                const int c = tid + t * G::kThreads;
-                const int dx = (c < side) ? R : -R + (c - side);
-                const int dy = (c < side) ? -R + c : R;
+                int dx, dy;
+                tail_candidate<R>(warp, lane, t, dx, dy);
                 if (dx < dxlo || dx > dxhi || dy < dylo || dy > dyhi) ta[t] = kInvalidSad;
             }
         }
@@ -338,9 +367,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     sf[(kTy * d + i) * side + (p + 4 * (4 * g + j))] = acc[j][i] == kInvalidSad ? 0xffffffffu : acc[j][i];
 #pragma unroll
             for (int t = 0; t < G::kTailPer; ++t) {
-                const int c = tid + t * G::kThreads;
-                const int dx = (c < side) ? R : -R + (c - side);
-                const int dy = (c < side) ? -R + c : R;
+                int dx, dy;
+                tail_candidate<R>(warp, lane, t, dx, dy);
                 sf[(dy + R) * side + (dx + R)] = ta[t] == kInvalidSad ? 0xffffffffu : ta[t];
             }
         }
@@ -361,9 +389,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         }
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) {
-            const int c = tid + t * G::kThreads;
-            const int dx = (c < side) ? R : -R + (c - side);
-            const int dy = (c < side) ? -R + c : R;
+            int dx, dy;
+            tail_candidate<R>(warp, lane, t, dx, dy);
             key = min(key, (ta[t] << 15) | tie_bits(dx, dy, R));
         }
         key = __reduce_min_sync(0xffffffffu, key);
