@@ -104,18 +104,20 @@ struct MeGeom {
 
 // 32-bit argmin key: lexicographic (SAD, |dx|+|dy|, dy, dx) in one unsigned compare.
 // Given |dx|+|dy| and dy, |dx| is fixed, so the sign of dx is the only dx information
-// left: key = SAD << 15 | l1 << 8 | (dy + R) << 1 | (dx > 0)   (SAD <= 65280, R <= 32).
-// Invalid candidates carry SAD = kInvalidSad, which keeps them above every valid key.
-constexpr uint32_t kInvalidSad = 0x1FFFFu;
+// left: tie = l1 << 8 | (dy + R) << 1 | (dx > 0) < 2^15 (R <= 32), and
+// key = SAD * kKeyMul + tie with kKeyMul = 2^15 + 1 > tie orders exactly like (SAD, tie)
+// — a multiplier that is not a power of two keeps the packing on the FMA pipe (IMAD)
+// instead of the ALU the SAD instructions need.  Invalid candidates carry SAD =
+// kInvalidSad, above every valid SAD (<= 65280) and still without 32-bit overflow.
+constexpr uint32_t kKeyMul = 32769u;
+constexpr uint32_t kInvalidSad = 0x1FFF0u;
 __device__ __forceinline__ uint32_t tie_bits(int dx, int dy, int R) {
     return ((uint32_t)(abs(dx) + abs(dy)) << 8) | ((uint32_t)(dy + R) << 1) | (dx > 0 ? 1u : 0u);
 }
 
 // Tail candidate t of thread (warp, lane): the candidates outside the 2R x 2R register
 // tiling — column dx = +R (dy < R) and row dy = +R (dx < R); the corner (R, R) is split
-// over warp 0.  Column and row tails sit in different warps (or different t), so the
-// load path is warp-uniform: a column tail reads 16 aligned bytes (LDS.128, rows 20 words
-// apart: conflict-free per quarter warp), a row tail four words of consecutive dx.
+// over warp 0.  Row tails of one warp read consecutive dx (conflict-free words).
 template <int R>
 __device__ __forceinline__ bool tail_candidate(int warp, int lane, int t, int& dx, int& dy) {
     const bool col = MeGeom<R>::kWarps == 4 ? warp < 2 : t == 0;
@@ -174,13 +176,14 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const Pos q = locate(mbp);
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         const bool lvalid = A.unrestricted || ((x0 + R + 16 <= W) && (y0 + R + 16 <= Hf));
-        if (lvalid) b = min(b, (lsad << 15) | tie_bits(R, R, R));
+        if (lvalid) b = min(b, lsad * kKeyMul + tie_bits(R, R, R));
         const size_t idx = ((size_t)q.pair * A.mb_rows + q.byr) * mbx + q.bx;
-        const int dy = (int)((b >> 1) & 127) - R;
-        const int adx = (int)((b >> 8) & 127) - abs(dy);
-        A.mv[2 * idx] = (int16_t)((b & 1) ? adx : -adx);
+        const uint32_t sad = b / kKeyMul, tie = b - sad * kKeyMul;
+        const int dy = (int)((tie >> 1) & 127) - R;
+        const int adx = (int)((tie >> 8) & 127) - abs(dy);
+        A.mv[2 * idx] = (int16_t)((tie & 1) ? adx : -adx);
         A.mv[2 * idx + 1] = (int16_t)dy;
-        A.sad[idx] = b >> 15;
+        A.sad[idx] = sad;
         if (A.surface) A.surface[idx * side * side + (size_t)side * side - 1] = lvalid ? lsad : 0xffffffffu;
     };
 
@@ -197,6 +200,46 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     // thread's candidate tile: dx = -R + p + 4*(4g + j), dy = -R + 8d + i (a quarter warp
     // spans the four byte phases: conflict-free LDS.128)
     const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
+    // per-thread constants of the epilogue, kept in shared memory instead of registers:
+    // tie bits A_j = |dx_j| << 8 | (dx_j > 0) per (p, g), B_i = |dy_i| << 8 | (dy_i + R) << 1
+    // per d (tie(j, i) = A_j + B_i, no carries between the fields)
+    constexpr int kDy = G::kThreads / (4 * G::kGx);
+    __shared__ uint4 tieA[4 * G::kGx];
+    __shared__ uint4 tieB[kDy][2];
+    if (tid < 4 * G::kGx) {
+        uint32_t a[4];
+        for (int j = 0; j < 4; ++j) {
+            const int dx = -R + (tid & 3) + 4 * (4 * (tid >> 2) + j);
+            a[j] = ((uint32_t)abs(dx) << 8) | (dx > 0 ? 1u : 0u);
+        }
+        tieA[tid] = make_uint4(a[0], a[1], a[2], a[3]);
+    }
+    if (tid < kDy) {
+        uint32_t b[8];
+        for (int i = 0; i < 8; ++i) {
+            const int dy = -R + kTy * tid + i;
+            b[i] = ((uint32_t)abs(dy) << 8) | ((uint32_t)(dy + R) << 1);
+        }
+        tieB[tid][0] = make_uint4(b[0], b[1], b[2], b[3]);
+        tieB[tid][1] = make_uint4(b[4], b[5], b[6], b[7]);
+    }
+    // tail candidates: tie bits and staged-copy offsets (stage 0, stage 1), per thread
+    __shared__ uint32_t tinfo[G::kTailPer][3][G::kThreads];
+#pragma unroll
+    for (int t = 0; t < G::kTailPer; ++t) {
+        int dxt, dyt;
+        tail_candidate<R>(warp, lane, t, dxt, dyt);
+        tinfo[t][0][tid] = tie_bits(dxt, dyt, R);
+#pragma unroll
+        for (int st = 0; st < 2; ++st)
+            tinfo[t][1 + st][tid] =
+                (uint32_t)(phase_copy(st, (dxt + R) & 3) - smem) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
+    }
+    // macroblock position (pair, MB row, MB column) per stage, written by thread 0 one
+    // macroblock ahead, read after the barrier
+    __shared__ Pos posS[2];
+    if (tid == 0) posS[0] = locate(blockIdx.x < total ? blockIdx.x : 0);
+    __syncthreads();
 #if SP_ME_EXP & 16
     __shared__ unsigned prof_s[nwarps][8];
     if (lane == 0)
@@ -206,8 +249,6 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     int it = 0;
     for (uint32_t mb = blockIdx.x; mb < total; mb += Gs, ++it) {
         const int s = it & 1;
-        const Pos q = locate(mb);
-        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         mbar_wait(&full[s], (it >> 1) & 1);
         PMARK(0);
         {   // byte-phase copies (word q of copy p = bytes [4q+p, 4q+p+4) of the row):
@@ -244,6 +285,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         if (tid == 0 && mb + Gs < total) {
             fence_proxy_async_smem();
             issue(mb + Gs, s ^ 1);
+            posS[s ^ 1] = locate(mb + Gs);
         }
         if (tid == G::kThreads - 32 && it > 0) finalize(mb - Gs, s ^ 1);
         PMARK(2);
@@ -257,12 +299,9 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             for (int i = 0; i < kTy; ++i) acc[j][i] = 0;
         uint32_t ta[G::kTailPer];
         const uint8_t* tp[G::kTailPer];
-        bool tcol[G::kTailPer];
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) {
-            int dxt, dyt;
-            tcol[t] = tail_candidate<R>(warp, lane, t, dxt, dyt);
-            tp[t] = phase_copy(s, (dxt + R) & 3) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
+            tp[t] = smem + tinfo[t][1 + s][tid];
             ta[t] = 0;
         }
         {
@@ -298,14 +337,11 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                     if (!(SP_ME_EXP & 2)) {
 #pragma unroll
                         for (int t = 0; t < G::kTailPer; ++t) {
-                            uint32_t tw[4];
-                            if (tcol[t]) {  // warp-uniform
-                                const uint4 w = *reinterpret_cast<const uint4*>(tp[t] + v * win);
-                                tw[0] = w.x; tw[1] = w.y; tw[2] = w.z; tw[3] = w.w;
-                            } else {
-                                const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
-                                tw[0] = tq[0]; tw[1] = tq[1]; tw[2] = tq[2]; tw[3] = tq[3];
-                            }
+                            // four LDS.32 for every tail (one uniform path: a predicated
+                            // LDS.128 variant for the aligned column costs more issue slots
+                            // than the column's 4-way bank conflicts)
+                            const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
+                            const uint32_t tw[4] = {tq[0], tq[1], tq[2], tq[3]};
 #pragma unroll
                             for (int k = 0; k < 4; ++k) ta[t] = sad4(tw[k], Cv[k], ta[t]);
                         }
@@ -338,6 +374,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         PMARK(4);
 
         // ---- validity (restricted vectors) only matters near the frame border ----------
+        const Pos q = posS[s];  // (written one macroblock ahead; stable until the next barrier)
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
         const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
         const bool interior = A.unrestricted || (dxlo == -R && dxhi == R && dylo == -R && dyhi == R);
@@ -372,27 +410,24 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
                 sf[(dy + R) * side + (dx + R)] = ta[t] == kInvalidSad ? 0xffffffffu : ta[t];
             }
         }
-        // ---- argmin: min over this thread's keys, key(j, i) = acc << 15 | A_j + B_i with
-        //      A_j = |dx_j| << 8 | (dx_j > 0) and B_i = |dy_i| << 8 | (dy_i + R) << 1
-        //      (no carries between the fields), then one CREDUX per warp ----
+        // ---- argmin: min over this thread's keys, key(j, i) = acc * kKeyMul + A_j + B_i,
+        //      then one CREDUX per warp ----
         uint32_t key = 0xffffffffu;
+        {
+            const uint4 a4 = tieA[p + 4 * g];
+            const uint32_t Aj[4] = {a4.x, a4.y, a4.z, a4.w};
+            const uint4 b0 = tieB[d][0], b1 = tieB[d][1];
+            const uint32_t Bi[8] = {b0.x, b0.y, b0.z, b0.w, b1.x, b1.y, b1.z, b1.w};
 #pragma unroll
-        for (int i = 0; i < kTy; ++i) {
-            const int dy = -R + kTy * d + i;
-            uint32_t ki = 0xffffffffu;
+            for (int i = 0; i < kTy; ++i) {
+                uint32_t ki = 0xffffffffu;
 #pragma unroll
-            for (int j = 0; j < kTx; ++j) {
-                const int dx = -R + p + 4 * (4 * g + j);
-                ki = min(ki, (acc[j][i] << 15) + (((uint32_t)abs(dx) << 8) | (dx > 0 ? 1u : 0u)));
+                for (int j = 0; j < kTx; ++j) ki = min(ki, acc[j][i] * kKeyMul + Aj[j]);
+                key = min(key, ki + Bi[i]);
             }
-            key = min(key, ki + (((uint32_t)abs(dy) << 8) | ((uint32_t)(dy + R) << 1)));
         }
 #pragma unroll
-        for (int t = 0; t < G::kTailPer; ++t) {
-            int dx, dy;
-            tail_candidate<R>(warp, lane, t, dx, dy);
-            key = min(key, (ta[t] << 15) | tie_bits(dx, dy, R));
-        }
+        for (int t = 0; t < G::kTailPer; ++t) key = min(key, ta[t] * kKeyMul + tinfo[t][0][tid]);
         key = __reduce_min_sync(0xffffffffu, key);
         if (lane == 0) red32[s][warp] = key;
         PMARK(7);
