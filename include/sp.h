@@ -361,6 +361,79 @@ int sp_me_sad_search_direct(const uint8_t* ref, const uint8_t* cur, int64_t pitc
                             int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
                             int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream);
 
+/* =====================================================================================
+ * 6. Generic staged-tile executor: runs an arbitrary small affine
+ *    program block on the GPU exactly as the framework prescribes — local buffers from
+ *    sp_plan_buffers (PER_ARRAY bounding boxes, Alg. 2 / Figure 1),
+ *    accesses rewritten to the local access functions F'(y) - g, move-in
+ *    of the read data spaces before and move-out of the written data spaces after the
+ *    block, tiles mapped to CTAs (outer-level parallel units,
+ *    §5) and consecutive tiles of one CTA sharing a buffer whose movement is
+ *    hoisted out of the tile loop when its data spaces do not change (§4.2).
+ *    Inner-level parallelism: statement instances of a tile are grouped into dependence
+ *    levels (exact flow/anti/output dependences between instances, computed on the host
+ *    in original program order); the CTA's threads run one level at a time.
+ * ===================================================================================== */
+enum { SP_OP_LOAD = 0, SP_OP_CONST = 1, SP_OP_ADD = 2, SP_OP_SUB = 3, SP_OP_MUL = 4 };
+/* One postfix instruction of a statement's right-hand side (fp32, round to nearest, no
+ * contraction).  SP_OP_LOAD pushes the value of read reference `ref` (index into
+ * blk->refs; must belong to the statement and have is_write = 0); SP_OP_CONST pushes
+ * `value`; ADD/SUB/MUL pop b, a and push a op b.  Stack depth <= 16. */
+typedef struct {
+    int32_t op;
+    int32_t ref;
+    float value;
+    int32_t reserved;
+} sp_op;
+/* Body of statement s (the paper prints statement bodies only as S1, S2; Figure 1 gives
+ * A[i][j+1] = A[i+j][j+1]*3 and B[i][j+k] = A[i][k] + B[i+j][k]). */
+typedef struct {
+    int32_t write_ref;    /* the statement's write reference (is_write = 1) */
+    int32_t n_ops;
+    const sp_op* ops;     /* [n_ops] postfix program of the right-hand side */
+    const int32_t* beta;  /* [depth + 1] textual positions: instances execute in the
+                             lexicographic order of (beta_0, i_0, beta_1, ..., i_{d-1}, beta_d),
+                             the original program order (2d+1 schedule) */
+} sp_stmt_body;
+/* Global array `id` (the sp_ref.array ids index this table): fp32, row-major, device memory. */
+typedef struct {
+    float* data;
+    int32_t rank;
+    int32_t reserved;
+    int64_t extent[SP_MAX_RANK];
+} sp_array_desc;
+typedef struct {
+    int32_t n_tiles;             /* the block is instantiated once per tile ... */
+    int32_t tiles_per_cta;       /* ... and consecutive groups of tiles run in one CTA, in order */
+    const int64_t* tile_params;  /* [n_tiles][blk->n_params]: the parameter values of each
+                                    tile (NULL with n_tiles = 1: blk->params) */
+    int32_t hoist;               /* 1: a buffer whose read and write data spaces are identical
+                                    for consecutive tiles of a CTA stays resident (moved in
+                                    before the first, out after the last), §4.2 */
+    int32_t reuse_filter;        /* 1: stage only what Alg. 1 marks beneficial; other
+                                    references access global memory directly */
+    int64_t max_points;          /* planner enumeration budget (0 = default) */
+} sp_exec_opts;
+typedef struct {
+    int64_t instances;           /* statement instances executed */
+    int64_t moved_in;            /* elements moved global -> shared */
+    int64_t moved_out;           /* elements moved shared -> global */
+    int64_t moves_hoisted;       /* element moves saved by hoisting */
+    int32_t max_levels;          /* most dependence levels in one tile */
+    int32_t smem_bytes;          /* dynamic shared memory per CTA */
+    int32_t ctas;                /* CTAs launched */
+    int32_t reserved;
+} sp_exec_stats;
+/* Execute the block.  Tiles in different CTAs must be independent (the caller's FORALL);
+ * tiles of one CTA may depend on each other (they run in order).  Every accessed element
+ * must lie inside its array's extents (else SP_ERR_INVALID_ARG); the staged buffers of a
+ * CTA must fit in shared memory (else SP_ERR_SMEM_LIMIT).  Compiles the per-CTA programs
+ * on the host (synchronous), then launches one kernel on `stream`; the compiled program
+ * lives in device memory allocated and freed stream-ordered (cudaMallocAsync /
+ * cudaFreeAsync) — this is a tool entry point, not a hot path.  stats is nullable. */
+int sp_exec_block(const sp_block* blk, const sp_stmt_body* bodies, const sp_array_desc* arrays, int32_t n_arrays,
+                  const sp_exec_opts* opts, sp_exec_stats* stats, void* stream);
+
 #ifdef __cplusplus
 }
 #endif

@@ -84,6 +84,28 @@ class sp_peer_links(ctypes.Structure):
                 ("left_flags", vp), ("right_flags", vp), ("my_flags", vp), ("epoch0", ctypes.c_uint64)]
 
 
+class sp_op(ctypes.Structure):
+    _fields_ = [("op", i32), ("ref", i32), ("value", ctypes.c_float), ("reserved", i32)]
+
+
+class sp_stmt_body(ctypes.Structure):
+    _fields_ = [("write_ref", i32), ("n_ops", i32), ("ops", ctypes.POINTER(sp_op)), ("beta", ctypes.POINTER(i32))]
+
+
+class sp_array_desc(ctypes.Structure):
+    _fields_ = [("data", vp), ("rank", i32), ("reserved", i32), ("extent", i64 * 8)]
+
+
+class sp_exec_opts(ctypes.Structure):
+    _fields_ = [("n_tiles", i32), ("tiles_per_cta", i32), ("tile_params", ctypes.POINTER(i64)), ("hoist", i32),
+                ("reuse_filter", i32), ("max_points", i64)]
+
+
+class sp_exec_stats(ctypes.Structure):
+    _fields_ = [("instances", i64), ("moved_in", i64), ("moved_out", i64), ("moves_hoisted", i64),
+                ("max_levels", i32), ("smem_bytes", i32), ("ctas", i32), ("reserved", i32)]
+
+
 class sp_tile_problem(ctypes.Structure):
     _fields_ = [("depth", i32), ("n_refs", i32), ("extent", ctypes.POINTER(i64)), ("refs", ctypes.POINTER(sp_ref)),
                 ("n_cand", ctypes.POINTER(i32)), ("cand", ctypes.POINTER(i64)), ("mup_elems", i64), ("procs", i32),
@@ -128,6 +150,8 @@ SYMBOLS = {
     "sp_ipc_close_handle": (ctypes.c_int, [vp]),
     "sp_me_sad_search_direct": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp,
                                                vp, vp]),
+    "sp_exec_block": (ctypes.c_int, [ctypes.POINTER(sp_block), ctypes.POINTER(sp_stmt_body), ctypes.POINTER(sp_array_desc),
+                                     i32, ctypes.POINTER(sp_exec_opts), ctypes.POINTER(sp_exec_stats), vp]),
 }
 
 
@@ -183,12 +207,11 @@ def halo_of(time_tile: int) -> int:
 # ---------------------------------------------------------------------------------------
 # Planner
 # ---------------------------------------------------------------------------------------
-def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_filter: bool = False,
-                 mup_elems: int = 0, max_points: int = 0, cap: int = 64) -> dict:
-    """sp_plan_buffers on a block given as {"params": [...], "stmts": [{"depth", "rows"}],
-    "refs": [{"stmt", "array", "is_write", "rank", "rows"}]} (extra keys ignored)."""
+def _marshal_block(block: dict, P: int | None = None):
+    """sp_block for {"params": [...], "stmts": [{"depth", "rows"}], "refs": [{"stmt", "array",
+    "is_write", "rank", "rows"}]}; returns (blk, keepalive)."""
     params = [int(p) for p in block.get("params", [])]
-    P = len(params)
+    P = len(params) if P is None else P
     keep = []
     doms = (sp_domain * max(1, len(block["stmts"])))()
     for k, s in enumerate(block["stmts"]):
@@ -202,8 +225,19 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
         keep.append(rows)
         refs[k] = sp_ref(int(r["stmt"]), int(r["array"]), int(bool(r["is_write"])), int(r["rank"]),
                          rows.ctypes.data_as(ctypes.POINTER(i64)))
-    par = np.ascontiguousarray(np.asarray(params if params else [0], dtype=np.int64))
+    par = np.ascontiguousarray(np.asarray(params if params else [0] * max(1, P), dtype=np.int64))
+    keep += [doms, refs, par]
     blk = sp_block(P, len(block["stmts"]), len(block["refs"]), 0, par.ctypes.data_as(ctypes.POINTER(i64)), doms, refs)
+    return blk, keep
+
+
+def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_filter: bool = False,
+                 mup_elems: int = 0, max_points: int = 0, cap: int = 64) -> dict:
+    """sp_plan_buffers on a block given as {"params": [...], "stmts": [{"depth", "rows"}],
+    "refs": [{"stmt", "array", "is_write", "rank", "rows"}]} (extra keys ignored)."""
+    params = [int(p) for p in block.get("params", [])]
+    P = len(params)
+    blk, keep = _marshal_block(block)
     opts = sp_plan_opts(int(mode), int(bool(reuse_filter)), float(delta), int(mup_elems), int(max_points))
     n_refs = len(block["refs"])
     ref_buf = (i32 * max(1, n_refs))()
@@ -239,6 +273,48 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
         out["local_rows"].append([list(local[pos + k * w: pos + (k + 1) * w]) for k in range(rk)])
         pos += rk * w
     return out
+
+
+OP_LOAD, OP_CONST, OP_ADD, OP_SUB, OP_MUL = 0, 1, 2, 3, 4
+_OPS = {"load": OP_LOAD, "const": OP_CONST, "add": OP_ADD, "sub": OP_SUB, "mul": OP_MUL}
+
+
+def exec_block(block: dict, bodies: list, arrays: list, tile_params=None, tiles_per_cta: int = 1,
+               hoist: bool = True, reuse_filter: bool = False, max_points: int = 0, stream=None) -> dict:
+    """sp_exec_block (staged-tile executor).  arrays: CUDA float32 contiguous
+    tensors indexed by array id (updated in place).  bodies[s] = {"write_ref": r, "beta": [...],
+    "ops": [(op, arg), ...]} with op in OP_LOAD (arg = ref index), OP_CONST (arg = value),
+    OP_ADD, OP_SUB, OP_MUL (arg ignored).  tile_params: [n_tiles][n_params] (None: one tile with
+    block["params"]).  Returns the sp_exec_stats fields."""
+    import torch
+    P = len(block.get("params", [])) if tile_params is None else (len(tile_params[0]) if len(tile_params) else 0)
+    blk, keep = _marshal_block(block, P)
+    S = len(block["stmts"])
+    bl = (sp_stmt_body * max(1, S))()
+    for k, b in enumerate(bodies):
+        ops = (sp_op * max(1, len(b["ops"])))()
+        for q, (op, arg) in enumerate(b["ops"]):
+            op = _OPS[op] if isinstance(op, str) else int(op)
+            ops[q] = sp_op(op, int(arg) if op == OP_LOAD else 0, float(arg) if op == OP_CONST else 0.0, 0)
+        beta = (i32 * (len(b["beta"])))(*[int(v) for v in b["beta"]])
+        keep += [ops, beta]
+        bl[k] = sp_stmt_body(int(b["write_ref"]), len(b["ops"]), ops, beta)
+    ad = (sp_array_desc * len(arrays))()
+    for k, a in enumerate(arrays):
+        assert a.is_cuda and a.dtype == torch.float32 and a.is_contiguous()
+        ext = (i64 * 8)(*list(a.shape))
+        ad[k] = sp_array_desc(a.data_ptr(), a.dim(), 0, ext)
+    if tile_params is None:
+        tp, n_tiles = None, 1
+    else:
+        tparr = np.ascontiguousarray(np.asarray(tile_params, dtype=np.int64).reshape(len(tile_params), -1))
+        keep.append(tparr)
+        tp, n_tiles = tparr.ctypes.data_as(ctypes.POINTER(i64)), tparr.shape[0]
+    opts = sp_exec_opts(n_tiles, int(tiles_per_cta), tp, int(bool(hoist)), int(bool(reuse_filter)), int(max_points))
+    stats = sp_exec_stats()
+    _check(lib.sp_exec_block(ctypes.byref(blk), bl, ad, len(arrays), ctypes.byref(opts), ctypes.byref(stats),
+                             _stream(stream)), "sp_exec_block")
+    return {f: getattr(stats, f) for f, _ in sp_exec_stats._fields_ if f != "reserved"}
 
 
 def tile_search(extent, refs, candidates, mup_elems: int = 0, procs: int = 32, sync_cost: float = 1.0,

@@ -18,7 +18,7 @@ CSRC = os.path.join(HERE, "csrc")
 LIB = os.path.join(HERE, "libsp.so")
 BUILD_DIR = os.path.join(ROOT, "build", "libsp")
 
-SOURCES = ["api.cpp", "planner.cpp", "comm.cpp", "jacobi.cu", "me.cu", "ablation.cu"]
+SOURCES = ["api.cpp", "planner.cpp", "comm.cpp", "jacobi.cu", "me.cu", "ablation.cu", "exec.cu"]
 HEADERS = ["sp_internal.h", "sm100_ptx.cuh", "sp_nccl_min.h"]
 ARCH = ["-gencode", "arch=compute_100a,code=sm_100a"]
 

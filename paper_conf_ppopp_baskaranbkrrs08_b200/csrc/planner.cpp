@@ -702,3 +702,40 @@ extern "C" int sp_tile_search(const sp_tile_problem* prob, sp_tile_result* out) 
         return SP_ERR_UNSUPPORTED;
     }
 }
+
+// ---------------------------------------------------------------------------------------
+// Domain enumeration for the staged-tile executor (exec.cu): the integer points of one
+// statement polytope with concrete parameters, in lexicographic loop order.
+// ---------------------------------------------------------------------------------------
+namespace sp {
+int enumerate_domain(const sp_domain& D, int n_params, const int64_t* params, int64_t max_points,
+                     std::vector<int64_t>& out, int64_t* count) {
+    try {
+        const int d = D.depth, W = d + n_params + 1;
+        if (d < 0 || d > SP_MAX_DEPTH || D.n_rows < 0 || (D.n_rows > 0 && !D.rows)) return SP_ERR_INVALID_ARG;
+        std::vector<Row> sys;
+        for (int q = 0; q < D.n_rows; ++q) {
+            const i64* row = D.rows + (size_t)q * W;
+            Row r(d + 1);
+            for (int k = 0; k < d; ++k) r[k] = row[k];
+            i128 c = row[d + n_params];
+            for (int p = 0; p < n_params; ++p) c += (i128)row[d + p] * params[p];
+            r[d] = to_i64(c);
+            sys.push_back(r);
+        }
+        const Scan sc = build_scan(sys, d);
+        i64 used = 0;
+        i64 n = 0;
+        scan_points(sc, max_points > 0 ? max_points : kDefaultMaxPoints, used, [&](const i64* x) {
+            out.insert(out.end(), x, x + d);
+            ++n;
+        });
+        *count = n;
+        return SP_OK;
+    } catch (const PlanError& e) {
+        return e.code;
+    } catch (...) {
+        return SP_ERR_UNSUPPORTED;
+    }
+}
+}  // namespace sp

@@ -1,8 +1,16 @@
 // sp_internal.h — private helpers shared by the libsp translation units.
 #pragma once
 #include <cstdint>
+#include <vector>
+
+#include "../../include/sp.h"
 
 namespace sp {
+// integer points of a statement domain with concrete parameters, lexicographic loop order,
+// appended to `out` as depth-long vectors, their number in *count (planner.cpp; used by
+// the executor, exec.cu)
+int enumerate_domain(const sp_domain& D, int n_params, const int64_t* params, int64_t max_points,
+                     std::vector<int64_t>& out, int64_t* count);
 // thread-local last CUDA / NCCL error (see sp_last_cuda_error / sp_last_nccl_error)
 void set_cuda_error(int e);
 void set_nccl_error(int e);
