@@ -413,7 +413,21 @@ typedef struct {
     int32_t reuse_filter;        /* 1: stage only what Alg. 1 marks beneficial; other
                                     references access global memory directly */
     int64_t max_points;          /* planner enumeration budget (0 = default) */
+    int32_t movement;            /* SP_MOVE_ALL or SP_MOVE_DATAFLOW (below) */
+    int32_t dry_run;             /* 1: compile only (stats, move_counts), launch nothing */
+    const int32_t* live_out;     /* [n_arrays] (nullable = all 1): SP_MOVE_DATAFLOW writes back
+                                    a final value only for live-out arrays */
+    int64_t* move_counts;        /* nullable [n_tiles][n_arrays][2]: elements moved in / out */
 } sp_exec_opts;
+/* Data movement of a tile (P:L397-405 default; §3.1.4 P:L450-482 optimised):
+ *   SP_MOVE_ALL      every element of the read data spaces in, of the write data spaces out;
+ *   SP_MOVE_DATAFLOW with the tiles in order as the program: in = elements the tile reads
+ *                    before writing them itself; out = elements whose last write in the tile
+ *                    is read by a later tile before being rewritten, or that no later tile
+ *                    rewrites while their array is live-out (the paper's stated future work,
+ *                    realised exactly on statement instances).  Hoisting is not combined
+ *                    with it (hoist is ignored). */
+enum { SP_MOVE_ALL = 0, SP_MOVE_DATAFLOW = 1 };
 typedef struct {
     int64_t instances;           /* statement instances executed */
     int64_t moved_in;            /* elements moved global -> shared */

@@ -73,3 +73,66 @@ def run_block(block: dict, bodies: list, arrays: list, tile_params=None, boxes=N
             ref = block["refs"][body["write_ref"]]
             out[ref["array"]][_subscript(ref, x, params)] = stack[0]
     return out
+
+
+def movement_sets(block: dict, bodies: list, shapes: list, tile_params=None, boxes=None, live_out=None):
+    """§3.1.4 by direct simulation, with the tiles in order as the program.
+
+    Returns [tile][array] -> (move_in set, move_out set) of element coordinates:
+    * move in  = elements the tile reads before it writes them itself (the value comes
+      from an earlier tile or from the input);
+    * move out = elements the tile writes such that the next later tile touching the
+      element reads it before writing it, or no later tile writes it and the array is
+      live-out (default: every array live-out)."""
+    tiles = tile_params if tile_params is not None else [block.get("params", [])]
+    n_arrays = len(shapes)
+    live = [True] * n_arrays if live_out is None else [bool(v) for v in live_out]
+    trace = []  # per tile: ordered list of (reads [(array, coords)], write (array, coords))
+    for params in tiles:
+        params = [int(p) for p in params]
+        insts = []
+        for s, stmt in enumerate(block["stmts"]):
+            box = boxes[s](params) if callable(boxes[s]) else boxes[s]
+            beta = bodies[s]["beta"]
+            for x in enumerate_domain(stmt, params, box):
+                key = []
+                for k in range(stmt["depth"]):
+                    key += [int(beta[k]), int(x[k])]
+                key.append(int(beta[stmt["depth"]]))
+                insts.append((key, s, tuple(int(v) for v in x)))
+        insts.sort(key=lambda t: (t[0], t[1]))
+        ops = []
+        for _, s, x in insts:
+            reads = [(block["refs"][a]["array"], _subscript(block["refs"][a], x, params))
+                     for op, a in bodies[s]["ops"] if op == LOAD]
+            w = block["refs"][bodies[s]["write_ref"]]
+            ops.append((reads, (w["array"], _subscript(w, x, params))))
+        trace.append(ops)
+
+    def first_access(t, e):  # 'r' (read before any write), 'w', or None
+        for reads, w in trace[t]:
+            if e in reads:
+                return "r"
+            if w == e:
+                return "w"
+        return None
+
+    out = []
+    for t, ops in enumerate(trace):
+        written, mi, mo = set(), [set() for _ in range(n_arrays)], [set() for _ in range(n_arrays)]
+        for reads, w in ops:
+            for e in reads:
+                if e not in written:
+                    mi[e[0]].add(e[1])
+            written.add(w)
+        for e in written:
+            need = live[e[0]]
+            for t2 in range(t + 1, len(trace)):
+                f = first_access(t2, e)
+                if f is not None:
+                    need = f == "r"
+                    break
+            if need:
+                mo[e[0]].add(e[1])
+        out.append([(mi[a], mo[a]) for a in range(n_arrays)])
+    return out

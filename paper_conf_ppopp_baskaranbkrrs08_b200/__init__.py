@@ -98,7 +98,8 @@ class sp_array_desc(ctypes.Structure):
 
 class sp_exec_opts(ctypes.Structure):
     _fields_ = [("n_tiles", i32), ("tiles_per_cta", i32), ("tile_params", ctypes.POINTER(i64)), ("hoist", i32),
-                ("reuse_filter", i32), ("max_points", i64)]
+                ("reuse_filter", i32), ("max_points", i64), ("movement", i32), ("dry_run", i32),
+                ("live_out", ctypes.POINTER(i32)), ("move_counts", ctypes.POINTER(i64))]
 
 
 class sp_exec_stats(ctypes.Structure):
@@ -279,8 +280,12 @@ OP_LOAD, OP_CONST, OP_ADD, OP_SUB, OP_MUL = 0, 1, 2, 3, 4
 _OPS = {"load": OP_LOAD, "const": OP_CONST, "add": OP_ADD, "sub": OP_SUB, "mul": OP_MUL}
 
 
+MOVE_ALL, MOVE_DATAFLOW = 0, 1
+
+
 def exec_block(block: dict, bodies: list, arrays: list, tile_params=None, tiles_per_cta: int = 1,
-               hoist: bool = True, reuse_filter: bool = False, max_points: int = 0, stream=None) -> dict:
+               hoist: bool = True, reuse_filter: bool = False, max_points: int = 0, movement: int = MOVE_ALL,
+               live_out=None, dry_run: bool = False, stream=None) -> dict:
     """sp_exec_block (staged-tile executor).  arrays: CUDA float32 contiguous
     tensors indexed by array id (updated in place).  bodies[s] = {"write_ref": r, "beta": [...],
     "ops": [(op, arg), ...]} with op in OP_LOAD (arg = ref index), OP_CONST (arg = value),
@@ -301,20 +306,25 @@ def exec_block(block: dict, bodies: list, arrays: list, tile_params=None, tiles_
         bl[k] = sp_stmt_body(int(b["write_ref"]), len(b["ops"]), ops, beta)
     ad = (sp_array_desc * len(arrays))()
     for k, a in enumerate(arrays):
-        assert a.is_cuda and a.dtype == torch.float32 and a.is_contiguous()
+        assert a.dtype == torch.float32 and a.is_contiguous() and (a.is_cuda or dry_run)
         ext = (i64 * 8)(*list(a.shape))
-        ad[k] = sp_array_desc(a.data_ptr(), a.dim(), 0, ext)
+        ad[k] = sp_array_desc(a.data_ptr() if a.is_cuda else 16, a.dim(), 0, ext)
     if tile_params is None:
         tp, n_tiles = None, 1
     else:
         tparr = np.ascontiguousarray(np.asarray(tile_params, dtype=np.int64).reshape(len(tile_params), -1))
         keep.append(tparr)
         tp, n_tiles = tparr.ctypes.data_as(ctypes.POINTER(i64)), tparr.shape[0]
-    opts = sp_exec_opts(n_tiles, int(tiles_per_cta), tp, int(bool(hoist)), int(bool(reuse_filter)), int(max_points))
+    lo = None if live_out is None else (i32 * len(arrays))(*[int(bool(v)) for v in live_out])
+    counts = (i64 * (2 * n_tiles * len(arrays)))()
+    opts = sp_exec_opts(n_tiles, int(tiles_per_cta), tp, int(bool(hoist)), int(bool(reuse_filter)), int(max_points),
+                        int(movement), int(bool(dry_run)), lo, counts)
     stats = sp_exec_stats()
     _check(lib.sp_exec_block(ctypes.byref(blk), bl, ad, len(arrays), ctypes.byref(opts), ctypes.byref(stats),
-                             _stream(stream)), "sp_exec_block")
-    return {f: getattr(stats, f) for f, _ in sp_exec_stats._fields_ if f != "reserved"}
+                             None if dry_run else _stream(stream)), "sp_exec_block")
+    out = {f: getattr(stats, f) for f, _ in sp_exec_stats._fields_ if f != "reserved"}
+    out["move_counts"] = np.array(counts[:], dtype=np.int64).reshape(n_tiles, len(arrays), 2)
+    return out
 
 
 def tile_search(extent, refs, candidates, mup_elems: int = 0, procs: int = 32, sync_cost: float = 1.0,

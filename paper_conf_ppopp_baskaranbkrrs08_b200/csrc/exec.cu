@@ -97,11 +97,26 @@ struct Error {
 };
 
 // ---- per-tile compilation -------------------------------------------------------------
+struct Inst {
+    std::vector<int64_t> key;      // 2d+1 schedule key (original order)
+    std::vector<int32_t> rec;      // device record
+    int64_t w_elem;                // element keys: array << 40 | global flat index
+    std::vector<int64_t> r_elems;
+    int level;
+};
+
 struct TileInfo {
     std::vector<sp_buffer> bufs;          // planner output
     std::vector<int32_t> ref_buf;         // per ref
     std::vector<int64_t> local_rows;      // per ref, rank x (depth + P + 1)
-    std::vector<std::vector<int64_t>> rd, wr;  // per array id: sorted global flat indices read / written via staged refs
+    std::vector<std::vector<int64_t>> rd, wr;  // per array id: sorted element keys read / written via staged refs
+    std::vector<Inst> list;                    // instances in original program order
+    std::vector<std::vector<int64_t>> din, dout;  // SP_MOVE_DATAFLOW: the §3.1.4 subsets of rd / wr
+};
+
+struct Group {  // the tiles one CTA runs, and its shared-memory slot per array
+    std::vector<TileInfo> tiles;
+    std::vector<int64_t> slot_off;
 };
 
 int64_t dot(const int64_t* row, const int64_t* x, int d, const int64_t* p, int P) {
@@ -120,6 +135,7 @@ struct Compiler {
     sp_exec_opts o;
     // outputs
     std::vector<int32_t> runs, segs, moves, insts, code, stmt_code;
+    std::vector<Group> groups;
     int rec = 3;
     int32_t smem_elems = 0;
     sp_exec_stats st{};
@@ -153,6 +169,44 @@ struct Compiler {
         t.rd.assign(n_arrays, {});
         t.wr.assign(n_arrays, {});
         return t;
+    }
+
+    bool live_out(int64_t e) const { return !o.live_out || o.live_out[e >> 40]; }
+
+    // §3.1.4, exact on instances, with the tiles in order as the program:
+    //   move in  = elements a tile reads before writing them itself (their value comes from
+    //              an earlier tile or from the input),
+    //   move out = elements whose last write in the tile is read by a later tile before it
+    //              is rewritten, or that no later tile rewrites while their array is live-out.
+    void dataflow() {
+        std::vector<TileInfo*> all;
+        for (Group& g : groups)
+            for (TileInfo& t : g.tiles) all.push_back(&t);
+        std::vector<std::unordered_map<int64_t, char>> exposed(all.size()), written(all.size());
+        for (size_t t = 0; t < all.size(); ++t) {
+            auto& W = written[t];
+            for (const Inst& I : all[t]->list) {
+                for (int64_t e : I.r_elems)
+                    if (!W.count(e)) exposed[t][e] = 1;
+                W[I.w_elem] = 1;
+            }
+        }
+        std::unordered_map<int64_t, char> needed;  // after tile t: is the value of e needed later?
+        for (size_t t = all.size(); t-- > 0;) {
+            TileInfo& T = *all[t];
+            T.din.assign(n_arrays, {});
+            T.dout.assign(n_arrays, {});
+            for (int a = 0; a < n_arrays; ++a) {
+                for (int64_t e : T.wr[a]) {
+                    auto it = needed.find(e);
+                    if (it != needed.end() ? it->second : live_out(e)) T.dout[a].push_back(e);
+                }
+                for (int64_t e : T.rd[a])
+                    if (exposed[t].count(e)) T.din[a].push_back(e);
+            }
+            for (auto& kv : written[t]) needed[kv.first] = 0;
+            for (auto& kv : exposed[t]) needed[kv.first] = 1;
+        }
     }
 
     void compile() {
@@ -218,14 +272,6 @@ struct Compiler {
             smem_elems = std::max<int32_t>(smem_elems, (int32_t)tot);
 
             // instances, operands, data spaces, levels — per tile
-            struct Inst {
-                std::vector<int64_t> key;
-                std::vector<int32_t> rec;
-                int64_t w_elem;
-                std::vector<int64_t> r_elems;
-                int level;
-            };
-            std::vector<std::vector<Inst>> per_tile(tiles.size());
             for (size_t ti = 0; ti < tiles.size(); ++ti) {
                 TileInfo& TI = tiles[ti];
                 const int64_t* params = tp + (size_t)(g0 + ti) * P;
@@ -238,7 +284,7 @@ struct Compiler {
                     lr_at[r] = lr_pos;
                     lr_pos += (size_t)blk.refs[r].rank * (blk.stmts[blk.refs[r].stmt].depth + P + 1);
                 }
-                std::vector<Inst>& list = per_tile[ti];
+                std::vector<Inst>& list = TI.list;
                 for (int s = 0; s < S; ++s) {
                     const sp_domain& D = blk.stmts[s];
                     const int d = D.depth;
@@ -327,10 +373,19 @@ struct Compiler {
                 }
             }
 
+            groups.push_back(Group{std::move(tiles), std::move(slot_off)});
+        }
+        if (o.movement == SP_MOVE_DATAFLOW) dataflow();
+        int64_t tile_base = 0;
+        for (Group& grp : groups) {
+            std::vector<TileInfo>& tiles = grp.tiles;
+            const std::vector<int64_t>& slot_off = grp.slot_off;
             // emit the CTA's segments
             const int32_t seg_first = (int32_t)(segs.size() / 3);
-            auto emit_moves = [&](int kind, const TileInfo& TI, int a) {
-                const std::vector<int64_t>& set = kind == kSegIn ? TI.rd[a] : TI.wr[a];
+            auto emit_moves = [&](int kind, const TileInfo& TI, int a, int64_t tile) {
+                const bool df = o.movement == SP_MOVE_DATAFLOW;
+                const std::vector<int64_t>& set = kind == kSegIn ? (df ? TI.din[a] : TI.rd[a]) : (df ? TI.dout[a] : TI.wr[a]);
+                if (o.move_counts) o.move_counts[(tile * n_arrays + a) * 2 + (kind == kSegIn ? 0 : 1)] = (int64_t)set.size();
                 if (set.empty()) return;
                 const sp_buffer* Bf = nullptr;
                 for (auto& b : TI.bufs)
@@ -361,14 +416,20 @@ struct Compiler {
             auto same_spaces = [&](const TileInfo& x, const TileInfo& y, int a) {
                 return x.rd[a] == y.rd[a] && x.wr[a] == y.wr[a];
             };
+            const bool hoist = o.hoist && o.movement != SP_MOVE_DATAFLOW;
             for (size_t ti = 0; ti < tiles.size(); ++ti) {
                 const TileInfo& TI = tiles[ti];
+                const int64_t tile = tile_base + (int64_t)ti;
                 for (int a = 0; a < n_arrays; ++a) {
-                    const bool resident = o.hoist && ti > 0 && same_spaces(tiles[ti - 1], TI, a);
-                    if (resident) st.moves_hoisted += (int64_t)TI.rd[a].size();
-                    else emit_moves(kSegIn, TI, a);
+                    const bool resident = hoist && ti > 0 && same_spaces(tiles[ti - 1], TI, a);
+                    if (resident) {
+                        st.moves_hoisted += (int64_t)TI.rd[a].size();
+                        if (o.move_counts) o.move_counts[(tile * n_arrays + a) * 2] = 0;
+                    } else {
+                        emit_moves(kSegIn, TI, a, tile);
+                    }
                 }
-                std::vector<Inst>& list = per_tile[ti];
+                std::vector<Inst>& list = tiles[ti].list;
                 int nl = 0;
                 for (auto& I : list) nl = std::max(nl, I.level + 1);
                 st.max_levels = std::max(st.max_levels, nl);
@@ -384,11 +445,16 @@ struct Compiler {
                     segs.push_back((int32_t)(insts.size() / rec) - first);
                 }
                 for (int a = 0; a < n_arrays; ++a) {
-                    const bool stays = o.hoist && ti + 1 < tiles.size() && same_spaces(tiles[ti + 1], TI, a);
-                    if (stays) st.moves_hoisted += (int64_t)TI.wr[a].size();
-                    else emit_moves(kSegOut, TI, a);
+                    const bool stays = hoist && ti + 1 < tiles.size() && same_spaces(tiles[ti + 1], TI, a);
+                    if (stays) {
+                        st.moves_hoisted += (int64_t)TI.wr[a].size();
+                        if (o.move_counts) o.move_counts[(tile * n_arrays + a) * 2 + 1] = 0;
+                    } else {
+                        emit_moves(kSegOut, TI, a, tile);
+                    }
                 }
             }
+            tile_base += (int64_t)tiles.size();
             runs.push_back(seg_first);
             runs.push_back((int32_t)(segs.size() / 3) - seg_first);
         }
@@ -411,6 +477,7 @@ extern "C" int sp_exec_block(const sp_block* blk, const sp_stmt_body* bodies, co
                              int32_t n_arrays, const sp_exec_opts* opts, sp_exec_stats* stats, void* stream) {
     if (!blk || !bodies || !arrays || n_arrays < 1 || !opts) return SP_ERR_INVALID_ARG;
     if (opts->n_tiles < 1 || opts->tiles_per_cta < 1) return SP_ERR_INVALID_ARG;
+    if (opts->movement != SP_MOVE_ALL && opts->movement != SP_MOVE_DATAFLOW) return SP_ERR_INVALID_ARG;
     if (blk->n_params > 0 && !opts->tile_params && !(opts->n_tiles == 1 && blk->params)) return SP_ERR_INVALID_ARG;
     for (int a = 0; a < n_arrays; ++a)
         if (arrays[a].rank < 1 || arrays[a].rank > SP_MAX_RANK) return SP_ERR_INVALID_ARG;
@@ -424,6 +491,7 @@ extern "C" int sp_exec_block(const sp_block* blk, const sp_stmt_body* bodies, co
         return SP_ERR_UNSUPPORTED;
     }
     if (stats) *stats = C.st;
+    if (opts->dry_run) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
     std::vector<float*> ptrs(n_arrays);
     for (int a = 0; a < n_arrays; ++a) ptrs[a] = arrays[a].data;

@@ -71,3 +71,17 @@ def chain(n, war=False):
         ops = [(LOAD, 1), (LOAD, 2), (ADD, 0)]
     blk = {"params": [], "stmts": [{"depth": 1, "rows": dom}], "refs": refs}
     return blk, [{"write_ref": 0, "beta": [0, 0], "ops": ops}], [[(0, n - 1)]]
+
+
+def pipeline(n):
+    """t[i] = a[i] * 2 (S1); b[i] = t[i] + 1 (S2), both in one loop over i (t is a temporary
+    when not live-out).  Arrays: a = 0, t = 1, b = 2."""
+    dom = [[1, 0], [-1, n - 1]]
+
+    def r(s, a, w):
+        return {"stmt": s, "array": a, "is_write": w, "rank": 1, "rows": [[1, 0]]}
+    blk = {"params": [], "stmts": [{"depth": 1, "rows": dom}, {"depth": 1, "rows": dom}],
+           "refs": [r(0, 1, 1), r(0, 0, 0), r(1, 2, 1), r(1, 1, 0)]}
+    bodies = [{"write_ref": 0, "beta": [0, 0], "ops": [(LOAD, 1), (CONST, 2.0), (MUL, 0)]},
+              {"write_ref": 2, "beta": [0, 1], "ops": [(LOAD, 3), (CONST, 1.0), (ADD, 0)]}]
+    return blk, bodies, [[(0, n - 1)], [(0, n - 1)]]

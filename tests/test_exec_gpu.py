@@ -83,3 +83,34 @@ def test_rejects_out_of_bounds_access():
     a = torch.zeros(5, device="cuda")  # the block touches a[0..9]
     with pytest.raises(sp.SPError):
         sp.exec_block(blk, bodies, [a])
+
+
+def test_dataflow_movement_results():
+    """§3.1.4 movement changes what is moved, never the live-out results."""
+    blk, bodies, boxes, _ = X.figure1()
+    rng = np.random.default_rng(5)
+    A = rng.standard_normal((200, 200)).astype(np.float32)
+    B = rng.standard_normal((200, 200)).astype(np.float32)
+    want = run_block(blk, bodies, [A, B], boxes=boxes)
+    got, st = _gpu([A, B], blk, bodies, movement=sp.MOVE_DATAFLOW)
+    assert np.array_equal(got[0], want[0]) and np.array_equal(got[1], want[1])
+    assert st["moved_in"] == 70 + 90 and st["moved_out"] == 25 + 70
+    n, m, t = 70, 100, 16
+    blk, bodies, boxes, tiles = X.matvec(n, m, t)
+    arrs = [rng.standard_normal(n).astype(np.float32), rng.standard_normal((n, m)).astype(np.float32),
+            rng.standard_normal(m).astype(np.float32)]
+    want = run_block(blk, bodies, arrs, tile_params=tiles, boxes=boxes)
+    got, st = _gpu(arrs, blk, bodies, tile_params=tiles, tiles_per_cta=(m + t - 1) // t, movement=sp.MOVE_DATAFLOW)
+    assert np.array_equal(got[0], want[0])
+
+
+def test_dataflow_temporary_stays_on_chip():
+    n = 1000
+    blk, bodies, boxes = X.pipeline(n)
+    rng = np.random.default_rng(6)
+    arrs = [rng.standard_normal(n).astype(np.float32), np.full(n, 7.0, np.float32), np.zeros(n, np.float32)]
+    want = run_block(blk, bodies, arrs, boxes=boxes)
+    got, st = _gpu(arrs, blk, bodies, movement=sp.MOVE_DATAFLOW, live_out=[1, 0, 1])
+    assert np.array_equal(got[2], want[2])  # b = a * 2 + 1
+    assert np.all(got[1] == 7.0)            # t was produced and consumed in shared memory only
+    assert st["moved_in"] == n and st["moved_out"] == n
