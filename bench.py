@@ -426,7 +426,7 @@ def main():
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--time-tile", type=int, default=32)
+    ap.add_argument("--time-tile", type=int, default=64)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--halo", choices=["peer", "nccl"], default="peer",
                     help="multi-GPU Jacobi halo exchange: fused peer stores in the pass kernel, or NCCL send/recv")

@@ -345,8 +345,8 @@ Variant make_variant() {
     return v;
 }
 
-constexpr int kNumVariants = 5;
-constexpr int kDefaultVariant = 0;
+constexpr int kNumVariants = 6;
+constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
 
 Variant* variants() {
     static Variant v[kNumVariants] = {
@@ -355,6 +355,7 @@ Variant* variants() {
         make_variant<JCfg<20, 4, 4>>(),  // 2: 40 cells/lane, <= 128 regs
         make_variant<JCfg<28, 4, 4>>(),  // 3: 56 cells/lane, <= 128 regs
         make_variant<JCfg<20, 2, 8>>(),  // 4: 40 cells/lane, 2 warps/CTA, <= 128 regs
+        make_variant<JCfg<28, 8, 2>>(),  // 5: 56 cells/lane, 8 warps/CTA (224 KB of stages per SM)
     };
     return v;
 }

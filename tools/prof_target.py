@@ -10,7 +10,7 @@ import sp_inputs  # noqa: E402
 
 what = sys.argv[1]
 if what == "jacobi":
-    tt = int(sys.argv[2]) if len(sys.argv) > 2 else 16
+    tt = int(sys.argv[2]) if len(sys.argv) > 2 else 64
     n = 1 << 26
     a = torch.from_numpy(sp_inputs.jacobi_input(n)).cuda()
     w = torch.empty_like(a)
