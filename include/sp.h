@@ -182,6 +182,19 @@ int sp_jacobi1d_tile_footprint(int64_t n, int32_t h, int64_t x0, int64_t space_t
  * staged footprint as the kernel computed it (for checking against the planner). */
 int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32_t time_tile,
                           int32_t space_tile, int64_t* footprint_log, void* stream);
+/* Same result as sp_jacobi1d_timetiled, with every pass in ONE persistent launch: a tile of
+ * pass p+1 starts as soon as the tiles of pass p within reach of its halo are done, so pass
+ * boundaries cost neither a launch nor a partly-filled last round of tiles (H8's inter-tile
+ * synchronisation, done per tile instead of per pass).
+ *   flags[flags_len] : caller-owned device int32 scratch, flags_len >= sp_jacobi1d_plan().tiles + 1;
+ *                      zeroed by the call (stream-ordered): one completion counter per tile and
+ *                      the work counter from which warps take (pass, tile) units in order.
+ * passes x tiles must stay below 2^31 (else SP_ERR_UNSUPPORTED).
+ * Every CTA of the launch must be co-resident (the grid is the occupancy limit); a tile whose
+ * dependences never complete traps after ~20 s instead of hanging.  footprint_log as in
+ * sp_jacobi1d_timetiled ([passes][tiles][2]). */
+int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n, int32_t steps,
+                                int32_t time_tile, int32_t space_tile, int64_t* footprint_log, void* stream);
 
 /* Segment form (building block of the multi-GPU layer and of its single-GPU loopback
  * test): one pass of height h over a window of the global domain.

@@ -129,6 +129,7 @@ SYMBOLS = {
     "sp_jacobi1d_tile_footprint": (ctypes.c_int, [i64, i32, i64, i64, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
     "sp_jacobi1d_timetiled": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, vp, vp]),
     "sp_jacobi1d_pass_segment": (ctypes.c_int, [vp, vp, i64, i64, i64, i64, i64, i32, i32, i32, vp]),
+    "sp_jacobi1d_timetiled_fused": (ctypes.c_int, [vp, vp, vp, i64, i64, i32, i32, i32, vp, vp]),
     "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
     "sp_me_ref_window": (ctypes.c_int, [i32, i32, i32, i32, i32, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
     "sp_get_unique_id": (ctypes.c_int, [ctypes.POINTER(ctypes.c_uint8)]),
@@ -379,6 +380,23 @@ def jacobi1d_timetiled(a, steps: int, time_tile: int = 16, space_tile: int = 0, 
     return a
 
 
+def jacobi1d_timetiled_fused(a, steps: int, time_tile: int = 64, space_tile: int = 0, work=None, flags=None,
+                             footprint_log=None, stream=None):
+    """All passes in one persistent launch (sp_jacobi1d_timetiled_fused).  flags: device int32
+    scratch of >= plan["tiles"] + 1 entries (allocated if None)."""
+    import torch
+    assert a.is_cuda and a.dtype == torch.float32 and a.is_contiguous()
+    if work is None:
+        work = torch.empty_like(a)
+    if flags is None:
+        flags = torch.empty(jacobi1d_plan(a.numel(), steps, time_tile, space_tile)["tiles"] + 1, dtype=torch.int32,
+                            device=a.device)
+    _check(lib.sp_jacobi1d_timetiled_fused(_ptr(a), _ptr(work), _ptr(flags), flags.numel(), a.numel(), int(steps),
+                                           int(time_tile), int(space_tile), _ptr(footprint_log), _stream(stream)),
+           "sp_jacobi1d_timetiled_fused")
+    return a
+
+
 def jacobi1d_untiled(a, steps: int, work=None, stream=None):
     """N1 ablation: no staging, no time tiling (one launch per step).  In place on a[n]."""
     import torch
@@ -412,7 +430,7 @@ def jacobi1d(a_host, steps: int, time_tile: int = 16, space_tile: int = 0, devic
     import torch
     h = torch.from_numpy(np.ascontiguousarray(a_host, dtype=np.float32)) if isinstance(a_host, np.ndarray) else a_host
     d = h.to(device, non_blocking=True)
-    jacobi1d_timetiled(d, steps, time_tile, space_tile)
+    jacobi1d_timetiled_fused(d, steps, time_tile, space_tile)
     out = torch.empty(h.shape, dtype=torch.float32, pin_memory=h.is_pinned())
     out.copy_(d, non_blocking=False)
     return out

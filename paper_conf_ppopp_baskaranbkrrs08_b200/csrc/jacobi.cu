@@ -21,6 +21,7 @@
 #include <cuda_runtime.h>
 
 #include <algorithm>
+#include <climits>
 #include <cstdint>
 #include <cstdlib>
 #include <cstring>
@@ -52,6 +53,10 @@ constexpr int kMaxTimeTile = 128;
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
 constexpr uint64_t kNegZero2 = 0x8000000080000000ull;
 
+#ifdef SP_JAC_DEBUG
+__device__ unsigned long long g_jac_dbg[16];
+#endif
+
 struct PassArgs {
     const float* src;  // src[j] holds global cell g0 + j
     float* dst;        // same indexing
@@ -82,6 +87,16 @@ struct PassArgs {
     // may still be reading in their last pass of that call
     const unsigned long long* done_left;
     const unsigned long long* done_right;
+    // Persistent mode (sp_jacobi1d_timetiled_fused; null otherwise): ONE launch runs every
+    // pass.  Tile index u = pass * tiles + tile; warps take u in increasing order; pass p
+    // reads bufs[p & 1] and writes bufs[(p + 1) & 1] (src/dst/h above are unused).  done[t]
+    // = passes of tile t completed; tile (p, t) starts once done[t-1..t+1] >= p (its halo
+    // sources and the readers of the cells it overwrites; tiles t +- ceil(H/S) when S < H).
+    // A warp publishes a finished tile
+    // before it ever waits on another's, and all warps are resident: no wait cycle.
+    int* done;
+    float* bufs[2];
+    int32_t passes, steps, Tt;
 };
 
 // Spin (acquire, system scope) until *flag >= e.  A peer that never arrives (crashed rank,
@@ -200,9 +215,48 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         lo = x0 - A.H > lo_avail ? x0 - A.H : lo_avail;
         hi = x0 + st + A.H < hi_avail ? x0 + st + A.H : hi_avail;
     };
-    auto issue = [&](int64_t t, int s) {  // lane 0 only
+    const bool pers = A.done != nullptr;
+    const int64_t total = pers ? (int64_t)A.passes * A.tiles : A.tiles;
+    // persistent mode: unit u -> (pass, tile), that pass's buffers and height
+    auto unit = [&](int64_t u, int64_t& t, int& pass) {
+        pass = pers ? (int)(u / A.tiles) : 0;
+        t = pers ? u - (int64_t)pass * A.tiles : u;
+    };
+    auto src_of = [&](int pass) -> const float* { return pers ? A.bufs[pass & 1] : A.src; };
+    auto dst_of = [&](int pass) -> float* { return pers ? A.bufs[(pass + 1) & 1] : A.dst; };
+    auto h_of = [&](int pass) -> int { return pers ? min(A.Tt, A.steps - pass * A.Tt) : A.h; };
+    // tiles within reach of a tile's halo: |q - t| <= ceil(H / S).  The flags are polled with
+    // relaxed L2-coherent loads and the data that depends on them never goes through L1 (TMA
+    // move-in; the ragged tail by ld.global.cg), so no L1 invalidation is needed per poll.
+    const int64_t reach = (A.H + A.S - 1) / A.S;
+    // Warp-uniform (every lane calls it): lane-divergent polling loops would leave the warp
+    // split through the step loop that follows (measured: 1.7x the instructions issued).
+    auto deps_ready = [&](int64_t t, int pass) -> bool {
+        if (!pers || pass == 0) return true;
+        bool ok = true;
+        for (int64_t q0 = t - reach; q0 <= t + reach; q0 += 32) {
+            const int64_t q = q0 + lane;
+            if (q >= 0 && q <= t + reach && q < A.tiles) ok &= ld_relaxed_gpu(A.done + q) >= pass;
+        }
+        return __all_sync(0xffffffffu, ok);
+    };
+    auto wait_deps = [&](int64_t t, int pass) {  // every lane; traps after ~20 s (never expected)
+        const long long t0 = clock64();
+        while (!deps_ready(t, pass)) {
+            __nanosleep(32);
+            if (clock64() - t0 > (40ll << 30)) __trap();
+        }
+#ifdef SP_JAC_DEBUG
+        if (lane == 0) {
+            atomicAdd(&g_jac_dbg[0], 1ull);
+            atomicAdd(&g_jac_dbg[1], (unsigned long long)(clock64() - t0));
+        }
+#endif
+    };
+    auto issue = [&](int64_t t, int pass, int s) {  // lane 0 only
         int64_t x0, st, lo, hi;
         tile_range(t, x0, st, lo, hi);
+        if (pers) fence_proxy_async_global();  // observed flags -> the async-proxy read below
         if (A.wait_left && lo < A.own_begin) {   // halo from the left neighbour (peer store)
             wait_epoch(A.wait_left, A.epoch);
             fence_proxy_async_global();
@@ -213,7 +267,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         }
         const uint32_t bytes = (uint32_t)(((hi - lo) & ~int64_t(3)) * 4);
         mbar_arrive_expect_tx(&bar[s], bytes);
-        if (bytes) tma_load_1d(stage0 + s * kStrip + (lo - (x0 - A.H)), A.src + (lo - A.g0), bytes, &bar[s]);
+        if (bytes) tma_load_1d(stage0 + s * kStrip + (lo - (x0 - A.H)), src_of(pass) + (lo - A.g0), bytes, &bar[s]);
     };
 
     if (blockIdx.x == 0 && warp == 0 && (A.push_left || A.push_right)) {
@@ -238,27 +292,101 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         mbar_init(&bar[0], 1);
         mbar_init(&bar[1], 1);
         fence_mbar_init();
-        if (first < A.tiles) issue(first, 0);
     }
     __syncwarp();
+    // persistent mode: this warp's finished, unpublished tiles (oldest first; at most two).
+    // A tile is published (done flag) once its TMA store has completed — at the next tile's
+    // prefetch point — and always before this warp waits on any other tile.
+    int64_t pub_t[2] = {-1, -1};
+    int pub_pass[2] = {0, 0};
+    bool pending = false;  // warp-uniform: the next tile's move-in waits for its dependences
+    // Unit schedule.  Per-pass launches: static, unit u = first + k * GW.  Persistent mode:
+    // dynamic — each warp takes the next unit from a global counter (flags[tiles]), so units
+    // start in nearly increasing order and a slow warp delays nobody (a static assignment
+    // couples warps through the dependences and drifts: 20 % of tiles then waited).
+    int* const next_unit = pers ? A.done + A.tiles : nullptr;
+    auto grab = [&](int64_t u_static) -> int64_t {  // warp-uniform
+        if (!pers) return u_static;
+        int v = 0;
+        if (lane == 0) v = atomicAdd(next_unit, 1);
+        return (int64_t)__shfl_sync(0xffffffffu, v, 0);
+    };
+    auto unit32 = [&](int64_t u, int64_t& t, int& pass) {  // u < 2^31 (host-checked)
+        pass = pers ? (int)((uint32_t)u / (uint32_t)A.tiles) : 0;
+        t = pers ? u - (int64_t)pass * A.tiles : u;
+    };
+    int64_t u_cur = grab(first);
+    int64_t cur_t;
+    int cur_pass;
+    unit32(u_cur, cur_t, cur_pass);
+    if (u_cur < total) {
+        pending = !deps_ready(cur_t, cur_pass);  // (a first unit beyond pass 0 may have to wait)
+        if (lane == 0 && !pending) issue(cur_t, cur_pass, 0);
+    }
+    __syncwarp();
+    auto publish = [&](bool all) {  // lane 0: the oldest unpublished tile (all: every one)
+        if (pub_t[0] < 0 || (!all && pub_t[1] < 0)) return;
+        if (all) bulk_wait0();
+        else bulk_wait1();            // every store but the newest tile's has completed
+        fence_proxy_async_global();   // async-proxy writes -> generic release below
+        st_release_gpu(A.done + pub_t[0], pub_pass[0] + 1);
+        if (all && pub_t[1] >= 0) st_release_gpu(A.done + pub_t[1], pub_pass[1] + 1);
+        pub_t[0] = all ? -1 : pub_t[1];
+        pub_pass[0] = pub_pass[1];
+        pub_t[1] = -1;
+    };
 
     int it = 0;
-    for (int64_t t = first; t < A.tiles; t += GW, ++it) {
+    for (int64_t u = u_cur; u < total; ++it) {
         const int s = it & 1;
         float* const buf = stage0 + s * kStrip;
         int64_t x0, st, lo, hi;
+        const int64_t t = cur_t;
+        const int pass = cur_pass;
+        const int64_t u_next = grab(u + GW);  // next unit of this warp
+        int64_t tn;
+        int pn;
+        unit32(u_next, tn, pn);
+        cur_t = tn;
+        cur_pass = pn;
+        // the next unit's dependence flags, loaded now and tested at the prefetch below, so
+        // the L2 round trip overlaps this tile's move-in wait and register loads
+        int next_flag = INT_MAX;
+        if (pers && pn > 0 && 2 * reach < 32) {
+            const int64_t q = tn - reach + lane;
+            if (lane <= 2 * reach && q >= 0 && q < A.tiles) next_flag = ld_relaxed_gpu(A.done + q);
+        }
+        const float* const src = src_of(pass);
+        float* const dst = dst_of(pass);
+        const int h = h_of(pass);
         tile_range(t, x0, st, lo, hi);
         const int64_t base = x0 - A.H;  // buf[j] <-> global base + j
+        if (pers && pending) {  // publish first: never wait while holding a finished tile
+            if (lane == 0) publish(true);
+            __syncwarp();
+            wait_deps(t, pass);
+            if (lane == 0) issue(t, pass, s);
+            pending = false;
+            __syncwarp();
+        }
         {
             const int64_t tail0 = lo + ((hi - lo) & ~int64_t(3));
-            if (lane < hi - tail0) buf[tail0 - base + lane] = A.src[tail0 + lane - A.g0];
+            if (lane < hi - tail0) buf[tail0 - base + lane] = __ldcg(src + (tail0 + lane - A.g0));
         }
         if (lane == 0 && A.flog) {
-            A.flog[2 * t] = x0 - A.h > 0 ? x0 - A.h : 0;
-            A.flog[2 * t + 1] = x0 + st - 1 + A.h < A.n - 1 ? x0 + st - 1 + A.h : A.n - 1;
+            int64_t* fl = A.flog + 2 * (pers ? u : t);
+            fl[0] = x0 - h > 0 ? x0 - h : 0;
+            fl[1] = x0 + st - 1 + h < A.n - 1 ? x0 + st - 1 + h : A.n - 1;
         }
+#ifdef SP_JAC_DEBUG
+        const long long tw0 = clock64();
+#endif
         mbar_wait(&bar[s], (it >> 1) & 1);
         __syncwarp();
+#ifdef SP_JAC_DEBUG
+        if (lane == 0 && pass > 0) atomicAdd(&g_jac_dbg[2], (unsigned long long)(clock64() - tw0));
+        if (lane == 0 && pass == 0) atomicAdd(&g_jac_dbg[3], (unsigned long long)(clock64() - tw0));
+#endif
 
         // ---- registers <- staged strip (conflict-free: stride 4K bytes, K/4 odd) ---------
         uint64_t P[kK];
@@ -275,10 +403,24 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             }
         }
         // ---- prefetch the next tile into the other stage once its store has drained ----
-        if (lane == 0 && t + GW < A.tiles) {
-            bulk_wait_read0();
-            issue(t + GW, s ^ 1);
+#ifdef SP_JAC_DEBUG
+        const long long tp0 = clock64();
+#endif
+        if (lane == 0 && pers) publish(true);  // (waiting for the newest store here beats a
+                                                // one-tile publication lag: 6.94 vs 7.01 ms on J3)
+        if (u_next < total) {
+            pending = (pers && pn > 0 && 2 * reach < 32) ? !__all_sync(0xffffffffu, next_flag >= pn) : !deps_ready(tn, pn);
+            if (lane == 0) {
+                bulk_wait_read0();
+                if (!pending) issue(tn, pn, s ^ 1);
+            }
         }
+        __syncwarp();
+#ifdef SP_JAC_DEBUG
+        __syncwarp();
+        const long long tp1 = clock64();
+        if (lane == 0) atomicAdd(&g_jac_dbg[4 + (pass > 0)], (unsigned long long)(tp1 - tp0));
+#endif
         // ---- h steps in registers ---------------------------------------------------
         {
             const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= A.n - 1 && A.n - 1 < base + kStrip);
@@ -294,9 +436,20 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
                 if (A.n - 1 - base < kStrip) vn = buf[A.n - 1 - base];
                 __syncwarp();  // these cells belong to other lanes, which overwrite them below
             }
-            if (boundary) run_steps<true>(P, A.h, lane, w2, A.mz, f0, fn, v0, vn);
-            else run_steps<false>(P, A.h, lane, w2, A.mz, 0ull, 0ull, 0.f, 0.f);
+#ifdef SP_JAC_DEBUG
+            if (lane == 0) {
+                atomicAdd(&g_jac_dbg[10 + (pass > 0)], (unsigned long long)boundary);
+                atomicAdd(&g_jac_dbg[12 + (pass > 0)], (unsigned long long)h);
+            }
+#endif
+            if (boundary) run_steps<true>(P, h, lane, w2, A.mz, f0, fn, v0, vn);
+            else run_steps<false>(P, h, lane, w2, A.mz, 0ull, 0ull, 0.f, 0.f);
         }
+#ifdef SP_JAC_DEBUG
+        __syncwarp();
+        if (lane == 0) atomicAdd(&g_jac_dbg[6 + (pass > 0)], (unsigned long long)(clock64() - tp1));
+        if (lane == 0) atomicAdd(&g_jac_dbg[8 + (pass > 0)], 1ull);
+#endif
         // ---- owned cells -> staged buffer -> TMA bulk store ------------------------------
         {
             const int own_hi = A.H + (int)st;  // strip offsets [H, H + st) are owned
@@ -316,13 +469,24 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         {
             const int64_t n16 = st & ~int64_t(3);
             if (lane == 0 && n16 > 0) {
-                tma_store_1d(A.dst + (x0 - A.g0), buf + A.H, (uint32_t)(n16 * 4));
+                tma_store_1d(dst + (x0 - A.g0), buf + A.H, (uint32_t)(n16 * 4));
                 bulk_commit();
             }
-            if (lane < st - n16) A.dst[x0 - A.g0 + n16 + lane] = buf[A.H + n16 + lane];
+            if (lane < st - n16) dst[x0 - A.g0 + n16 + lane] = buf[A.H + n16 + lane];
         }
+        if (pers) {
+            if (lane < st - (st & ~int64_t(3))) __threadfence();  // the ragged-tail stores above
+            __syncwarp();
+            const int k = pub_t[0] < 0 ? 0 : 1;
+            pub_t[k] = t;
+            pub_pass[k] = pass;
+        }
+        u = u_next;
     }
-    if (lane == 0) bulk_wait0();
+    if (lane == 0) {
+        if (pers) publish(true);
+        bulk_wait0();
+    }
 }
 
 // ---- host side: kernel variants (geometry sweep; SP_JACOBI_VARIANT selects one) ----------
@@ -515,6 +679,44 @@ extern "C" int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t s
         nxt = t;
     }
     if (cur != a) SP_CUDA_TRY(cudaMemcpyAsync(a, cur, (size_t)n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    return SP_OK;
+}
+
+// All passes in ONE persistent launch: tiles of pass p+1 start as soon as the tiles of pass p
+// within reach of their halo are done (per-tile flags in `flags`), so no pass boundary
+// idles the GPU (no launch gap, no partly-filled last round of tiles per pass).
+#ifdef SP_JAC_DEBUG
+extern "C" int sp_jac_dbg_read(unsigned long long* out) {
+    SP_CUDA_TRY(cudaMemcpyFromSymbol(out, g_jac_dbg, sizeof(unsigned long long) * 16));
+    static const unsigned long long z[16] = {};
+    SP_CUDA_TRY(cudaMemcpyToSymbol(g_jac_dbg, z, sizeof(z)));
+    return SP_OK;
+}
+#endif
+
+extern "C" int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n,
+                                           int32_t steps, int32_t time_tile, int32_t space_tile,
+                                           int64_t* footprint_log, void* stream) {
+    if (!a || !work || !flags || n < 3 || steps < 0 || a == work) return SP_ERR_INVALID_ARG;
+    if ((reinterpret_cast<uintptr_t>(a) & 15) || (reinterpret_cast<uintptr_t>(work) & 15)) return SP_ERR_INVALID_ARG;
+    int64_t S;
+    int32_t wo;
+    int st = geometry(time_tile, space_tile, S, wo);
+    if (st) return st;
+    const int64_t tiles = (n + S - 1) / S;
+    if (flags_len < tiles + 1) return SP_ERR_INVALID_ARG;
+    if (steps == 0) return SP_OK;
+    const int32_t passes = (steps + time_tile - 1) / time_tile;
+    if ((int64_t)passes * tiles + (int64_t(1) << 20) > INT32_MAX) return SP_ERR_UNSUPPORTED;  // 32-bit unit counter
+    Variant di;
+    if ((st = device_info(di))) return st;
+    const cudaStream_t s = (cudaStream_t)stream;
+    SP_CUDA_TRY(cudaMemsetAsync(flags, 0, (size_t)(tiles + 1) * sizeof(int32_t), s));
+    PassArgs p{nullptr, nullptr, n, 0, n, 0, n, S, tiles, time_tile, halo_of(time_tile), wo, footprint_log, kNegZero2,
+               nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, 0ull, nullptr, nullptr,
+               flags, {a, work}, passes, steps, time_tile};
+    if ((st = launch_pass(p, s, di))) return st;
+    if (passes & 1) SP_CUDA_TRY(cudaMemcpyAsync(a, work, (size_t)n * sizeof(float), cudaMemcpyDeviceToDevice, s));
     return SP_OK;
 }
 

@@ -30,11 +30,15 @@ def main():
     a0 = torch.from_numpy(sp_inputs.jacobi_input(n)).cuda()
     a = a0.clone()
     w = torch.empty_like(a)
+    flags = torch.empty(n, dtype=torch.int32, device="cuda")
     pos = [x for x in sys.argv[1:] if not x.startswith("--")]
     for tt in ([] if "--me-only" in sys.argv else [int(x) for x in (pos[0].split(",") if pos else ["16", "32"])]):
         def run():
             a.copy_(a0)
-            sp.jacobi1d_timetiled(a, T, tt, 0, work=w)
+            if "--fused" in sys.argv:
+                sp.jacobi1d_timetiled_fused(a, T, tt, 0, work=w, flags=flags)
+            else:
+                sp.jacobi1d_timetiled(a, T, tt, 0, work=w)
         copy_ms, _ = ev_time(lambda: a.copy_(a0))
         best, med = ev_time(run)
         t = best - copy_ms

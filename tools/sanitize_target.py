@@ -18,6 +18,9 @@ mark("sp.jacobi1d_timetiled")
 sp.jacobi1d_timetiled(a, 37, 16, 256)
 mark("sp.jacobi1d_timetiled")
 sp.jacobi1d_timetiled(a, 20, 5, 0)
+mark("sp.jacobi1d_timetiled_fused")
+sp.jacobi1d_timetiled_fused(a, 37, 16, 256)
+sp.jacobi1d_timetiled_fused(a, 20, 5, 8)
 mark("sp.jacobi1d_untiled")
 sp.jacobi1d_untiled(a, 3)
 fr = torch.from_numpy(sp_inputs.me_sequence(3, 352, 288, 16)).cuda()
