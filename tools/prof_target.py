@@ -1,5 +1,5 @@
 """Minimal launch sequence of one kernel at the bench configuration, for ncu captures:
-   python tools/prof_target.py jacobi [Tt]   |   python tools/prof_target.py me"""
+   python tools/prof_target.py jacobi [Tt] | jacobi_fused [Tt] | me"""
 import sys
 
 import torch
@@ -9,7 +9,14 @@ import paper_conf_ppopp_baskaranbkrrs08_b200 as sp  # noqa: E402
 import sp_inputs  # noqa: E402
 
 what = sys.argv[1]
-if what == "jacobi":
+if what == "jacobi_fused":  # the bench's N = 1 launch: all T = 1024 steps in one persistent kernel
+    tt = int(sys.argv[2]) if len(sys.argv) > 2 else 64
+    n = 1 << 26
+    a = torch.from_numpy(sp_inputs.jacobi_input(n)).cuda()
+    w = torch.empty_like(a)
+    for _ in range(2):
+        sp.jacobi1d_timetiled_fused(a, 1024, tt, 0, work=w)
+elif what == "jacobi":
     tt = int(sys.argv[2]) if len(sys.argv) > 2 else 64
     n = 1 << 26
     a = torch.from_numpy(sp_inputs.jacobi_input(n)).cuda()
