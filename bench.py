@@ -381,15 +381,18 @@ def run_ours(args, rank, world, local_rank):
     if world == 1:
         a_pin = torch.from_numpy(sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED)).pin_memory()
         f_pin = torch.from_numpy(frames_host).pin_memory()
+        # host-buffer Jacobi: the kernel reads a_pin and writes the result back over PCIe itself
+        # (sp_jacobi1d_host, wavefront order), in place: every call advances the state T steps
+        jac_host = sp.Jacobi1DHost(n_local, JAC_T, tt)
         for _ in range(1):
-            sp.jacobi1d(a_pin, JAC_T, tt)
+            jac_host.run(a_pin)
             sp.me_search(f_pin, ME_W, ME_H, ME_R)
         torch.cuda.synchronize()
         ke = max(1, min(K, 3))
         tj = tm = 0.0
         for _ in range(ke):
             t0 = time.perf_counter()
-            sp.jacobi1d(a_pin, JAC_T, tt)
+            jac_host.run(a_pin)
             torch.cuda.synchronize()
             t1 = time.perf_counter()
             sp.me_search(f_pin, ME_W, ME_H, ME_R)
@@ -397,9 +400,10 @@ def run_ours(args, rank, world, local_rank):
             t2 = time.perf_counter()
             tj += t1 - t0
             tm += t2 - t1
+        # Jacobi's own bytes: the state read from and written back to pinned host memory
         e2e = {"value": (n_local - 2) * JAC_T * ke / tj / 1e9, "unit": "GPoint-updates/s",
-               "h2d_bytes_per_step": 4 * n_local + frames_host.nbytes,
-               "d2h_bytes_per_step": 4 * n_local + ME_PAIRS * mby * mbx * (4 + 4)}
+               "h2d_bytes_per_step": 4 * n_local, "d2h_bytes_per_step": 4 * n_local,
+               "api": "sp_jacobi1d_host (kernel move-in/out over PCIe, wavefront order)"}
         me_e2e = {"value": me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * ke / tm / 1e9, "unit": "GSAD/s",
                   "h2d_bytes_per_step": frames_host.nbytes, "d2h_bytes_per_step": ME_PAIRS * mby * mbx * 8}
 

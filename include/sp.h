@@ -196,6 +196,37 @@ int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32
 int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n, int32_t steps,
                                 int32_t time_tile, int32_t space_tile, int64_t* footprint_log, void* stream);
 
+/* General form of the persistent launch: out = J^steps(in).
+ *   in, out   : n fp32, 16-byte aligned, device memory OR page-locked host memory
+ *               (cudaHostAlloc / cudaHostRegister; pageable memory -> SP_ERR_INVALID_ARG).
+ *               Pass 0's move-in reads `in` and the last pass's move-out writes `out`
+ *               directly (TMA bulk copies; over PCIe for host memory), so host<->device
+ *               transfer is part of the staged movement, overlapped with the other passes.
+ *               in and out may alias each other and buf0 (not buf1).
+ *   buf0, buf1: device scratch of n fp32 each (distinct), ping-pong between passes.
+ *   skew      : unit order.  0 = pass-major (all tiles of pass p, then pass p+1);
+ *               D > 0 = wavefront: tile t of pass p is scheduled at key t + D p (D a power
+ *               of two exceeding ceil(H/S)), so pass p runs D tiles behind pass p-1 — the passes of a
+ *               band of tiles follow each other while its data is still in L2, and pass 0's
+ *               reads / the last pass's writes stream concurrently with the middle passes;
+ *               < 0 = library default (wavefront, D = the least power of two >= 1024
+ *               exceeding ceil(H/S)).
+ *   flags as for sp_jacobi1d_timetiled_fused; passes x tiles < 2^31.
+ * If out is the array the last pass reads (e.g. passes == 1 and out == in), the last pass
+ * writes buf[passes & 1] and the result is copied to out (stream-ordered). */
+int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float* buf1, int32_t* flags,
+                                 int64_t flags_len, int64_t n, int32_t steps, int32_t time_tile,
+                                 int32_t space_tile, int64_t skew, int64_t* footprint_log, void* stream);
+
+/* End-to-end host-buffer call (the public API behind `e2e`): a_host[n] is PAGE-LOCKED host
+ * memory holding a^(0); on completion (stream-ordered) it holds a^(steps).  The input is
+ * read and the result written by the kernel's own move-in / move-out over PCIe, in the
+ * wavefront order of sp_jacobi1d_timetiled_stream (no separate H2D / D2H copies, no
+ * device copy of the whole array beyond buf0/buf1).  buf0, buf1, flags as above.
+ * Errors: SP_ERR_INVALID_ARG for pageable or misaligned a_host. */
+int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t* flags, int64_t flags_len, int64_t n,
+                     int32_t steps, int32_t time_tile, int32_t space_tile, void* stream);
+
 /* Segment form (building block of the multi-GPU layer and of its single-GPU loopback
  * test): one pass of height h over a window of the global domain.
  *   src/dst : device arrays holding global cells [g0, g0 + len); dst receives the new

@@ -16,6 +16,9 @@ C entry point -> Python name (same names, `sp_` prefix dropped):
   sp_jacobi1d_plan            -> jacobi1d_plan(n, steps, time_tile, space_tile)
   sp_jacobi1d_tile_footprint  -> jacobi1d_tile_footprint(n, h, x0, space_tile)
   sp_jacobi1d_timetiled       -> jacobi1d_timetiled(a, steps, ...)     (device tensor, in place)
+  sp_jacobi1d_timetiled_fused -> jacobi1d_timetiled_fused(a, steps, ...) (one persistent launch)
+  sp_jacobi1d_timetiled_stream -> jacobi1d_timetiled_stream(inp, out, steps, ...) (device or pinned host)
+  sp_jacobi1d_host            -> Jacobi1DHost(n, steps, ...).run(a_pinned)  (the e2e public call)
   sp_jacobi1d_pass_segment    -> jacobi1d_pass_segment(...)
   sp_jacobi1d_timetiled_loopback -> jacobi1d_timetiled_loopback(...)
   sp_jacobi1d_timetiled_dist  -> Comm.jacobi1d_timetiled_dist(...)
@@ -35,7 +38,7 @@ import numpy as np
 __all__ = [
     "SPError", "lib", "plan_buffers", "jacobi1d_plan", "jacobi1d_tile_footprint", "jacobi1d_timetiled",
     "jacobi1d_pass_segment", "jacobi1d_timetiled_loopback", "me_sad_search", "me_ref_window", "me_search_sequence",
-    "jacobi1d", "me_search", "Comm", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
+    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
 ]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
@@ -130,6 +133,8 @@ SYMBOLS = {
     "sp_jacobi1d_timetiled": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, vp, vp]),
     "sp_jacobi1d_pass_segment": (ctypes.c_int, [vp, vp, i64, i64, i64, i64, i64, i32, i32, i32, vp]),
     "sp_jacobi1d_timetiled_fused": (ctypes.c_int, [vp, vp, vp, i64, i64, i32, i32, i32, vp, vp]),
+    "sp_jacobi1d_timetiled_stream": (ctypes.c_int, [vp, vp, vp, vp, vp, i64, i64, i32, i32, i32, i64, vp, vp]),
+    "sp_jacobi1d_host": (ctypes.c_int, [vp, vp, vp, vp, i64, i64, i32, i32, i32, vp]),
     "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
     "sp_me_ref_window": (ctypes.c_int, [i32, i32, i32, i32, i32, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
     "sp_get_unique_id": (ctypes.c_int, [ctypes.POINTER(ctypes.c_uint8)]),
@@ -397,6 +402,49 @@ def jacobi1d_timetiled_fused(a, steps: int, time_tile: int = 64, space_tile: int
     return a
 
 
+def jacobi1d_timetiled_stream(inp, out, steps: int, time_tile: int = 64, space_tile: int = 0, skew: int = -1,
+                              buf0=None, buf1=None, flags=None, footprint_log=None, stream=None):
+    """out = J^steps(inp) in one persistent launch (sp_jacobi1d_timetiled_stream).  inp / out:
+    CUDA or PINNED CPU float32 tensors (host memory is streamed by the kernel's TMA move-in /
+    move-out); skew: 0 pass-major, D > 0 wavefront, < 0 library default."""
+    import torch
+    n = inp.numel()
+    assert inp.dtype == torch.float32 and out.dtype == torch.float32 and out.numel() == n
+    dev = inp.device if inp.is_cuda else (out.device if out.is_cuda else torch.device("cuda"))
+    if buf0 is None:
+        buf0 = torch.empty(n, dtype=torch.float32, device=dev)
+    if buf1 is None:
+        buf1 = torch.empty(n, dtype=torch.float32, device=dev)
+    if flags is None:
+        flags = torch.empty(jacobi1d_plan(n, steps, time_tile, space_tile)["tiles"] + 1, dtype=torch.int32, device=dev)
+    _check(lib.sp_jacobi1d_timetiled_stream(_ptr(inp), _ptr(out), _ptr(buf0), _ptr(buf1), _ptr(flags), flags.numel(), n,
+                                            int(steps), int(time_tile), int(space_tile), int(skew), _ptr(footprint_log),
+                                            _stream(stream)), "sp_jacobi1d_timetiled_stream")
+    return out
+
+
+class Jacobi1DHost:
+    """Reusable device scratch for the end-to-end host-buffer call (sp_jacobi1d_host): two
+    n-cell device buffers and the completion flags, allocated once."""
+
+    def __init__(self, n: int, steps: int, time_tile: int = 64, space_tile: int = 0, device="cuda"):
+        import torch
+        self.n, self.steps, self.time_tile, self.space_tile = n, steps, time_tile, space_tile
+        self.buf0 = torch.empty(n, dtype=torch.float32, device=device)
+        self.buf1 = torch.empty(n, dtype=torch.float32, device=device)
+        self.flags = torch.empty(jacobi1d_plan(n, steps, time_tile, space_tile)["tiles"] + 1, dtype=torch.int32,
+                                 device=device)
+
+    def run(self, a_pinned, stream=None):
+        """In place on a PINNED CPU float32 tensor: a_pinned <- J^steps(a_pinned) (stream-ordered;
+        synchronize before reading it)."""
+        assert a_pinned.is_pinned() and a_pinned.numel() == self.n and a_pinned.is_contiguous()
+        _check(lib.sp_jacobi1d_host(_ptr(a_pinned), _ptr(self.buf0), _ptr(self.buf1), _ptr(self.flags),
+                                    self.flags.numel(), self.n, int(self.steps), int(self.time_tile),
+                                    int(self.space_tile), _stream(stream)), "sp_jacobi1d_host")
+        return a_pinned
+
+
 def jacobi1d_untiled(a, steps: int, work=None, stream=None):
     """N1 ablation: no staging, no time tiling (one launch per step).  In place on a[n]."""
     import torch
@@ -424,15 +472,15 @@ def jacobi1d_timetiled_loopback(a_locals, work_locals, n_global: int, x_begins, 
                                               int(space_tile), _stream(stream)), "sp_jacobi1d_timetiled_loopback")
 
 
-def jacobi1d(a_host, steps: int, time_tile: int = 16, space_tile: int = 0, device="cuda"):
-    """End-to-end public call on a host array: H2D copy, time-tiled run, D2H copy.
-    Accepts a numpy array or a (preferably pinned) CPU torch tensor; returns a CPU tensor."""
+def jacobi1d(a_host, steps: int, time_tile: int = 64, space_tile: int = 0, device="cuda"):
+    """End-to-end public call on a host array (numpy or CPU tensor): returns J^steps(a_host) as
+    a pinned CPU tensor.  The input is copied into page-locked memory if it is not already
+    there; the kernel then reads it and writes the result over PCIe itself (sp_jacobi1d_host)."""
     import torch
     h = torch.from_numpy(np.ascontiguousarray(a_host, dtype=np.float32)) if isinstance(a_host, np.ndarray) else a_host
-    d = h.to(device, non_blocking=True)
-    jacobi1d_timetiled_fused(d, steps, time_tile, space_tile)
-    out = torch.empty(h.shape, dtype=torch.float32, pin_memory=h.is_pinned())
-    out.copy_(d, non_blocking=False)
+    out = h.contiguous().pin_memory() if not h.is_pinned() else h.clone().pin_memory()
+    Jacobi1DHost(out.numel(), steps, time_tile, space_tile, device).run(out)
+    torch.cuda.synchronize(device)
     return out
 
 

@@ -39,15 +39,18 @@ using namespace sp::ptx;
 // accesses at stride 4K bytes bank-conflict free), WARPS warps per CTA, MINB CTAs per SM
 // for the register budget.  A warp strip is 64K cells; a shared-memory stage holds
 // WARPS strips.
-template <int K_, int WARPS_, int MINB_>
+// SE_ selects the step with scalar edge cells (run_steps_se: no packing moves on the FMA
+// pipe, any K); the packed-edge step (run_steps) needs K <= 32 for its boundary bit masks.
+template <int K_, int WARPS_, int MINB_, bool SE_ = false>
 struct JCfg {
     static constexpr int K = K_;
     static constexpr int kWarps = WARPS_;
     static constexpr int kMinBlocks = MINB_;
+    static constexpr bool kScalarEdges = SE_;
     static constexpr int kThreads = 32 * WARPS_;
     static constexpr int kStrip = 64 * K_;
     static constexpr int kStage = WARPS_ * 2 * 64 * K_;  // floats of shared memory per CTA
-    static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && K_ <= 32, "K/4 must be odd, K <= 32");
+    static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && (SE_ || K_ <= 32), "K/4 must be odd, K <= 32 unless scalar edges");
 };
 constexpr int kMaxTimeTile = 128;
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
@@ -97,6 +100,15 @@ struct PassArgs {
     int* done;
     float* bufs[2];
     int32_t passes, steps, Tt;
+    // Pass 0 reads in0 instead of bufs[0] and the last pass writes outL instead of its
+    // bufs entry (device or mapped pinned host memory: the move-in / move-out TMA copies then
+    // stream over PCIe).  Unit order: skew == 0 -> pass-major (u = pass * tiles + tile);
+    // skew = D (a power of two > reach) -> wavefront: units sorted by key k = tile + D * pass,
+    // then pass, so pass p runs D tiles behind pass p-1 and a tile's dependences are always
+    // earlier units (keys <= k - D + reach < k).
+    const float* in0;
+    float* outL;
+    int64_t skew;
 };
 
 // Spin (acquire, system scope) until *flag >= e.  A peer that never arrives (crashed rank,
@@ -183,6 +195,90 @@ __device__ __forceinline__ void run_steps(uint64_t (&P)[kK], int h, int lane, ui
     }
 }
 
+// ---- scalar-edge variant ----------------------------------------------------------------
+// fl(x * w) rounded once, as fma(x, w, -0) with the -0 addend opaque (see f2_mul_nofuse):
+// FFMA with an immediate w issues at full rate.
+__device__ __forceinline__ float mul_w(float x, float mz) {
+    float d;
+    asm("fma.rn.f32 %0, %1, 0f3EAAAAAB, %2;" : "=f"(d) : "f"(x), "f"(mz));
+    return d;
+}
+__device__ __forceinline__ float add_rn(float a, float b) {
+    float d;
+    asm("add.rn.f32 %0, %1, %2;" : "=f"(d) : "f"(a), "f"(b));
+    return d;
+}
+__device__ __forceinline__ float upd1(float l, float c, float r, float mz) { return mul_w(add_rn(add_rn(l, c), r), mz); }
+
+// Lane neighbours from the new edge cells (scalars: no packing moves).
+__device__ __forceinline__ void neighbours_ip(float e0u, float e0v, float eNu, float eNv, int lane, float& lu, float& lv,
+                                              float& ru, float& rv) {
+    const float a = __shfl_sync(0xffffffffu, eNu, (lane + 31) & 31);  // lane-1's last u
+    const float b = __shfl_sync(0xffffffffu, eNv, (lane + 31) & 31);  // lane-1's last v
+    const float c = __shfl_sync(0xffffffffu, e0u, (lane + 1) & 31);   // lane+1's first u
+    const float d = __shfl_sync(0xffffffffu, e0v, (lane + 1) & 31);   // lane+1's first v
+    lu = a;
+    lv = lane == 0 ? a : b;
+    ru = lane == 31 ? d : c;
+    rv = d;
+}
+
+// Ping-pong form of the same step (P -> Q, two register arrays), scalar edge cells.
+template <bool kBoundary, int kK>
+__device__ __forceinline__ void step_pp(const uint64_t (&P)[kK], uint64_t (&Q)[kK], float& lu, float& lv, float& ru,
+                                        float& rv, int lane, uint64_t w2, uint64_t mz2, float mz, int ju0, int jv0,
+                                        int jun, int jvn, float v0, float vn) {
+    float e0u = upd1(lu, f2_lo(P[0]), f2_lo(P[1]), mz);
+    float e0v = upd1(lv, f2_hi(P[0]), f2_hi(P[1]), mz);
+    float eNu = upd1(f2_lo(P[kK - 2]), f2_lo(P[kK - 1]), ru, mz);
+    float eNv = upd1(f2_hi(P[kK - 2]), f2_hi(P[kK - 1]), rv, mz);
+    if (kBoundary) {
+        if (ju0 == 0) e0u = v0;
+        if (jun == 0) e0u = vn;
+        if (jv0 == 0) e0v = v0;
+        if (jvn == 0) e0v = vn;
+        if (ju0 == kK - 1) eNu = v0;
+        if (jun == kK - 1) eNu = vn;
+        if (jv0 == kK - 1) eNv = v0;
+        if (jvn == kK - 1) eNv = vn;
+    }
+    neighbours_ip(e0u, e0v, eNu, eNv, lane, lu, lv, ru, rv);
+    Q[0] = f2_pack(e0u, e0v);
+    Q[kK - 1] = f2_pack(eNu, eNv);
+#pragma unroll
+    for (int j = 1; j < kK - 1; ++j) {
+        Q[j] = f2_mul_nofuse(f2_add(f2_add(P[j - 1], P[j]), P[j + 1]), w2, mz2);
+        if (kBoundary) {
+            float u = f2_lo(Q[j]), v = f2_hi(Q[j]);
+            if (ju0 == j) u = v0;
+            if (jun == j) u = vn;
+            if (jv0 == j) v = v0;
+            if (jvn == j) v = vn;
+            Q[j] = f2_pack(u, v);
+        }
+    }
+}
+
+// h steps, ping-ponging between P and Q (two steps per iteration), scalar edge cells.
+template <bool kBoundary, int kK>
+__device__ __forceinline__ void run_steps_se(uint64_t (&P)[kK], int h, int lane, uint64_t w2, uint64_t mz2, int ju0,
+                                             int jv0, int jun, int jvn, float v0, float vn) {
+    const float mz = f2_lo(mz2);
+    float lu, lv, ru, rv;
+    neighbours_ip(f2_lo(P[0]), f2_hi(P[0]), f2_lo(P[kK - 1]), f2_hi(P[kK - 1]), lane, lu, lv, ru, rv);
+    uint64_t Q[kK];
+    int k = 0;
+    for (; k + 2 <= h; k += 2) {
+        step_pp<kBoundary>(P, Q, lu, lv, ru, rv, lane, w2, mz2, mz, ju0, jv0, jun, jvn, v0, vn);
+        step_pp<kBoundary>(Q, P, lu, lv, ru, rv, lane, w2, mz2, mz, ju0, jv0, jun, jvn, v0, vn);
+    }
+    if (k < h) {
+        step_pp<kBoundary>(P, Q, lu, lv, ru, rv, lane, w2, mz2, mz, ju0, jv0, jun, jvn, v0, vn);
+#pragma unroll
+        for (int j = 0; j < kK; ++j) P[j] = Q[j];
+    }
+}
+
 // One launch = one time tile (pass).  Every WARP is an independent outer-level process
 // (processes on one multiprocessor divide its scratchpad): it owns a sequence of
 // space tiles of S cells, each staged as the warp strip [x0 - H, x0 - H + 64K) in the warp's
@@ -216,14 +312,15 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         hi = x0 + st + A.H < hi_avail ? x0 + st + A.H : hi_avail;
     };
     const bool pers = A.done != nullptr;
+    const int64_t keys = A.tiles + A.skew * (A.passes - 1);
     const int64_t total = pers ? (int64_t)A.passes * A.tiles : A.tiles;
-    // persistent mode: unit u -> (pass, tile), that pass's buffers and height
-    auto unit = [&](int64_t u, int64_t& t, int& pass) {
-        pass = pers ? (int)(u / A.tiles) : 0;
-        t = pers ? u - (int64_t)pass * A.tiles : u;
+    // persistent mode: that pass's buffers and height
+    auto src_of = [&](int pass) -> const float* {
+        return pers ? (pass == 0 && A.in0 ? A.in0 : A.bufs[pass & 1]) : A.src;
     };
-    auto src_of = [&](int pass) -> const float* { return pers ? A.bufs[pass & 1] : A.src; };
-    auto dst_of = [&](int pass) -> float* { return pers ? A.bufs[(pass + 1) & 1] : A.dst; };
+    auto dst_of = [&](int pass) -> float* {
+        return pers ? (pass == A.passes - 1 && A.outL ? A.outL : A.bufs[(pass + 1) & 1]) : A.dst;
+    };
     auto h_of = [&](int pass) -> int { return pers ? min(A.Tt, A.steps - pass * A.Tt) : A.h; };
     // tiles within reach of a tile's halo: |q - t| <= ceil(H / S).  The flags are polled with
     // relaxed L2-coherent loads and the data that depends on them never goes through L1 (TMA
@@ -305,15 +402,43 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     // start in nearly increasing order and a slow warp delays nobody (a static assignment
     // couples warps through the dependences and drifts: 20 % of tiles then waited).
     int* const next_unit = pers ? A.done + A.tiles : nullptr;
+    // wavefront order (skew D = 2^lg): unit index -> (key k, pass).  cnt(k) = units with key
+    // < k = sum_p clamp(k - D p, 0, tiles) in closed form; the key of unit u is the largest k
+    // with cnt(k) <= u, found by a 32-ary search (every lane evaluates one candidate).
+    const int lg = A.skew ? __ffsll(A.skew) - 1 : 0;
+    auto cnt = [&](int64_t k) -> int64_t {
+        if (k <= 0) return 0;
+        const int64_t m = min((int64_t)A.passes, (k + A.skew - 1) >> lg);  // passes with D p < k
+        const int64_t q = k >= A.tiles ? min(m, ((k - A.tiles) >> lg) + 1) : 0;  // ... and k - D p >= tiles
+        return q * A.tiles + (m - q) * k - (((m - q) * (m + q - 1) / 2) << lg);
+    };
+    auto unit32 = [&](int64_t u, int64_t& t, int& pass) {  // warp-uniform; u < 2^31 (host-checked)
+        if (!pers) {
+            pass = 0;
+            t = u;
+        } else if (A.skew) {
+            int64_t lo = 0, span = keys;  // answer in [lo, lo + span)
+            while (span > 1) {
+                const int64_t step = (span + 31) >> 5;
+                const int64_t c = lo + lane * step;
+                const unsigned okm = __ballot_sync(0xffffffffu, c < lo + span && cnt(c) <= u);
+                const int64_t nlo = lo + (int64_t)(31 - __clz(okm)) * step;
+                span = min(step, lo + span - nlo);
+                lo = nlo;
+            }
+            const int64_t p_lo = lo >= A.tiles ? ((lo - A.tiles) >> lg) + 1 : 0;
+            pass = (int)(p_lo + (u - cnt(lo)));
+            t = lo - ((int64_t)pass << lg);
+        } else {
+            pass = (int)((uint32_t)u / (uint32_t)A.tiles);
+            t = u - (int64_t)pass * A.tiles;
+        }
+    };
     auto grab = [&](int64_t u_static) -> int64_t {  // warp-uniform
         if (!pers) return u_static;
         int v = 0;
         if (lane == 0) v = atomicAdd(next_unit, 1);
         return (int64_t)__shfl_sync(0xffffffffu, v, 0);
-    };
-    auto unit32 = [&](int64_t u, int64_t& t, int& pass) {  // u < 2^31 (host-checked)
-        pass = pers ? (int)((uint32_t)u / (uint32_t)A.tiles) : 0;
-        t = pers ? u - (int64_t)pass * A.tiles : u;
     };
     int64_t u_cur = grab(first);
     int64_t cur_t;
@@ -374,7 +499,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             if (lane < hi - tail0) buf[tail0 - base + lane] = __ldcg(src + (tail0 + lane - A.g0));
         }
         if (lane == 0 && A.flog) {
-            int64_t* fl = A.flog + 2 * (pers ? u : t);
+            int64_t* fl = A.flog + 2 * (pers ? (int64_t)pass * A.tiles + t : t);
             fl[0] = x0 - h > 0 ? x0 - h : 0;
             fl[1] = x0 + st - 1 + h < A.n - 1 ? x0 + st - 1 + h : A.n - 1;
         }
@@ -424,6 +549,24 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         // ---- h steps in registers ---------------------------------------------------
         {
             const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= A.n - 1 && A.n - 1 < base + kStrip);
+            if constexpr (Cfg::kScalarEdges) {
+                // pair index holding global cell 0 / n-1 in this lane's u / v range (-1: none)
+                int ju0 = -1, jv0 = -1, jun = -1, jvn = -1;
+                float v0 = 0.f, vn = 0.f;
+                if (boundary) {
+                    const int64_t cu = base + lane * kK, cv = base + 32 * kK + lane * kK;
+                    if (cu <= 0 && 0 < cu + kK) ju0 = (int)(0 - cu);
+                    if (cv <= 0 && 0 < cv + kK) jv0 = (int)(0 - cv);
+                    if (cu <= A.n - 1 && A.n - 1 < cu + kK) jun = (int)(A.n - 1 - cu);
+                    if (cv <= A.n - 1 && A.n - 1 < cv + kK) jvn = (int)(A.n - 1 - cv);
+                    if (0 >= base) v0 = buf[0 - base];
+                    if (A.n - 1 - base < kStrip) vn = buf[A.n - 1 - base];
+                    __syncwarp();
+                    run_steps_se<true>(P, h, lane, w2, A.mz, ju0, jv0, jun, jvn, v0, vn);
+                } else {
+                    run_steps_se<false>(P, h, lane, w2, A.mz, -1, -1, -1, -1, 0.f, 0.f);
+                }
+            } else {
             uint64_t f0 = 0, fn = 0;
             float v0 = 0.f, vn = 0.f;
             if (boundary) {
@@ -444,6 +587,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 #endif
             if (boundary) run_steps<true>(P, h, lane, w2, A.mz, f0, fn, v0, vn);
             else run_steps<false>(P, h, lane, w2, A.mz, 0ull, 0ull, 0.f, 0.f);
+            }
         }
 #ifdef SP_JAC_DEBUG
         __syncwarp();
@@ -509,8 +653,9 @@ Variant make_variant() {
     return v;
 }
 
-constexpr int kNumVariants = 6;
+constexpr int kNumVariants = 11;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
+constexpr int64_t kDefaultSkew = 1024;  // wavefront order: tiles between consecutive passes (host path sweep: 256 -> 9.6 ms, 1024 -> 8.9, 2048 -> 10.3 on J3)
 
 Variant* variants() {
     static Variant v[kNumVariants] = {
@@ -520,6 +665,11 @@ Variant* variants() {
         make_variant<JCfg<28, 4, 4>>(),  // 3: 56 cells/lane, <= 128 regs
         make_variant<JCfg<20, 2, 8>>(),  // 4: 40 cells/lane, 2 warps/CTA, <= 128 regs
         make_variant<JCfg<28, 8, 2>>(),  // 5: 56 cells/lane, 8 warps/CTA (224 KB of stages per SM)
+        make_variant<JCfg<28, 8, 2, true>>(),  // 6: as 5, scalar edge cells
+        make_variant<JCfg<52, 8, 1, true>>(),  // 7: 104 cells/lane, scalar edges, 8 warps/SM (208 KB of stages)
+        make_variant<JCfg<44, 8, 1, true>>(),  // 8: 88 cells/lane, scalar edges, 8 warps/SM
+        make_variant<JCfg<36, 12, 1, true>>(),  // 9: 72 cells/lane, scalar edges, 12 warps/SM (216 KB)
+        make_variant<JCfg<44, 4, 2, true>>(),  // 10: as 8 as two 4-warp CTAs per SM
     };
     return v;
 }
@@ -694,30 +844,94 @@ extern "C" int sp_jac_dbg_read(unsigned long long* out) {
 }
 #endif
 
-extern "C" int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n,
-                                           int32_t steps, int32_t time_tile, int32_t space_tile,
-                                           int64_t* footprint_log, void* stream) {
-    if (!a || !work || !flags || n < 3 || steps < 0 || a == work) return SP_ERR_INVALID_ARG;
-    if ((reinterpret_cast<uintptr_t>(a) & 15) || (reinterpret_cast<uintptr_t>(work) & 15)) return SP_ERR_INVALID_ARG;
+namespace {
+// A pointer the kernel can dereference: device memory as is, page-locked host memory through
+// its device mapping (UVA: usually the same address).  Pageable host memory is rejected.
+int device_view(const void* p, const void** out) {
+    cudaPointerAttributes at;
+    SP_CUDA_TRY(cudaPointerGetAttributes(&at, p));
+    if (at.type == cudaMemoryTypeDevice || at.type == cudaMemoryTypeManaged) {
+        *out = p;
+        return SP_OK;
+    }
+    if (at.type == cudaMemoryTypeHost) {
+        void* d = nullptr;
+        SP_CUDA_TRY(cudaHostGetDevicePointer(&d, const_cast<void*>(p), 0));
+        *out = d;
+        return SP_OK;
+    }
+    return SP_ERR_INVALID_ARG;
+}
+}  // namespace
+
+extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float* buf1, int32_t* flags,
+                                            int64_t flags_len, int64_t n, int32_t steps, int32_t time_tile,
+                                            int32_t space_tile, int64_t skew, int64_t* footprint_log, void* stream) {
+    if (!in || !out || !buf0 || !buf1 || !flags || n < 3 || steps < 0 || buf0 == buf1 || in == buf1)
+        return SP_ERR_INVALID_ARG;
+    for (const void* q : {(const void*)in, (const void*)out, (const void*)buf0, (const void*)buf1})
+        if (reinterpret_cast<uintptr_t>(q) & 15) return SP_ERR_INVALID_ARG;
     int64_t S;
     int32_t wo;
     int st = geometry(time_tile, space_tile, S, wo);
     if (st) return st;
     const int64_t tiles = (n + S - 1) / S;
     if (flags_len < tiles + 1) return SP_ERR_INVALID_ARG;
-    if (steps == 0) return SP_OK;
+    const cudaStream_t s = (cudaStream_t)stream;
+    const float *din = nullptr, *dout = nullptr;
+    if ((st = device_view(in, (const void**)&din)) || (st = device_view(out, (const void**)&dout))) return st;
+    if (steps == 0) {
+        if (out != in) SP_CUDA_TRY(cudaMemcpyAsync(out, in, (size_t)n * sizeof(float), cudaMemcpyDefault, s));
+        return SP_OK;
+    }
     const int32_t passes = (steps + time_tile - 1) / time_tile;
-    if ((int64_t)passes * tiles + (int64_t(1) << 20) > INT32_MAX) return SP_ERR_UNSUPPORTED;  // 32-bit unit counter
+    const int32_t H = halo_of(time_tile);
+    const int64_t reach = (H + S - 1) / S;
+    if (skew < 0) {
+        static const int64_t dflt = [] {  // SP_JACOBI_SKEW overrides the default (sweeps)
+            const char* e = std::getenv("SP_JACOBI_SKEW");
+            const long long v = e ? std::atoll(e) : 0;
+            return v > 0 ? (int64_t)v : kDefaultSkew;
+        }();
+        skew = dflt;
+        while (skew <= reach) skew <<= 1;
+    }
+    if (skew > 0 && (skew <= reach || (skew & (skew - 1)))) return SP_ERR_INVALID_ARG;
+    if ((int64_t)passes * tiles + (int64_t(1) << 20) > INT32_MAX || tiles + skew * (passes - 1) > INT32_MAX)
+        return SP_ERR_UNSUPPORTED;  // 32-bit unit counter
     Variant di;
     if ((st = device_info(di))) return st;
-    const cudaStream_t s = (cudaStream_t)stream;
+    float* bufs[2] = {buf0, buf1};
+    // the last pass must not write the array it reads: then it writes bufs[passes & 1] and the
+    // result is copied to out afterwards
+    const float* last_src = passes == 1 ? din : bufs[(passes - 1) & 1];
+    const bool redirect = dout == last_src;
     SP_CUDA_TRY(cudaMemsetAsync(flags, 0, (size_t)(tiles + 1) * sizeof(int32_t), s));
-    PassArgs p{nullptr, nullptr, n, 0, n, 0, n, S, tiles, time_tile, halo_of(time_tile), wo, footprint_log, kNegZero2,
+    PassArgs p{nullptr, nullptr, n, 0, n, 0, n, S, tiles, time_tile, H, wo, footprint_log, kNegZero2,
                nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, 0ull, nullptr, nullptr,
-               flags, {a, work}, passes, steps, time_tile};
+               flags, {buf0, buf1}, passes, steps, time_tile, din, redirect ? nullptr : const_cast<float*>(dout), skew};
     if ((st = launch_pass(p, s, di))) return st;
-    if (passes & 1) SP_CUDA_TRY(cudaMemcpyAsync(a, work, (size_t)n * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    if (redirect)
+        SP_CUDA_TRY(cudaMemcpyAsync(out, bufs[passes & 1], (size_t)n * sizeof(float), cudaMemcpyDefault, s));
     return SP_OK;
+}
+
+extern "C" int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n,
+                                           int32_t steps, int32_t time_tile, int32_t space_tile,
+                                           int64_t* footprint_log, void* stream) {
+    if (!a || !work || a == work) return SP_ERR_INVALID_ARG;
+    return sp_jacobi1d_timetiled_stream(a, a, a, work, flags, flags_len, n, steps, time_tile, space_tile, 0,
+                                        footprint_log, stream);
+}
+
+extern "C" int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t* flags, int64_t flags_len, int64_t n,
+                                int32_t steps, int32_t time_tile, int32_t space_tile, void* stream) {
+    if (!a_host) return SP_ERR_INVALID_ARG;
+    cudaPointerAttributes at;
+    SP_CUDA_TRY(cudaPointerGetAttributes(&at, a_host));
+    if (at.type != cudaMemoryTypeHost) return SP_ERR_INVALID_ARG;  // page-locked host memory only
+    return sp_jacobi1d_timetiled_stream(a_host, a_host, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile,
+                                        -1, nullptr, stream);
 }
 
 __global__ void peer_done_kernel(unsigned long long* left_done, unsigned long long* right_done, unsigned long long e) {
