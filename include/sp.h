@@ -263,6 +263,23 @@ int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int3
                      int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
                      int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream);
 
+/* End-to-end host-buffer search of a frame sequence (the public API behind the ME `e2e`):
+ * pairs p = (ref = frame p, cur = frame p+1), p < n_frames - 1, exactly as sp_me_sad_search
+ * over the whole frame.
+ *   frames_host : PAGE-LOCKED host memory [n_frames][height][pitch] uint8 (pitch multiple of 16)
+ *   frames_dev  : device buffer of the same size (staging; contents overwritten)
+ *   ready       : device int32 [n_frames - 1] (scratch; cleared by the call)
+ *   mv, best_sad: outputs as in sp_me_sad_search for mb rows [0, height/16), in device memory
+ *                 or PAGE-LOCKED host memory (the kernel then stores them over PCIe itself)
+ *   copy_stream : stream for the H2D frame copies (nullable: a library-owned stream)
+ * The frames are copied frame by frame on copy_stream, each copy followed by a copy-engine write
+ * of ready[f-1] = 1; the search on `stream` starts at once and the move-in of every macroblock
+ * waits for its pair's flag, so the transfer overlaps the search.  `stream` completes after
+ * both the search and the copies.  range must be 16 or 32 (SP_ERR_UNSUPPORTED otherwise). */
+int sp_me_search_host(const uint8_t* frames_host, int64_t pitch, int32_t width, int32_t height, int32_t n_frames,
+                      int32_t range, uint8_t* frames_dev, int32_t* ready, int16_t* mv, uint32_t* best_sad,
+                      void* stream, void* copy_stream);
+
 /* Unrestricted motion vectors (reading R-M7): candidates may point
  * outside the frame; out-of-frame reference pixels take the value of the nearest frame pixel
  * (edge extension, as in MPEG-4 / H.264 unrestricted MVs), so all (2R+1)^2 candidates are

@@ -24,6 +24,7 @@ C entry point -> Python name (same names, `sp_` prefix dropped):
   sp_jacobi1d_timetiled_dist  -> Comm.jacobi1d_timetiled_dist(...)
   sp_me_sad_search            -> me_sad_search(ref, cur, ...)          (device tensors)
   sp_me_ref_window            -> me_ref_window(...)
+  sp_me_search_host           -> MESearchHost(F, W, H, pitch, R).run(frames_pinned)  (the e2e public call)
   sp_get_unique_id / sp_comm_init / sp_comm_destroy / sp_allgather -> Comm
 Host-buffer convenience (the end-to-end public API used for bench.py's `e2e`):
   jacobi1d(host_array, steps, ...), me_search(host_frames, ...)
@@ -38,7 +39,7 @@ import numpy as np
 __all__ = [
     "SPError", "lib", "plan_buffers", "jacobi1d_plan", "jacobi1d_tile_footprint", "jacobi1d_timetiled",
     "jacobi1d_pass_segment", "jacobi1d_timetiled_loopback", "me_sad_search", "me_ref_window", "me_search_sequence",
-    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
+    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
 ]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
@@ -136,6 +137,7 @@ SYMBOLS = {
     "sp_jacobi1d_timetiled_stream": (ctypes.c_int, [vp, vp, vp, vp, vp, i64, i64, i32, i32, i32, i64, vp, vp]),
     "sp_jacobi1d_host": (ctypes.c_int, [vp, vp, vp, vp, i64, i64, i32, i32, i32, vp]),
     "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
+    "sp_me_search_host": (ctypes.c_int, [vp, i64, i32, i32, i32, i32, vp, vp, vp, vp, vp, vp]),
     "sp_me_ref_window": (ctypes.c_int, [i32, i32, i32, i32, i32, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
     "sp_get_unique_id": (ctypes.c_int, [ctypes.POINTER(ctypes.c_uint8)]),
     "sp_comm_init": (ctypes.c_int, [ctypes.POINTER(vp), ctypes.POINTER(ctypes.c_uint8), i32, i32, i32]),
@@ -587,14 +589,44 @@ def me_search_sequence(frames, width: int, frame_height: int, search_range: int,
     return me_sad_search(frames[:-1], frames[1:], width, frame_height, search_range, **kw)
 
 
+class MESearchHost:
+    """Reusable device staging for the end-to-end host-buffer search (sp_me_search_host): the
+    frame buffer and ready flags on the device, the outputs in pinned host memory (the kernel
+    stores them over PCIe), and a copy stream — allocated once."""
+
+    def __init__(self, n_frames: int, width: int, height: int, pitch: int, search_range: int, device="cuda"):
+        import torch
+        self.n_frames, self.width, self.height, self.pitch, self.range = n_frames, width, height, pitch, search_range
+        self.frames_dev = torch.empty((n_frames, height, pitch), dtype=torch.uint8, device=device)
+        self.ready = torch.empty(max(1, n_frames - 1), dtype=torch.int32, device=device)
+        mbx, mby = width // 16, height // 16
+        self.mv = torch.empty((max(0, n_frames - 1), mby, mbx, 2), dtype=torch.int16).pin_memory()
+        self.sad = torch.empty((max(0, n_frames - 1), mby, mbx), dtype=torch.int32).pin_memory()
+        self.copy_stream = torch.cuda.Stream(device=device)
+
+    def run(self, frames_pinned, stream=None):
+        """frames_pinned: PINNED uint8 tensor [n_frames, height, pitch]; returns (mv, sad) pinned
+        CPU tensors, valid after the stream synchronizes."""
+        assert frames_pinned.is_pinned() and tuple(frames_pinned.shape) == (self.n_frames, self.height, self.pitch)
+        _check(lib.sp_me_search_host(_ptr(frames_pinned), self.pitch, self.width, self.height, self.n_frames,
+                                     self.range, _ptr(self.frames_dev), _ptr(self.ready), _ptr(self.mv), _ptr(self.sad),
+                                     _stream(stream), _stream(self.copy_stream)), "sp_me_search_host")
+        return self.mv, self.sad
+
+
 def me_search(frames_host, width: int, frame_height: int, search_range: int, device="cuda"):
-    """End-to-end public call on a host frame sequence [F, H, pitch] (numpy or pinned
-    tensor): H2D copy, search of the F-1 consecutive pairs, D2H copy of MV and SAD."""
+    """End-to-end public call on a host frame sequence [F, H, pitch] (numpy or CPU tensor):
+    frame-by-frame H2D copies overlapped with the search (sp_me_search_host; R in {16, 32}),
+    MV / SAD stored into pinned host memory by the kernel.  Returns (mv, sad) CPU tensors."""
     import torch
     h = torch.from_numpy(np.ascontiguousarray(frames_host)) if isinstance(frames_host, np.ndarray) else frames_host
-    d = h.to(device, non_blocking=True)
-    mv, sad, _ = me_search_sequence(d, width, frame_height, search_range)
-    return mv.cpu(), sad.cpu()
+    if not h.is_pinned():
+        h = h.contiguous().pin_memory()
+    F, H, pitch = h.shape
+    ctx = MESearchHost(F, width, frame_height, pitch, search_range, device)
+    mv, sad = ctx.run(h)
+    torch.cuda.synchronize(device)
+    return mv, sad
 
 
 # ---------------------------------------------------------------------------------------

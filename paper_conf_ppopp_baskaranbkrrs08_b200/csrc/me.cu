@@ -66,6 +66,10 @@ struct MeArgs {
     int16_t* mv;
     uint32_t* sad;
     uint32_t* surface;
+    // nullable: ready[pair] != 0 once both frames of the pair are resident (written by the
+    // stream-ordered H2D copies of sp_me_search_host, concurrently with the search); the
+    // move-in of a macroblock waits for its pair's flag
+    const int32_t* ready;
 };
 
 __device__ __forceinline__ uint64_t make_key(uint32_t s, int dx, int dy, int R) {
@@ -162,6 +166,16 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     };
     auto issue = [&](uint32_t mb, int st) {  // single thread: stage the window + cur of mb
         const Pos q = locate(mb);
+        if (A.ready) {  // frames still streaming in: wait for this pair's (relaxed poll, then a
+                        // proxy fence orders the observed copy before the TMA reads below)
+            const long long t0 = clock64();
+            while (ld_relaxed_gpu(A.ready + q.pair) == 0) {
+                __nanosleep(256);
+                if (clock64() - t0 > (40ll << 30)) __trap();
+            }
+            (void)ld_acquire_gpu(A.ready + q.pair);  // (flags only go 0 -> 1)
+            fence_proxy_async_global();
+        }
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         mbar_arrive_expect_tx(&full[st], (uint32_t)(G::kCopy + kMB * kMB));
         tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair, &full[st]);
@@ -181,8 +195,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const uint32_t sad = b / kKeyMul, tie = b - sad * kKeyMul;
         const int dy = (int)((tie >> 1) & 127) - R;
         const int adx = (int)((tie >> 8) & 127) - abs(dy);
-        A.mv[2 * idx] = (int16_t)((tie & 1) ? adx : -adx);
-        A.mv[2 * idx + 1] = (int16_t)dy;
+        // (dx, dy) as one 32-bit store (the outputs may be mapped host memory: fewer PCIe writes)
+        *reinterpret_cast<uint32_t*>(A.mv + 2 * idx) = (uint32_t)(uint16_t)((tie & 1) ? adx : -adx) | ((uint32_t)(uint16_t)dy << 16);
         A.sad[idx] = sad;
         if (A.surface) A.surface[idx * side * side + (size_t)side * side - 1] = lvalid ? lsad : 0xffffffffu;
     };
@@ -577,9 +591,12 @@ namespace {
 int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width, int32_t rows_in_buffer,
                    int32_t row0_global, int32_t frame_height, int32_t n_pairs, int64_t pair_stride, int32_t block,
                    int32_t range, int32_t mb_row_begin, int32_t mb_row_end, int16_t* mv, uint32_t* best_sad,
-                   uint32_t* surface, void* stream, int32_t pad) {
+                   uint32_t* surface, void* stream, int32_t pad, const int32_t* ready = nullptr) {
     if (block != kMB) return SP_ERR_UNSUPPORTED;
-    if (!ref || !cur || !mv || !best_sad) return SP_ERR_INVALID_ARG;
+    if (ready && !fast_range(range)) return SP_ERR_UNSUPPORTED;  // streamed frames: fast path only
+    if (!ref || !cur || !mv || !best_sad || (reinterpret_cast<uintptr_t>(mv) & 3) ||
+        (reinterpret_cast<uintptr_t>(best_sad) & 3))
+        return SP_ERR_INVALID_ARG;
     if (range < 0 || range > 63 || width < kMB || frame_height < kMB || n_pairs < 0 || rows_in_buffer < 1)
         return SP_ERR_INVALID_ARG;
     if (pitch < width + 2 * pad || (pitch & 15) || (pair_stride & 15) || (reinterpret_cast<uintptr_t>(ref) & 15) ||
@@ -596,7 +613,7 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
     if (n_pairs == 0 || rows == 0 || mbx == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
     MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, pad,
-             pad > 0 ? 1 : 0, mv, best_sad, surface};
+             pad > 0 ? 1 : 0, mv, best_sad, surface, ready};
     if (fast_range(range)) {
         CUtensorMap rm, cm;
         int st;
@@ -641,6 +658,95 @@ extern "C" int sp_me_sad_search_unrestricted(const uint8_t* ref_padded, const ui
     if (range < 0 || pad < range || (fast_range(range) && (pad % 16)) || pad < 1) return SP_ERR_INVALID_ARG;
     return me_search_impl(ref_padded, cur_padded, pitch, width, height + 2 * pad, 0, height, n_pairs, pair_stride,
                           block, range, 0, height / kMB, mv, best_sad, surface, stream, pad);
+}
+
+namespace {
+// A pointer the kernel can store to: device memory as is, page-locked host memory through its
+// device mapping.  Pageable host memory is rejected.
+int me_device_view(void* p, void** out) {
+    cudaPointerAttributes at;
+    SP_CUDA_TRY(cudaPointerGetAttributes(&at, p));
+    if (at.type == cudaMemoryTypeDevice || at.type == cudaMemoryTypeManaged) {
+        *out = p;
+        return SP_OK;
+    }
+    if (at.type == cudaMemoryTypeHost) {
+        SP_CUDA_TRY(cudaHostGetDevicePointer(out, p, 0));
+        return SP_OK;
+    }
+    return SP_ERR_INVALID_ARG;
+}
+
+// library-owned page-locked constant 1: the source of the ready-flag copies (a stream-ordered
+// H2D copy, executed by the copy engine: no SM is needed while the search occupies them all)
+const int32_t* pinned_one() {
+    static int32_t* one = nullptr;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        void* p = nullptr;
+        if (cudaHostAlloc(&p, 64, cudaHostAllocPortable) == cudaSuccess) {
+            one = static_cast<int32_t*>(p);
+            *one = 1;
+        }
+    });
+    return one;
+}
+
+cudaStream_t own_copy_stream() {  // per process; used when the caller passes no copy stream
+    static cudaStream_t cs = nullptr;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        if (cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking) != cudaSuccess) cs = nullptr;
+    });
+    return cs;
+}
+}  // namespace
+
+extern "C" int sp_me_search_host(const uint8_t* frames_host, int64_t pitch, int32_t width, int32_t height,
+                                 int32_t n_frames, int32_t range, uint8_t* frames_dev, int32_t* ready, int16_t* mv,
+                                 uint32_t* best_sad, void* stream, void* copy_stream) {
+    if (!frames_host || !frames_dev || !ready || !mv || !best_sad || n_frames < 1 || height < kMB || width < kMB)
+        return SP_ERR_INVALID_ARG;
+    if (!fast_range(range)) return SP_ERR_UNSUPPORTED;
+    if ((pitch & 15) || pitch < width) return SP_ERR_INVALID_ARG;
+    {
+        cudaPointerAttributes at;
+        SP_CUDA_TRY(cudaPointerGetAttributes(&at, frames_host));
+        if (at.type != cudaMemoryTypeHost) return SP_ERR_INVALID_ARG;  // page-locked frames only
+    }
+    if (n_frames == 1) return SP_OK;
+    void *dmv = nullptr, *dsad = nullptr;
+    int st;
+    if ((st = me_device_view(mv, &dmv)) || (st = me_device_view(best_sad, &dsad))) return st;
+    const int32_t* one = pinned_one();
+    cudaStream_t cs = copy_stream ? (cudaStream_t)copy_stream : own_copy_stream();
+    if (!one || !cs) {
+        sp::set_cuda_error((int)cudaErrorMemoryAllocation);
+        return SP_ERR_CUDA;
+    }
+    const cudaStream_t s = (cudaStream_t)stream;
+    const size_t fbytes = (size_t)pitch * height;
+    const int32_t pairs = n_frames - 1;
+    // ready flags cleared in stream order before the copies may set them
+    cudaEvent_t ev0, ev1;
+    SP_CUDA_TRY(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming));
+    SP_CUDA_TRY(cudaEventCreateWithFlags(&ev1, cudaEventDisableTiming));
+    SP_CUDA_TRY(cudaMemsetAsync(ready, 0, (size_t)pairs * sizeof(int32_t), s));
+    SP_CUDA_TRY(cudaEventRecord(ev0, s));
+    SP_CUDA_TRY(cudaStreamWaitEvent(cs, ev0, 0));
+    for (int32_t f = 0; f < n_frames; ++f) {
+        SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f * fbytes, frames_host + f * fbytes, fbytes, cudaMemcpyHostToDevice, cs));
+        if (f >= 1) SP_CUDA_TRY(cudaMemcpyAsync(ready + (f - 1), one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
+    }
+    SP_CUDA_TRY(cudaEventRecord(ev1, cs));
+    st = me_search_impl(frames_dev, frames_dev + fbytes, pitch, width, height, 0, height, pairs, (int64_t)fbytes, kMB,
+                        range, 0, height / kMB, static_cast<int16_t*>(dmv), static_cast<uint32_t*>(dsad), nullptr,
+                        stream, 0, ready);
+    // the caller's stream completes only after the copies did (frames_dev / ready reusable)
+    SP_CUDA_TRY(cudaStreamWaitEvent(s, ev1, 0));
+    cudaEventDestroy(ev0);
+    cudaEventDestroy(ev1);
+    return st;
 }
 
 namespace {

@@ -72,5 +72,34 @@ def main():
             print(f"jacobi copy+run+copy Tt={tt}: best {best:.3f} ms", flush=True)
 
 
-if __name__ == "__main__":
+if __name__ == "__main__" and "--me" not in sys.argv:
     main()
+
+
+def me_main():
+    W, H, R, F = 1920, 1080, 32, 65
+    fr = sp_inputs.me_sequence(F, W, H, R)
+    h = torch.from_numpy(fr).pin_memory()
+    d = h.cuda()
+    ctx = sp.MESearchHost(F, W, H, fr.shape[2], R)
+    best, med = ev_time(lambda: sp.me_search_sequence(d, W, H, R), reps=3)
+    print(f"ME device-resident: best {best:.3f} ms", flush=True)
+    best, med = ev_time(lambda: ctx.run(h), reps=3)
+    t0 = time.perf_counter()
+    for _ in range(3):
+        ctx.run(h)
+    torch.cuda.synchronize()
+    wall = (time.perf_counter() - t0) / 3 * 1e3
+    print(f"ME host e2e: events best {best:.3f} ms; wall {wall:.3f} ms -> {32934600 * 64 / (wall * 1e-3) / 1e9:.1f} GSAD/s",
+          flush=True)
+    t0 = time.perf_counter()
+    for _ in range(3):
+        dd = h.to("cuda", non_blocking=True)
+        mv, sad, _ = sp.me_search_sequence(dd, W, H, R)
+        mv.cpu(), sad.cpu()
+    torch.cuda.synchronize()
+    print(f"ME copy+run+copy wall {(time.perf_counter() - t0) / 3 * 1e3:.3f} ms", flush=True)
+
+
+if __name__ == "__main__" and "--me" in sys.argv:
+    me_main()
