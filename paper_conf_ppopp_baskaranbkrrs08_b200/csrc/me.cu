@@ -43,6 +43,14 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 #ifndef SP_ME_EXP
 #define SP_ME_EXP 0
 #endif
+#if SP_ME_EXP & 32  // development instrumentation: (smid, start, end) global timer per CTA
+__device__ unsigned long long g_me_cta[4096][3];
+__device__ __forceinline__ unsigned long long globaltimer() {
+    unsigned long long t;
+    asm volatile("mov.u64 %0, %%globaltimer;" : "=l"(t));
+    return t;
+}
+#endif
 #if SP_ME_EXP & 16  // development instrumentation: per-section cycle counts per warp
 __device__ unsigned long long g_me_prof[8];
 #define PMARK(k)                                              \
@@ -70,6 +78,11 @@ struct MeArgs {
     // stream-ordered H2D copies of sp_me_search_host, concurrently with the search); the
     // move-in of a macroblock waits for its pair's flag
     const int32_t* ready;
+    // dynamic macroblock distribution: CTA c takes macroblock c first, then the next index
+    // from this counter (zeroed before the launch) + gridDim.x.  Co-resident CTAs progress at
+    // very different rates (measured: the first of four CTAs on an SM finished after 2.8 ms,
+    // the last after 8.8 ms under a static assignment), so static shares left SMs idle.
+    uint32_t* counter;
 };
 
 __device__ __forceinline__ uint64_t make_key(uint32_t s, int dx, int dy, int R) {
@@ -131,7 +144,20 @@ __device__ __forceinline__ bool tail_candidate(int warp, int lane, int t, int& d
     return col;
 }
 
-template <int R>
+// Frames still streaming in (sp_me_search_host): wait for a pair's ready flag (relaxed poll,
+// then an acquire and a proxy fence order the observed copy before the TMA reads that follow).
+// Out of line: the common device-resident path keeps its register / uniform-datapath layout.
+__device__ __noinline__ void wait_ready(const int32_t* flag) {
+    const long long t0 = clock64();
+    while (ld_relaxed_gpu(flag) == 0) {
+        __nanosleep(256);
+        if (clock64() - t0 > (40ll << 30)) __trap();
+    }
+    (void)ld_acquire_gpu(flag);  // (flags only go 0 -> 1)
+    fence_proxy_async_global();
+}
+
+template <int R, bool kStream>
 __global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
 me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
     using G = MeGeom<R>;
@@ -166,16 +192,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     };
     auto issue = [&](uint32_t mb, int st) {  // single thread: stage the window + cur of mb
         const Pos q = locate(mb);
-        if (A.ready) {  // frames still streaming in: wait for this pair's (relaxed poll, then a
-                        // proxy fence orders the observed copy before the TMA reads below)
-            const long long t0 = clock64();
-            while (ld_relaxed_gpu(A.ready + q.pair) == 0) {
-                __nanosleep(256);
-                if (clock64() - t0 > (40ll << 30)) __trap();
-            }
-            (void)ld_acquire_gpu(A.ready + q.pair);  // (flags only go 0 -> 1)
-            fence_proxy_async_global();
-        }
+        if (kStream) wait_ready(A.ready + q.pair);
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         mbar_arrive_expect_tx(&full[st], (uint32_t)(G::kCopy + kMB * kMB));
         tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair, &full[st]);
@@ -201,6 +218,14 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         if (A.surface) A.surface[idx * side * side + (size_t)side * side - 1] = lvalid ? lsad : 0xffffffffu;
     };
 
+#if SP_ME_EXP & 32
+    if (tid == 0 && blockIdx.x < 4096) {
+        unsigned sm;
+        asm volatile("mov.u32 %0, %%smid;" : "=r"(sm));
+        g_me_cta[blockIdx.x][0] = sm;
+        g_me_cta[blockIdx.x][1] = globaltimer();
+    }
+#endif
     if (tid == 0) {
         prefetch_tmap(&ref_map);
         prefetch_tmap(&cur_map);
@@ -249,10 +274,14 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             tinfo[t][1 + st][tid] =
                 (uint32_t)(phase_copy(st, (dxt + R) & 3) - smem) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
     }
-    // macroblock position (pair, MB row, MB column) per stage, written by thread 0 one
-    // macroblock ahead, read after the barrier
+    // macroblock index and position (pair, MB row, MB column) per stage, written by thread 0
+    // one macroblock ahead (before the barrier that precedes their reading)
     __shared__ Pos posS[2];
-    if (tid == 0) posS[0] = locate(blockIdx.x < total ? blockIdx.x : 0);
+    __shared__ uint32_t mbS[2];
+    if (tid == 0) {
+        posS[0] = locate(blockIdx.x < total ? blockIdx.x : 0);
+        mbS[0] = blockIdx.x;
+    }
     __syncthreads();
 #if SP_ME_EXP & 16
     __shared__ unsigned prof_s[nwarps][8];
@@ -261,8 +290,12 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     unsigned t_prev = (unsigned)clock();
 #endif
     int it = 0;
-    for (uint32_t mb = blockIdx.x; mb < total; mb += Gs, ++it) {
+    uint32_t prev_mb = 0;
+    for (uint32_t mb = blockIdx.x; mb < total; ++it) {
         const int s = it & 1;
+        // the next macroblock of this CTA, published in mbS[s^1] before this iteration's barrier
+        // (the atomic's latency hides under the move-in wait and the phase build)
+        if (tid == 0) mbS[s ^ 1] = atomicAdd(A.counter, 1u) + Gs;
         mbar_wait(&full[s], (it >> 1) & 1);
         PMARK(0);
         {   // byte-phase copies (word q of copy p = bytes [4q+p, 4q+p+4) of the row):
@@ -296,12 +329,13 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // the only CTA barrier per macroblock: phase copies of stage s complete; every warp
         // is done with stage s^1 (previous macroblock) and has posted its key for it
         __syncthreads();
-        if (tid == 0 && mb + Gs < total) {
+        const uint32_t next_mb = mbS[s ^ 1];
+        if (tid == 0 && next_mb < total) {
             fence_proxy_async_smem();
-            issue(mb + Gs, s ^ 1);
-            posS[s ^ 1] = locate(mb + Gs);
+            issue(next_mb, s ^ 1);
+            posS[s ^ 1] = locate(next_mb);
         }
-        if (tid == G::kThreads - 32 && it > 0) finalize(mb - Gs, s ^ 1);
+        if (tid == G::kThreads - 32 && it > 0) finalize(prev_mb, s ^ 1);
         PMARK(2);
 
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
@@ -445,13 +479,18 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         key = __reduce_min_sync(0xffffffffu, key);
         if (lane == 0) red32[s][warp] = key;
         PMARK(7);
+        prev_mb = mb;
+        mb = next_mb;
     }
 #if SP_ME_EXP & 16
     if (lane == 0)
         for (int k = 0; k < 8; ++k) atomicAdd(&g_me_prof[k], (unsigned long long)prof_s[warp][k]);
 #endif
     __syncthreads();
-    if (tid == G::kThreads - 32 && it > 0) finalize(blockIdx.x + (uint32_t)(it - 1) * Gs, (it - 1) & 1);
+    if (tid == G::kThreads - 32 && it > 0) finalize(prev_mb, (it - 1) & 1);
+#if SP_ME_EXP & 32
+    if (tid == 0 && blockIdx.x < 4096) g_me_cta[blockIdx.x][2] = globaltimer();
+#endif
 }
 
 // Generic path (any 0 <= R <= 63): window staged byte-wise with zero fill, one thread per
@@ -550,7 +589,32 @@ int make_map(CUtensorMap* m, const uint8_t* base, int32_t width, int32_t rows, i
 
 bool fast_range(int R) { return R == 16 || R == 32; }
 
-template <int R>
+// The fast kernel's macroblock counter: one slot of a small per-device ring (library-owned,
+// allocated once), zeroed on the launch stream; concurrent launches on different streams
+// take different slots.
+int counter_slot(cudaStream_t s, uint32_t** out) {
+    constexpr int kSlots = 4096;
+    static std::mutex mu;
+    static uint32_t* ring[64] = {};
+    static uint32_t next[64] = {};
+    int dev = 0;
+    SP_CUDA_TRY(cudaGetDevice(&dev));
+    uint32_t* slot;
+    {
+        std::lock_guard<std::mutex> lk(mu);
+        if (!ring[dev & 63]) {
+            void* p = nullptr;
+            SP_CUDA_TRY(cudaMalloc(&p, kSlots * sizeof(uint32_t)));
+            ring[dev & 63] = static_cast<uint32_t*>(p);
+        }
+        slot = ring[dev & 63] + (next[dev & 63]++ % kSlots);
+    }
+    SP_CUDA_TRY(cudaMemsetAsync(slot, 0, sizeof(uint32_t), s));
+    *out = slot;
+    return SP_OK;
+}
+
+template <int R, bool kStream>
 int launch_fast(const CUtensorMap& rm, const CUtensorMap& cm, const MeArgs& a, int64_t total, cudaStream_t s) {
     using G = MeGeom<R>;
     static int grid_cap = 0;
@@ -561,14 +625,14 @@ int launch_fast(const CUtensorMap& rm, const CUtensorMap& cm, const MeArgs& a, i
         err = cudaGetDevice(&dev);
         if (err == cudaSuccess) err = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
         if (err == cudaSuccess)
-            err = cudaFuncSetAttribute(me_sad_kernel<R>, cudaFuncAttributeMaxDynamicSharedMemorySize, G::kSmem);
+            err = cudaFuncSetAttribute(me_sad_kernel<R, kStream>, cudaFuncAttributeMaxDynamicSharedMemorySize, G::kSmem);
         if (err == cudaSuccess)
-            err = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, me_sad_kernel<R>, G::kThreads, G::kSmem);
+            err = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, me_sad_kernel<R, kStream>, G::kThreads, G::kSmem);
         grid_cap = sms * (occ > 0 ? occ : 1);
     });
     SP_CUDA_TRY(err);
     const int grid = (int)(total < grid_cap ? total : grid_cap);
-    me_sad_kernel<R><<<grid, G::kThreads, G::kSmem, s>>>(rm, cm, a);
+    me_sad_kernel<R, kStream><<<grid, G::kThreads, G::kSmem, s>>>(rm, cm, a);
     return SP_OK;
 }
 
@@ -613,8 +677,10 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
     if (n_pairs == 0 || rows == 0 || mbx == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
     MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, pad,
-             pad > 0 ? 1 : 0, mv, best_sad, surface, ready};
+             pad > 0 ? 1 : 0, mv, best_sad, surface, ready, nullptr};
     if (fast_range(range)) {
+        int st0;
+        if ((st0 = counter_slot(s, &a.counter))) return st0;
         CUtensorMap rm, cm;
         int st;
         const int64_t ps = n_pairs > 1 ? pair_stride : pitch * rows_in_buffer;
@@ -624,8 +690,10 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
         a.n_pairs = n_pairs;
         const int64_t total = (int64_t)mbx * rows * n_pairs;
         if (total >= (int64_t(1) << 31)) return SP_ERR_UNSUPPORTED;  // 32-bit macroblock indices in the kernel
-        if (range == 32) st = launch_fast<32>(rm, cm, a, total, s);
-        else st = launch_fast<16>(rm, cm, a, total, s);
+        // (the streamed-frames variant is a separate instantiation: the flag wait in its move-in
+        // costs the device-resident kernel its uniform-datapath index math, 2 % of M4)
+        if (range == 32) st = ready ? launch_fast<32, true>(rm, cm, a, total, s) : launch_fast<32, false>(rm, cm, a, total, s);
+        else st = ready ? launch_fast<16, true>(rm, cm, a, total, s) : launch_fast<16, false>(rm, cm, a, total, s);
         if (st) return st;
     } else {
         const int smem = a.win * a.win + kMB * kMB;
@@ -780,6 +848,12 @@ extern "C" int sp_me_pad_frames(const uint8_t* src, int64_t src_pitch, int64_t s
     return SP_OK;
 }
 
+#if SP_ME_EXP & 32
+extern "C" int sp_me_cta_read(unsigned long long* out) {
+    SP_CUDA_TRY(cudaMemcpyFromSymbol(out, g_me_cta, sizeof(unsigned long long) * 4096 * 3));
+    return SP_OK;
+}
+#endif
 #if SP_ME_EXP & 16
 // development instrumentation only (tools/me_sections.py): read and reset the section counters
 extern "C" int sp_me_prof_read(unsigned long long* out) {
