@@ -21,6 +21,14 @@ sp.jacobi1d_timetiled(a, 20, 5, 0)
 mark("sp.jacobi1d_timetiled_fused")
 sp.jacobi1d_timetiled_fused(a, 37, 16, 256)
 sp.jacobi1d_timetiled_fused(a, 20, 5, 8)
+mark("sp.jacobi1d_timetiled_stream (wavefront, device)")
+o = torch.empty_like(a)
+sp.jacobi1d_timetiled_stream(a, o, 37, 16, 256, 4)
+mark("sp.jacobi1d_host (pinned in/out, 3 passes)")
+h = a.cpu().pin_memory()
+sp.Jacobi1DHost(4099, 37, 16, 256).run(h)
+mark("sp.jacobi1d_host (1 pass: redirect + copy)")
+sp.Jacobi1DHost(4099, 9, 16, 0).run(h)
 mark("sp.jacobi1d_untiled")
 sp.jacobi1d_untiled(a, 3)
 fr = torch.from_numpy(sp_inputs.me_sequence(3, 352, 288, 16)).cuda()
@@ -33,6 +41,8 @@ mark("sp.me_search_sequence")
 sp.me_search_sequence(fr2, 130, 70, 5)
 mark("sp.me_search_sequence_unrestricted")
 sp.me_search_sequence_unrestricted(fr2, 130, 70, 32)
+mark("sp.me_search_host (streamed frames, pinned outputs)")
+sp.MESearchHost(3, 352, 288, fr.shape[2], 16).run(fr.cpu().pin_memory())
 mark("sp.me_sad_search_direct")
 sp.me_sad_search_direct(fr2[:-1], fr2[1:], 130, 70, 8)
 torch.cuda.synchronize()
