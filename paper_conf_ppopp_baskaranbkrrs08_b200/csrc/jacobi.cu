@@ -531,8 +531,11 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 #ifdef SP_JAC_DEBUG
         const long long tp0 = clock64();
 #endif
-        if (lane == 0 && pers) publish(true);  // (waiting for the newest store here beats a
-                                                // one-tile publication lag: 6.94 vs 7.01 ms on J3)
+        // Publication: pass-major order publishes a tile one tile late (its store has long
+        // completed by then, so the warp never waits for it: 6.89 vs 6.97 ms on J3, A/B on one
+        // box); in the wavefront order dependents follow closely, so the newest store is waited
+        // for and published at once.
+        if (lane == 0 && pers) publish(A.skew != 0);
         if (u_next < total) {
             pending = (pers && pn > 0 && 2 * reach < 32) ? !__all_sync(0xffffffffu, next_flag >= pn) : !deps_ready(tn, pn);
             if (lane == 0) {

@@ -39,11 +39,18 @@ def emit(**kw):
     print(json.dumps(kw), flush=True)
 
 
-def jacobi_pair(n, T, tt=32, S=0, untiled=True):
+def jacobi_pair(n, T, tt=32, S=0, untiled=True, per_pass=False):
+    """staged time (persistent all-pass launch, the product path), DRAM-only time; with
+    per_pass the one-launch-per-time-tile staged path is timed instead of the persistent one"""
     a0 = torch.from_numpy(sp_inputs.jacobi_input(n, seed=2008)).cuda()
     a = a0.clone()
     w = torch.empty_like(a)
-    t_st = ev(lambda: sp.jacobi1d_timetiled(a, T, tt, S, work=w))
+    plan = sp.jacobi1d_plan(n, T, tt, S)
+    fl = torch.empty(plan["tiles"] + 1 + plan["passes"], dtype=torch.int32, device="cuda")
+    if per_pass:
+        t_st = ev(lambda: sp.jacobi1d_timetiled(a, T, tt, S, work=w))
+    else:
+        t_st = ev(lambda: sp.jacobi1d_timetiled_fused(a, T, tt, S, work=w, flags=fl))
     t_un = ev(lambda: sp.jacobi1d_untiled(a, T, work=w)) if untiled else None
     return t_st, t_un
 
@@ -52,9 +59,11 @@ def main():
     quick = len(sys.argv) > 1 and sys.argv[1] == "quick"
     # ---- Figs. 4/5 + speedup claims at the BASELINE configs -------------------------------
     n, T = 1 << 26, 1024
-    t_st, t_un = jacobi_pair(n, T)
-    emit(exp="jacobi_staged_vs_dram_only", n=n, T=T, time_tile=32, staged_ms=t_st, dram_only_ms=t_un,
-         speedup=t_un / t_st, paper_speedup_8800gtx=10.0, updates_per_s_staged=(n - 2) * T / (t_st * 1e-3))
+    t_st, t_un = jacobi_pair(n, T, 64)
+    t_pp, _ = jacobi_pair(n, T, 64, untiled=False, per_pass=True)
+    emit(exp="jacobi_staged_vs_dram_only", n=n, T=T, time_tile=64, staged_ms=t_st, staged_per_pass_ms=t_pp,
+         dram_only_ms=t_un, speedup=t_un / t_st, paper_speedup_8800gtx=10.0,
+         updates_per_s_staged=(n - 2) * T / (t_st * 1e-3))
     W, H, R = 1920, 1080, 32
     fr = torch.from_numpy(sp_inputs.me_sequence(9 if quick else 65, W, H, R)).cuda()
     t_me = ev(lambda: sp.me_search_sequence(fr, W, H, R))
@@ -64,7 +73,9 @@ def main():
     # ---- Fig. 5 problem-size range (8k..512k), T = 4096 ------------------------------------
     for n in [8 << 10, 32 << 10, 128 << 10, 512 << 10]:
         t_st, t_un = jacobi_pair(n, 4096)
-        emit(exp="fig5_jacobi_size", n=n, T=4096, staged_ms=t_st, dram_only_ms=t_un, speedup=t_un / t_st)
+        t_pp, _ = jacobi_pair(n, 4096, untiled=False, per_pass=True)
+        emit(exp="fig5_jacobi_size", n=n, T=4096, staged_ms=t_st, staged_per_pass_ms=t_pp, dram_only_ms=t_un,
+             speedup=t_un / t_st)
     # ---- Fig. 8: (time, space) tiles at 64k..512k, T = 4096 --------------------------------
     for n in [64 << 10, 512 << 10]:
         for tt, S in [(32, 64), (32, 128), (16, 256), (32, 256), (64, 256), (32, 1024), (32, 0)]:
@@ -81,7 +92,8 @@ def main():
                 t_st, _ = jacobi_pair(n, 4096, 32, S, untiled=False)
             except sp.SPError:
                 continue
-            emit(exp="fig7_jacobi_tiles_count", n=n, T=4096, space_tile=S, tiles=-(-n // S), ms=t_st)
+            t_pp, _ = jacobi_pair(n, 4096, 32, S, untiled=False, per_pass=True)
+            emit(exp="fig7_jacobi_tiles_count", n=n, T=4096, space_tile=S, tiles=-(-n // S), ms=t_st, per_pass_ms=t_pp)
     # ---- staged Jacobi across time tiles at J3 (HBM <-> FP32 cross-over) --------------------
     for tt in [4, 8, 16, 24, 32, 48, 64]:
         t_st, _ = jacobi_pair(1 << 26, 1024, tt, 0, untiled=False)
