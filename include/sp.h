@@ -227,6 +227,18 @@ int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float
 int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t* flags, int64_t flags_len, int64_t n,
                      int32_t steps, int32_t time_tile, int32_t space_tile, void* stream);
 
+/* Cluster-resident form for small domains (the paper's "fits in the scratchpad" regime,
+ * P:L964-1052, Figs. 5 and 7): the whole array is moved in once into the registers of ONE
+ * thread-block cluster (up to 16 CTAs x 8 warps, 1,764 owned cells per warp), all `steps`
+ * run on chip, and it is moved out once.  Warps exchange 14-cell halos every 14 steps
+ * (shared memory inside a CTA, distributed shared memory across the cluster, one cluster
+ * barrier per exchange) — the time tile is fixed at 14, the halo equal to it.
+ *   in, out : device arrays of n fp32 (may alias); n >= 3, steps >= 0.
+ * Errors: SP_ERR_UNSUPPORTED if n exceeds sp_jacobi1d_resident_capacity (which reports the
+ * largest n the device can hold in one cluster: 16 x 8 x 1764 = 225,792 cells on B200). */
+int sp_jacobi1d_resident_capacity(int64_t* max_cells);
+int sp_jacobi1d_resident(const float* in, float* out, int64_t n, int32_t steps, void* stream);
+
 /* Segment form (building block of the multi-GPU layer and of its single-GPU loopback
  * test): one pass of height h over a window of the global domain.
  *   src/dst : device arrays holding global cells [g0, g0 + len); dst receives the new

@@ -19,6 +19,7 @@ C entry point -> Python name (same names, `sp_` prefix dropped):
   sp_jacobi1d_timetiled_fused -> jacobi1d_timetiled_fused(a, steps, ...) (one persistent launch)
   sp_jacobi1d_timetiled_stream -> jacobi1d_timetiled_stream(inp, out, steps, ...) (device or pinned host)
   sp_jacobi1d_host            -> Jacobi1DHost(n, steps, ...).run(a_pinned)  (the e2e public call)
+  sp_jacobi1d_resident        -> jacobi1d_resident(a, steps)   (small domains: one cluster)
   sp_jacobi1d_pass_segment    -> jacobi1d_pass_segment(...)
   sp_jacobi1d_timetiled_loopback -> jacobi1d_timetiled_loopback(...)
   sp_jacobi1d_timetiled_dist  -> Comm.jacobi1d_timetiled_dist(...)
@@ -39,7 +40,7 @@ import numpy as np
 __all__ = [
     "SPError", "lib", "plan_buffers", "jacobi1d_plan", "jacobi1d_tile_footprint", "jacobi1d_timetiled",
     "jacobi1d_pass_segment", "jacobi1d_timetiled_loopback", "me_sad_search", "me_ref_window", "me_search_sequence",
-    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
+    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "jacobi1d_resident", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
 ]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
@@ -136,6 +137,8 @@ SYMBOLS = {
     "sp_jacobi1d_timetiled_fused": (ctypes.c_int, [vp, vp, vp, i64, i64, i32, i32, i32, vp, vp]),
     "sp_jacobi1d_timetiled_stream": (ctypes.c_int, [vp, vp, vp, vp, vp, i64, i64, i32, i32, i32, i64, vp, vp]),
     "sp_jacobi1d_host": (ctypes.c_int, [vp, vp, vp, vp, i64, i64, i32, i32, i32, vp]),
+    "sp_jacobi1d_resident_capacity": (ctypes.c_int, [ctypes.POINTER(i64)]),
+    "sp_jacobi1d_resident": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
     "sp_me_search_host": (ctypes.c_int, [vp, i64, i32, i32, i32, i32, vp, vp, vp, vp, vp, vp]),
     "sp_me_ref_window": (ctypes.c_int, [i32, i32, i32, i32, i32, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
@@ -170,6 +173,8 @@ def _load():
                           " There is no CPU fallback.")
     L = ctypes.CDLL(LIB_PATH)
     for name, (res, args) in SYMBOLS.items():
+        if os.environ.get("SP_LIB") and not hasattr(L, name):
+            continue  # an experimental build (SP_LIB) may predate a symbol; the product lib may not
         fn = getattr(L, name)
         fn.restype = res
         fn.argtypes = args
@@ -422,6 +427,23 @@ def jacobi1d_timetiled_stream(inp, out, steps: int, time_tile: int = 64, space_t
     _check(lib.sp_jacobi1d_timetiled_stream(_ptr(inp), _ptr(out), _ptr(buf0), _ptr(buf1), _ptr(flags), flags.numel(), n,
                                             int(steps), int(time_tile), int(space_tile), int(skew), _ptr(footprint_log),
                                             _stream(stream)), "sp_jacobi1d_timetiled_stream")
+    return out
+
+
+def jacobi1d_resident_capacity() -> int:
+    c = i64()
+    _check(lib.sp_jacobi1d_resident_capacity(ctypes.byref(c)), "sp_jacobi1d_resident_capacity")
+    return c.value
+
+
+def jacobi1d_resident(inp, steps: int, out=None, stream=None):
+    """Small domains: out = J^steps(inp) in one thread-block cluster (sp_jacobi1d_resident);
+    inp / out CUDA float32 (out defaults to inp, in place)."""
+    import torch
+    assert inp.is_cuda and inp.dtype == torch.float32 and inp.is_contiguous()
+    out = inp if out is None else out
+    _check(lib.sp_jacobi1d_resident(_ptr(inp), _ptr(out), inp.numel(), int(steps), _stream(stream)),
+           "sp_jacobi1d_resident")
     return out
 
 

@@ -18,6 +18,7 @@
 //     shared memory -> coalesced 128-bit global stores.
 // Arithmetic is b = ((a[i-1] + a[i]) + a[i+1]) * w, each op rounded to nearest fp32, never
 // contracted (PTX add.rn/mul.rn), w = fl32(1/3) — bit-identical to the definition.
+#include <cooperative_groups.h>
 #include <cuda_runtime.h>
 
 #include <algorithm>
@@ -190,6 +191,146 @@ __device__ __forceinline__ void run_steps(uint64_t (&P)[kK], int h, int lane, ui
     if (k < h) {
         step(P, Q, left, right, lane, w2, mz);
         if (kBoundary) restore(Q, f0, fn, v0, vn);
+#pragma unroll
+        for (int j = 0; j < kK; ++j) P[j] = Q[j];
+    }
+}
+
+// The cluster-resident kernel describes a fixed cell warp-uniformly as
+// fx = j | hi << 8 | lane << 9 (pair j, component hi, owning lane; -1: none), so its restore
+// is one warp-uniform jump to pair j and a single-lane move — a few instructions per step
+// instead of the ~4K mask tests above, which made its boundary warps the critical path of
+// every exchange barrier (8192 cells x 4096 steps: 4.32 -> 1.55 ms).  (The pass kernel keeps
+// the mask form: with the jump table its common path lost registers, 6.89 -> 7.03 ms.)
+struct FixedCells {
+    int fx0, fx1;  // descriptors of cell 0 and cell n-1 in this strip (-1: not in it)
+    float v0, v1;  // their values
+    bool edge;     // one of them sits in an edge pair (0 or K-1): the shuffles must be redone
+};
+template <int kK>
+__device__ __forceinline__ FixedCells fixed_cells(int64_t base, int64_t n, float v0, float vn) {
+    FixedCells f{-1, -1, v0, vn, false};
+    auto desc = [&](int64_t c) -> int {
+        const int64_t s = c - base;
+        if (s < 0 || s >= 64 * kK) return -1;
+        const int hi = s >= 32 * kK, r = (int)(s - (hi ? 32 * kK : 0));
+        return (r % kK) | (hi << 8) | ((r / kK) << 9);
+    };
+    f.fx0 = desc(0);
+    f.fx1 = desc(n - 1);
+    for (int fx : {f.fx0, f.fx1})
+        if (fx >= 0 && ((fx & 255) == 0 || (fx & 255) == kK - 1)) f.edge = true;
+    return f;
+}
+template <int kK>
+__device__ __forceinline__ void restore_one(uint64_t (&Q)[kK], int lane, int fx, float val) {
+    if (fx < 0) return;  // warp-uniform
+    const bool me = lane == (fx >> 9), hi = (fx >> 8) & 1;
+#define SP_FIX_CASE(J)                                                                          \
+    case J:                                                                                     \
+        if constexpr (J < kK) {                                                                 \
+            if (me) Q[J] = hi ? f2_pack(f2_lo(Q[J]), val) : f2_pack(val, f2_hi(Q[J]));          \
+        }                                                                                       \
+        break;
+    switch (fx & 255) {
+        SP_FIX_CASE(0)
+        SP_FIX_CASE(1)
+        SP_FIX_CASE(2)
+        SP_FIX_CASE(3)
+        SP_FIX_CASE(4)
+        SP_FIX_CASE(5)
+        SP_FIX_CASE(6)
+        SP_FIX_CASE(7)
+        SP_FIX_CASE(8)
+        SP_FIX_CASE(9)
+        SP_FIX_CASE(10)
+        SP_FIX_CASE(11)
+        SP_FIX_CASE(12)
+        SP_FIX_CASE(13)
+        SP_FIX_CASE(14)
+        SP_FIX_CASE(15)
+        SP_FIX_CASE(16)
+        SP_FIX_CASE(17)
+        SP_FIX_CASE(18)
+        SP_FIX_CASE(19)
+        SP_FIX_CASE(20)
+        SP_FIX_CASE(21)
+        SP_FIX_CASE(22)
+        SP_FIX_CASE(23)
+        SP_FIX_CASE(24)
+        SP_FIX_CASE(25)
+        SP_FIX_CASE(26)
+        SP_FIX_CASE(27)
+        SP_FIX_CASE(28)
+        SP_FIX_CASE(29)
+        SP_FIX_CASE(30)
+        SP_FIX_CASE(31)
+        SP_FIX_CASE(32)
+        SP_FIX_CASE(33)
+        SP_FIX_CASE(34)
+        SP_FIX_CASE(35)
+        SP_FIX_CASE(36)
+        SP_FIX_CASE(37)
+        SP_FIX_CASE(38)
+        SP_FIX_CASE(39)
+        SP_FIX_CASE(40)
+        SP_FIX_CASE(41)
+        SP_FIX_CASE(42)
+        SP_FIX_CASE(43)
+        SP_FIX_CASE(44)
+        SP_FIX_CASE(45)
+        SP_FIX_CASE(46)
+        SP_FIX_CASE(47)
+        SP_FIX_CASE(48)
+        SP_FIX_CASE(49)
+        SP_FIX_CASE(50)
+        SP_FIX_CASE(51)
+        SP_FIX_CASE(52)
+        SP_FIX_CASE(53)
+        SP_FIX_CASE(54)
+        SP_FIX_CASE(55)
+        SP_FIX_CASE(56)
+        SP_FIX_CASE(57)
+        SP_FIX_CASE(58)
+        SP_FIX_CASE(59)
+        SP_FIX_CASE(60)
+        SP_FIX_CASE(61)
+        SP_FIX_CASE(62)
+        SP_FIX_CASE(63)
+        default: break;
+    }
+#undef SP_FIX_CASE
+}
+template <int kK>
+__device__ __forceinline__ void restore(uint64_t (&Q)[kK], int lane, const FixedCells& f) {
+    restore_one(Q, lane, f.fx0, f.v0);
+    restore_one(Q, lane, f.fx1, f.v1);
+}
+
+// run_steps with the jump-table restore (the cluster-resident kernel, where the boundary
+// warps are on every exchange barrier's critical path)
+template <bool kBoundary, int kK>
+__device__ __forceinline__ void run_steps_fx(uint64_t (&P)[kK], int h, int lane, uint64_t w2, uint64_t mz,
+                                             const FixedCells& f) {
+    uint64_t Q[kK];
+    uint64_t left, right;
+    neighbours<kK>(P[0], P[kK - 1], lane, left, right);
+    int k = 0;
+    for (; k + 2 <= h; k += 2) {
+        step(P, Q, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore(Q, lane, f);
+            if (f.edge) neighbours<kK>(Q[0], Q[kK - 1], lane, left, right);
+        }
+        step(Q, P, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore(P, lane, f);
+            if (f.edge) neighbours<kK>(P[0], P[kK - 1], lane, left, right);
+        }
+    }
+    if (k < h) {
+        step(P, Q, left, right, lane, w2, mz);
+        if (kBoundary) restore(Q, lane, f);
 #pragma unroll
         for (int j = 0; j < kK; ++j) P[j] = Q[j];
     }
@@ -737,6 +878,81 @@ int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v) {
     return SP_OK;
 }
 
+
+// ---- cluster-resident time stepping (small domains) --------------------------------------
+// When the whole domain fits in the registers of one thread-block cluster, the staged tile is
+// the domain itself: it is moved in once, all T steps run on chip, and it is moved out once.
+// The warps of the cluster own consecutive segments of L = 64K - 2E cells; each holds its
+// segment plus E halo cells per side (a 64K-cell strip) and, every E steps, replaces its halos
+// with the neighbours' edge cells — through shared memory inside a CTA and distributed shared
+// memory (DSMEM) across the CTAs of the cluster, one cluster barrier per exchange (the
+// hardware form of the paper's "synchronization across all thread blocks" per time tile,
+// P:L1009-1017).  Redundant updates: 2E per 64K cells (1.6 % at K = 28, E = 14).
+template <int kK, int kWarps, int kE>
+__global__ void __launch_bounds__(32 * kWarps, 1)
+    jacobi1d_cluster_kernel(const float* __restrict__ src, float* __restrict__ dst, int64_t n, int32_t steps,
+                            uint64_t mz) {
+    static_assert(2 * kE <= kK, "exports must lie in one lane's cells");
+    namespace cg = cooperative_groups;
+    cg::cluster_group cluster = cg::this_cluster();
+    __shared__ float xch[2][2][kWarps][kE];  // [exchange parity][0: left edge, 1: right edge][warp][cell]
+    const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+    const int rank = (int)cluster.block_rank();
+    const int G = (int)gridDim.x * kWarps;  // the grid is one cluster
+    const int g = rank * kWarps + warp;
+    constexpr int kStrip = 64 * kK, L = kStrip - 2 * kE;
+    const int64_t base = (int64_t)g * L - kE;  // strip cell j <-> global cell base + j
+    const uint64_t w2 = (uint64_t(kW) << 32) | kW;
+    uint64_t P[kK];
+#pragma unroll
+    for (int j = 0; j < kK; ++j) {
+        const int64_t cu = base + lane * kK + j, cv = base + 32 * kK + lane * kK + j;
+        P[j] = f2_pack(cu >= 0 && cu < n ? src[cu] : 0.f, cv >= 0 && cv < n ? src[cv] : 0.f);
+    }
+    const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= n - 1 && n - 1 < base + kStrip);
+    const FixedCells fc = boundary ? fixed_cells<kK>(base, n, src[0], src[n - 1]) : FixedCells{-1, -1, 0.f, 0.f, false};
+    cluster.sync();  // every read of src precedes any write of dst (in place allowed)
+    int q = 0;
+    for (int done = 0; done < steps; done += kE) {
+        const int h = steps - done < kE ? steps - done : kE;
+        if (boundary) run_steps_fx<true>(P, h, lane, w2, mz, fc);
+        else run_steps_fx<false>(P, h, lane, w2, mz, fc);
+        if (done + h >= steps) break;
+        // exchange: edges out (strip cells [E, 2E) and [64K-2E, 64K-E)), barrier, halos in
+        if (lane == 0) {
+#pragma unroll
+            for (int j = 0; j < kE; ++j) xch[q][0][warp][j] = f2_lo(P[kE + j]);
+        }
+        if (lane == 31) {
+#pragma unroll
+            for (int j = 0; j < kE; ++j) xch[q][1][warp][j] = f2_hi(P[kK - 2 * kE + j]);
+        }
+        cluster.sync();
+        if (lane == 0 && g > 0) {
+            const float* e = warp > 0 ? &xch[q][1][warp - 1][0] : cluster.map_shared_rank(&xch[q][1][kWarps - 1][0], rank - 1);
+#pragma unroll
+            for (int j = 0; j < kE; ++j) P[j] = f2_pack(e[j], f2_hi(P[j]));
+        }
+        if (lane == 31 && g < G - 1) {
+            const float* e = warp < kWarps - 1 ? &xch[q][0][warp + 1][0] : cluster.map_shared_rank(&xch[q][0][0][0], rank + 1);
+#pragma unroll
+            for (int j = 0; j < kE; ++j) P[kK - kE + j] = f2_pack(f2_lo(P[kK - kE + j]), e[j]);
+        }
+        q ^= 1;  // (the next exchange writes the other slots; the one after that follows a barrier
+                 //  that every reader of these slots has passed)
+    }
+    // move-out: owned strip cells [E, 64K - E)
+#pragma unroll
+    for (int j = 0; j < kK; ++j) {
+        const int su = lane * kK + j, sv = 32 * kK + lane * kK + j;
+        const int64_t cu = base + su, cv = base + sv;
+        if (su >= kE && su < kStrip - kE && cu >= 0 && cu < n) dst[cu] = f2_lo(P[j]);
+        if (sv >= kE && sv < kStrip - kE && cv >= 0 && cv < n) dst[cv] = f2_hi(P[j]);
+    }
+    cluster.sync();  // (no CTA of the cluster exits while a neighbour may still read its slots)
+}
+constexpr int kResK = 28, kResWarps = 8, kResE = 14;
+
 }  // namespace
 
 extern "C" int sp_jacobi1d_plan(int64_t n, int32_t steps, int32_t time_tile, int32_t space_tile, sp_jacobi_plan* out) {
@@ -1030,5 +1246,65 @@ extern "C" int sp_ipc_open_handle(const uint8_t handle[64], void** ptr) {
 extern "C" int sp_ipc_close_handle(void* ptr) {
     if (!ptr) return SP_ERR_INVALID_ARG;
     SP_CUDA_TRY(cudaIpcCloseMemHandle(ptr));
+    return SP_OK;
+}
+
+extern "C" int sp_jacobi1d_resident_capacity(int64_t* max_cells) {
+    if (!max_cells) return SP_ERR_INVALID_ARG;
+    static int64_t cap = -1;
+    static std::once_flag once;
+    static cudaError_t err = cudaSuccess;
+    std::call_once(once, [] {
+        auto k = jacobi1d_cluster_kernel<kResK, kResWarps, kResE>;
+        err = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+        int best = 0;
+        for (int c = 16; c >= 1 && err == cudaSuccess && !best; c /= 2) {  // largest cluster that fits
+            cudaLaunchConfig_t cfg = {};
+            cudaLaunchAttribute at[1];
+            at[0].id = cudaLaunchAttributeClusterDimension;
+            at[0].val.clusterDim.x = c;
+            at[0].val.clusterDim.y = 1;
+            at[0].val.clusterDim.z = 1;
+            cfg.gridDim = dim3(c);
+            cfg.blockDim = dim3(32 * kResWarps);
+            cfg.attrs = at;
+            cfg.numAttrs = 1;
+            int nc = 0;
+            err = cudaOccupancyMaxActiveClusters(&nc, k, &cfg);
+            if (err == cudaSuccess && nc >= 1) best = c;
+        }
+        cap = (int64_t)best * kResWarps * (64 * kResK - 2 * kResE);
+    });
+    SP_CUDA_TRY(err);
+    *max_cells = cap;
+    return SP_OK;
+}
+
+extern "C" int sp_jacobi1d_resident(const float* in, float* out, int64_t n, int32_t steps, void* stream) {
+    if (!in || !out || n < 3 || steps < 0) return SP_ERR_INVALID_ARG;
+    int64_t cap = 0;
+    int st = sp_jacobi1d_resident_capacity(&cap);
+    if (st) return st;
+    if (n > cap) return SP_ERR_UNSUPPORTED;
+    const cudaStream_t s = (cudaStream_t)stream;
+    if (steps == 0) {
+        if (out != in) SP_CUDA_TRY(cudaMemcpyAsync(out, in, (size_t)n * sizeof(float), cudaMemcpyDefault, s));
+        return SP_OK;
+    }
+    constexpr int64_t L = 64 * kResK - 2 * kResE;
+    const int64_t G = (n + L - 1) / L;
+    const unsigned c = (unsigned)((G + kResWarps - 1) / kResWarps);
+    cudaLaunchConfig_t cfg = {};
+    cudaLaunchAttribute at[1];
+    at[0].id = cudaLaunchAttributeClusterDimension;
+    at[0].val.clusterDim.x = c;
+    at[0].val.clusterDim.y = 1;
+    at[0].val.clusterDim.z = 1;
+    cfg.gridDim = dim3(c);
+    cfg.blockDim = dim3(32 * kResWarps);
+    cfg.stream = s;
+    cfg.attrs = at;
+    cfg.numAttrs = 1;
+    SP_CUDA_TRY(cudaLaunchKernelEx(&cfg, jacobi1d_cluster_kernel<kResK, kResWarps, kResE>, in, out, n, steps, kNegZero2));
     return SP_OK;
 }

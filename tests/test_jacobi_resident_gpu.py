@@ -1,0 +1,60 @@
+"""GPU parity of the cluster-resident Jacobi (sp_jacobi1d_resident: the whole domain in one
+thread-block cluster, halos exchanged every 14 steps through shared / distributed shared
+memory) against the oracle, bit-exact: single warp, several warps, several CTAs of the
+cluster (DSMEM exchanges), the capacity limit, steps around multiples of the exchange
+interval, in place and out of place."""
+import numpy as np
+import pytest
+import torch
+
+import oracle
+import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
+import sp_inputs
+
+pytestmark = pytest.mark.gpu
+SEG = 64 * 28 - 2 * 14  # owned cells per warp
+CTA = 8 * SEG
+
+
+def _check(got, want):
+    got = got.cpu().numpy() if isinstance(got, torch.Tensor) else got
+    assert np.array_equal(got.view(np.uint32), want.view(np.uint32)), "not bit-exact"
+
+
+def test_capacity():
+    assert sp.jacobi1d_resident_capacity() >= CTA
+
+
+@pytest.mark.parametrize("n", [3, 4, 5, 33, 1000, SEG - 1, SEG, SEG + 1, 4096, CTA - 1, CTA, CTA + 1,
+                               3 * CTA + 17, 8192, 32768])
+@pytest.mark.parametrize("steps", [0, 1, 13, 14, 15, 28, 29, 64, 101])
+def test_shapes(n, steps):
+    a = sp_inputs.jacobi_input(n, seed=n + steps)
+    d = torch.from_numpy(a.copy()).cuda()
+    o = torch.empty_like(d)
+    sp.jacobi1d_resident(d, steps, out=o)
+    torch.cuda.synchronize()
+    _check(o, oracle.jacobi1d(a, steps))
+    sp.jacobi1d_resident(d, steps)  # in place
+    torch.cuda.synchronize()
+    _check(d, oracle.jacobi1d(a, steps))
+
+
+def test_J1_and_long_run_at_capacity():
+    a = sp_inputs.jacobi_input(4096, seed=2008)
+    d = torch.from_numpy(a.copy()).cuda()
+    sp.jacobi1d_resident(d, 64)
+    torch.cuda.synchronize()
+    _check(d, oracle.jacobi1d(a, 64))
+    n = sp.jacobi1d_resident_capacity()
+    a = sp_inputs.jacobi_input(n, seed=7)
+    d = torch.from_numpy(a.copy()).cuda()
+    sp.jacobi1d_resident(d, 4096)
+    torch.cuda.synchronize()
+    got = d.cpu().numpy()
+    rng = np.random.default_rng(3)
+    idx = [0, 1, 2, n - 3, n - 2, n - 1] + [k * SEG + o for k in (1, 7, 8, 9, 100) for o in (-1, 0, 1) if k * SEG + o < n]
+    idx = np.unique(np.array(idx + rng.integers(0, n, 30).tolist(), dtype=np.int64))
+    _check(got[idx], oracle.jacobi1d_points(a, 4096, idx))
+    with pytest.raises(sp.SPError):
+        sp.jacobi1d_resident(torch.zeros(n + 1, device="cuda"), 4)

@@ -74,8 +74,12 @@ def main():
     for n in [8 << 10, 32 << 10, 128 << 10, 512 << 10]:
         t_st, t_un = jacobi_pair(n, 4096)
         t_pp, _ = jacobi_pair(n, 4096, untiled=False, per_pass=True)
-        emit(exp="fig5_jacobi_size", n=n, T=4096, staged_ms=t_st, staged_per_pass_ms=t_pp, dram_only_ms=t_un,
-             speedup=t_un / t_st)
+        t_res = None
+        if n <= sp.jacobi1d_resident_capacity():  # the whole domain in one cluster
+            a = torch.from_numpy(sp_inputs.jacobi_input(n, seed=2008)).cuda()
+            t_res = ev(lambda: sp.jacobi1d_resident(a, 4096))
+        emit(exp="fig5_jacobi_size", n=n, T=4096, staged_ms=t_st, staged_per_pass_ms=t_pp, cluster_resident_ms=t_res,
+             dram_only_ms=t_un, speedup=t_un / min(t_st, t_res or t_st))
     # ---- Fig. 8: (time, space) tiles at 64k..512k, T = 4096 --------------------------------
     for n in [64 << 10, 512 << 10]:
         for tt, S in [(32, 64), (32, 128), (16, 256), (32, 256), (64, 256), (32, 1024), (32, 0)]:
