@@ -229,10 +229,11 @@ int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t* flags, in
 
 /* Cluster-resident form for small domains (the paper's "fits in the scratchpad" regime,
  * P:L964-1052, Figs. 5 and 7): the whole array is moved in once into the registers of ONE
- * thread-block cluster (up to 16 CTAs x 8 warps, 1,764 owned cells per warp), all `steps`
- * run on chip, and it is moved out once.  Warps exchange 14-cell halos every 14 steps
- * (shared memory inside a CTA, distributed shared memory across the cluster, one cluster
- * barrier per exchange) — the time tile is fixed at 14, the halo equal to it.
+ * thread-block cluster (up to 16 CTAs x 8 warps), all `steps` run on chip, and it is moved
+ * out once.  Warps exchange E-cell halos every E steps (shared memory inside a CTA,
+ * distributed shared memory across the cluster, one cluster barrier per exchange): E = 6
+ * with 756 owned cells per warp up to 96,768 cells, E = 14 with 1,764 above — the time
+ * tile equals the halo.
  *   in, out : device arrays of n fp32 (may alias); n >= 3, steps >= 0.
  * Errors: SP_ERR_UNSUPPORTED if n exceeds sp_jacobi1d_resident_capacity (which reports the
  * largest n the device can hold in one cluster: 16 x 8 x 1764 = 225,792 cells on B200). */

@@ -951,7 +951,6 @@ __global__ void __launch_bounds__(32 * kWarps, 1)
     }
     cluster.sync();  // (no CTA of the cluster exits while a neighbour may still read its slots)
 }
-constexpr int kResK = 28, kResWarps = 8, kResE = 14;
 
 }  // namespace
 
@@ -1249,62 +1248,92 @@ extern "C" int sp_ipc_close_handle(void* ptr) {
     return SP_OK;
 }
 
+namespace {
+// Cluster-resident configurations: K pairs per lane, warps per CTA, exchange interval E.
+// Fewer cells per warp shorten each warp's latency-bound step (the regime is latency-, not
+// throughput-bound) at the price of capacity; the smallest configuration that holds n runs.
+template <int kK, int kWarps, int kE>
+struct Resident {
+    static constexpr int64_t kSeg = 64 * kK - 2 * kE;  // owned cells per warp
+    static int64_t capacity(cudaError_t& err) {  // largest n one cluster of this shape can hold
+        static int64_t cap = -1;
+        static std::once_flag once;
+        static cudaError_t e0 = cudaSuccess;
+        std::call_once(once, [] {
+            auto k = jacobi1d_cluster_kernel<kK, kWarps, kE>;
+            e0 = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
+            int best = 0;
+            for (int c = 16; c >= 1 && e0 == cudaSuccess && !best; c /= 2) {
+                cudaLaunchConfig_t cfg = {};
+                cudaLaunchAttribute at[1];
+                at[0].id = cudaLaunchAttributeClusterDimension;
+                at[0].val.clusterDim.x = c;
+                at[0].val.clusterDim.y = 1;
+                at[0].val.clusterDim.z = 1;
+                cfg.gridDim = dim3(c);
+                cfg.blockDim = dim3(32 * kWarps);
+                cfg.attrs = at;
+                cfg.numAttrs = 1;
+                int nc = 0;
+                e0 = cudaOccupancyMaxActiveClusters(&nc, k, &cfg);
+                if (e0 == cudaSuccess && nc >= 1) best = c;
+            }
+            cap = (int64_t)best * kWarps * kSeg;
+        });
+        err = e0;
+        return cap;
+    }
+    static int launch(const float* in, float* out, int64_t n, int32_t steps, cudaStream_t s) {
+        const int64_t G = (n + kSeg - 1) / kSeg;
+        cudaLaunchConfig_t cfg = {};
+        cudaLaunchAttribute at[1];
+        at[0].id = cudaLaunchAttributeClusterDimension;
+        at[0].val.clusterDim.x = (unsigned)((G + kWarps - 1) / kWarps);
+        at[0].val.clusterDim.y = 1;
+        at[0].val.clusterDim.z = 1;
+        cfg.gridDim = dim3(at[0].val.clusterDim.x);
+        cfg.blockDim = dim3(32 * kWarps);
+        cfg.stream = s;
+        cfg.attrs = at;
+        cfg.numAttrs = 1;
+        SP_CUDA_TRY(cudaLaunchKernelEx(&cfg, jacobi1d_cluster_kernel<kK, kWarps, kE>, in, out, n, steps, kNegZero2));
+        return SP_OK;
+    }
+};
+using ResidentSmall = Resident<12, 8, 6>;
+using ResidentLarge = Resident<28, 8, 14>;
+int resident_choice() {  // SP_JACOBI_RESIDENT = small | large forces one (sweeps)
+    static int c = [] {
+        const char* e = std::getenv("SP_JACOBI_RESIDENT");
+        return e ? (std::strcmp(e, "small") == 0 ? 1 : std::strcmp(e, "large") == 0 ? 2 : 0) : 0;
+    }();
+    return c;
+}
+}  // namespace
+
 extern "C" int sp_jacobi1d_resident_capacity(int64_t* max_cells) {
     if (!max_cells) return SP_ERR_INVALID_ARG;
-    static int64_t cap = -1;
-    static std::once_flag once;
-    static cudaError_t err = cudaSuccess;
-    std::call_once(once, [] {
-        auto k = jacobi1d_cluster_kernel<kResK, kResWarps, kResE>;
-        err = cudaFuncSetAttribute(k, cudaFuncAttributeNonPortableClusterSizeAllowed, 1);
-        int best = 0;
-        for (int c = 16; c >= 1 && err == cudaSuccess && !best; c /= 2) {  // largest cluster that fits
-            cudaLaunchConfig_t cfg = {};
-            cudaLaunchAttribute at[1];
-            at[0].id = cudaLaunchAttributeClusterDimension;
-            at[0].val.clusterDim.x = c;
-            at[0].val.clusterDim.y = 1;
-            at[0].val.clusterDim.z = 1;
-            cfg.gridDim = dim3(c);
-            cfg.blockDim = dim3(32 * kResWarps);
-            cfg.attrs = at;
-            cfg.numAttrs = 1;
-            int nc = 0;
-            err = cudaOccupancyMaxActiveClusters(&nc, k, &cfg);
-            if (err == cudaSuccess && nc >= 1) best = c;
-        }
-        cap = (int64_t)best * kResWarps * (64 * kResK - 2 * kResE);
-    });
-    SP_CUDA_TRY(err);
+    cudaError_t e = cudaSuccess;
+    const int64_t cap = resident_choice() == 1 ? ResidentSmall::capacity(e) : ResidentLarge::capacity(e);
+    SP_CUDA_TRY(e);
     *max_cells = cap;
     return SP_OK;
 }
 
 extern "C" int sp_jacobi1d_resident(const float* in, float* out, int64_t n, int32_t steps, void* stream) {
     if (!in || !out || n < 3 || steps < 0) return SP_ERR_INVALID_ARG;
-    int64_t cap = 0;
-    int st = sp_jacobi1d_resident_capacity(&cap);
-    if (st) return st;
-    if (n > cap) return SP_ERR_UNSUPPORTED;
+    cudaError_t e = cudaSuccess;
+    const int64_t cap_s = ResidentSmall::capacity(e);
+    SP_CUDA_TRY(e);
+    const int64_t cap_l = ResidentLarge::capacity(e);
+    SP_CUDA_TRY(e);
+    const int ch = resident_choice();
+    const bool small = ch == 1 || (ch == 0 && n <= cap_s);
+    if (n > (small ? cap_s : cap_l)) return SP_ERR_UNSUPPORTED;
     const cudaStream_t s = (cudaStream_t)stream;
     if (steps == 0) {
         if (out != in) SP_CUDA_TRY(cudaMemcpyAsync(out, in, (size_t)n * sizeof(float), cudaMemcpyDefault, s));
         return SP_OK;
     }
-    constexpr int64_t L = 64 * kResK - 2 * kResE;
-    const int64_t G = (n + L - 1) / L;
-    const unsigned c = (unsigned)((G + kResWarps - 1) / kResWarps);
-    cudaLaunchConfig_t cfg = {};
-    cudaLaunchAttribute at[1];
-    at[0].id = cudaLaunchAttributeClusterDimension;
-    at[0].val.clusterDim.x = c;
-    at[0].val.clusterDim.y = 1;
-    at[0].val.clusterDim.z = 1;
-    cfg.gridDim = dim3(c);
-    cfg.blockDim = dim3(32 * kResWarps);
-    cfg.stream = s;
-    cfg.attrs = at;
-    cfg.numAttrs = 1;
-    SP_CUDA_TRY(cudaLaunchKernelEx(&cfg, jacobi1d_cluster_kernel<kResK, kResWarps, kResE>, in, out, n, steps, kNegZero2));
-    return SP_OK;
+    return small ? ResidentSmall::launch(in, out, n, steps, s) : ResidentLarge::launch(in, out, n, steps, s);
 }

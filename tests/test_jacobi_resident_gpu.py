@@ -1,8 +1,9 @@
 """GPU parity of the cluster-resident Jacobi (sp_jacobi1d_resident: the whole domain in one
-thread-block cluster, halos exchanged every 14 steps through shared / distributed shared
-memory) against the oracle, bit-exact: single warp, several warps, several CTAs of the
-cluster (DSMEM exchanges), the capacity limit, steps around multiples of the exchange
-interval, in place and out of place."""
+thread-block cluster, halos exchanged every E steps through shared / distributed shared
+memory; small configuration K = 12, E = 6 up to 96,768 cells, large K = 28, E = 14 above)
+against the oracle, bit-exact: single warp, several warps, several CTAs of the cluster (DSMEM
+exchanges), both configurations and the switch between them, the capacity limit, steps
+around multiples of both exchange intervals, in place and out of place."""
 import numpy as np
 import pytest
 import torch
@@ -12,8 +13,9 @@ import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
 import sp_inputs
 
 pytestmark = pytest.mark.gpu
-SEG = 64 * 28 - 2 * 14  # owned cells per warp
+SEG = 64 * 12 - 2 * 6  # owned cells per warp (small configuration, n <= 16 x 8 x SEG)
 CTA = 8 * SEG
+SMALL_CAP = 16 * CTA  # above it the large configuration (K = 28, E = 14) runs
 
 
 def _check(got, want):
@@ -26,8 +28,8 @@ def test_capacity():
 
 
 @pytest.mark.parametrize("n", [3, 4, 5, 33, 1000, SEG - 1, SEG, SEG + 1, 4096, CTA - 1, CTA, CTA + 1,
-                               3 * CTA + 17, 8192, 32768])
-@pytest.mark.parametrize("steps", [0, 1, 13, 14, 15, 28, 29, 64, 101])
+                               3 * CTA + 17, 8192, 32768, SMALL_CAP, SMALL_CAP + 1, 150001])
+@pytest.mark.parametrize("steps", [0, 1, 5, 6, 7, 13, 14, 15, 28, 29, 64, 101])
 def test_shapes(n, steps):
     a = sp_inputs.jacobi_input(n, seed=n + steps)
     d = torch.from_numpy(a.copy()).cuda()
@@ -53,7 +55,8 @@ def test_J1_and_long_run_at_capacity():
     torch.cuda.synchronize()
     got = d.cpu().numpy()
     rng = np.random.default_rng(3)
-    idx = [0, 1, 2, n - 3, n - 2, n - 1] + [k * SEG + o for k in (1, 7, 8, 9, 100) for o in (-1, 0, 1) if k * SEG + o < n]
+    seg = 64 * 28 - 2 * 14
+    idx = [0, 1, 2, n - 3, n - 2, n - 1] + [k * seg + o for k in (1, 7, 8, 9, 100) for o in (-1, 0, 1) if k * seg + o < n]
     idx = np.unique(np.array(idx + rng.integers(0, n, 30).tolist(), dtype=np.int64))
     _check(got[idx], oracle.jacobi1d_points(a, 4096, idx))
     with pytest.raises(sp.SPError):
