@@ -113,8 +113,15 @@ struct MeGeom {
     static constexpr int kTailPer = 4 * R / kThreads;    // tail candidates per thread (+ the corner, split)
     static constexpr int kOffCur = 2 * kCopy;            // cur[2] after raw[2]
     static constexpr int kOffPh = 2 * kCopy + 512;       // phase copies (128-byte aligned)
-    static constexpr int kSmem = kOffPh + 6 * kCopy + 3 * 32 + 128;  // + bank offsets + alignment slack
+    // Phase copy slots are kSlot apart and copy ph sits 32*ph bytes into its slot (bank
+    // offsets), so a slot must hold kCopy + 96 bytes: with slots only kCopy apart, the last
+    // 64 bytes of stage 0's phase-3 copy (window row 2R+15, read by the dy = +R tails) were
+    // the first 64 bytes of stage 1's phase-1 copy (row 0), which a warp already building
+    // the next macroblock's copies overwrote — a cross-warp race, rare with balanced warps.
+    static constexpr int kSlot = kCopy + 128;
+    static constexpr int kSmem = kOffPh + 6 * kSlot + 128;  // + alignment slack
     static_assert(kCopy % 128 == 0, "copies must keep 128-byte alignment");
+    static_assert(kSlot >= kCopy + 3 * 32 && kSlot % 128 == 0, "phase copy slots must not overlap");
     static_assert(kWarps == 1 || kWarps == 4, "tail mapping assumes 1 or 4 warps");
     static_assert(kTailPer * kThreads == 4 * R, "tail candidates must spread evenly");
 };
@@ -180,7 +187,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     // byte phase ph of stage st (ph = 0: the TMA'd window).  Copy ph starts 32*ph bytes past
     // a 128-byte boundary, so the four phases a quarter warp reads hit distinct banks.
     auto phase_copy = [&](int st, int ph) -> uint8_t* {
-        return ph == 0 ? smem + st * G::kCopy : smem + G::kOffPh + (3 * st + ph - 1) * G::kCopy + 32 * ph;
+        return ph == 0 ? smem + st * G::kCopy : smem + G::kOffPh + (3 * st + ph - 1) * G::kSlot + 32 * ph;
     };
     struct Pos {
         int pair, byr, bx;
@@ -338,6 +345,10 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         if (tid == G::kThreads - 32 && it > 0) finalize(prev_mb, s ^ 1);
         PMARK(2);
 
+#if SP_ME_EXP & 64  // race stress (tests/test_me_stress_gpu.py): the upper warps start late, so the
+        // lower ones build the next macroblock's copies while these still read this one's
+        if (warp >= nwarps / 2) __nanosleep(20000);
+#endif
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
         //      thread's tail candidates, all in one row loop ----
         uint32_t acc[kTx][kTy];
