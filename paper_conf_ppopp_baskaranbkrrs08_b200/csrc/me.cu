@@ -26,6 +26,7 @@
 #include <cuda_runtime.h>
 
 #include <cstdint>
+#include <cstdlib>
 #include <mutex>
 
 #include "../../include/sp.h"
@@ -640,6 +641,10 @@ int launch_fast(const CUtensorMap& rm, const CUtensorMap& cm, const MeArgs& a, i
         if (err == cudaSuccess)
             err = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, me_sad_kernel<R, kStream>, G::kThreads, G::kSmem);
         grid_cap = sms * (occ > 0 ? occ : 1);
+        // SP_ME_GRID_CAP (sanitizer runs): a few CTAs then walk many macroblocks each, so
+        // racecheck sees both pipeline stages in use within one CTA
+        if (const char* e = std::getenv("SP_ME_GRID_CAP"))
+            if (std::atoi(e) > 0 && std::atoi(e) < grid_cap) grid_cap = std::atoi(e);
     });
     SP_CUDA_TRY(err);
     const int grid = (int)(total < grid_cap ? total : grid_cap);

@@ -1,8 +1,11 @@
 """Small invocations of every device entry point, for compute-sanitizer runs (T6)."""
+import os
 import sys
 
 import torch
 
+# a few ME CTAs walking many macroblocks each: racecheck then sees both pipeline stages of a CTA
+os.environ.setdefault("SP_ME_GRID_CAP", "4")
 sys.path.insert(0, ".")
 import paper_conf_ppopp_baskaranbkrrs08_b200 as sp  # noqa: E402
 import sp_inputs  # noqa: E402
@@ -43,6 +46,11 @@ mark("sp.me_search_sequence_unrestricted")
 sp.me_search_sequence_unrestricted(fr2, 130, 70, 32)
 mark("sp.me_search_host (streamed frames, pinned outputs)")
 sp.MESearchHost(3, 352, 288, fr.shape[2], 16).run(fr.cpu().pin_memory())
+fr3 = torch.from_numpy(sp_inputs.me_sequence(2, 352, 288, 32)).cuda()
+mark("sp.me_search_sequence (CIF +-32: 4-warp CTAs, two stages per CTA)")
+sp.me_search_sequence(fr3, 352, 288, 32)
+mark("sp.me_search_host (CIF +-32, streamed)")
+sp.MESearchHost(2, 352, 288, fr3.shape[2], 32).run(fr3.cpu().pin_memory())
 mark("sp.me_sad_search_direct")
 sp.me_sad_search_direct(fr2[:-1], fr2[1:], 130, 70, 8)
 torch.cuda.synchronize()
