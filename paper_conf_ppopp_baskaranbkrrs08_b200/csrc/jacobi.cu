@@ -871,7 +871,14 @@ int geometry(int32_t time_tile, int32_t space_tile, int64_t& S, int32_t& wo) {
 
 int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v) {
     if (a.tiles <= 0) return SP_OK;
-    const int64_t cap = (int64_t)v.sms * v.occ;
+    // SP_JACOBI_GRID_CAP (sanitizer runs): a few CTAs then take many tiles per warp, so
+    // racecheck sees both stages of every warp's double buffer in use
+    static const int64_t env_cap = [] {
+        const char* e = std::getenv("SP_JACOBI_GRID_CAP");
+        return e ? (int64_t)std::atoll(e) : (int64_t)0;
+    }();
+    int64_t cap = (int64_t)v.sms * v.occ;
+    if (env_cap > 0 && env_cap < cap) cap = env_cap;
     const int grid = (int)(a.tiles < cap ? a.tiles : cap);
     v.kernel<<<grid, v.threads, smem_bytes(v), stream>>>(a);
     SP_CUDA_TRY(cudaGetLastError());

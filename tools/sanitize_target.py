@@ -6,6 +6,7 @@ import torch
 
 # a few ME CTAs walking many macroblocks each: racecheck then sees both pipeline stages of a CTA
 os.environ.setdefault("SP_ME_GRID_CAP", "4")
+os.environ.setdefault("SP_JACOBI_GRID_CAP", "2")  # likewise: many tiles per Jacobi warp
 sys.path.insert(0, ".")
 import paper_conf_ppopp_baskaranbkrrs08_b200 as sp  # noqa: E402
 import sp_inputs  # noqa: E402
@@ -32,6 +33,18 @@ h = a.cpu().pin_memory()
 sp.Jacobi1DHost(4099, 37, 16, 256).run(h)
 mark("sp.jacobi1d_host (1 pass: redirect + copy)")
 sp.Jacobi1DHost(4099, 9, 16, 0).run(h)
+mark("sp.jacobi1d_resident (one cluster, small and large shapes)")
+sp.jacobi1d_resident(a, 45)
+big = torch.from_numpy(sp_inputs.jacobi_input(150000, seed=2)).cuda()
+sp.jacobi1d_resident(big, 33)
+mark("sp.exec_block (Figure 1 program, tiled mat-vec with hoisting)")
+from tests import exec_programs as X  # noqa: E402
+blk, bodies, boxes, printed = X.figure1()
+g = torch.Generator().manual_seed(0)
+sp.exec_block(blk, bodies, [torch.randn(200, 200, generator=g).cuda(), torch.randn(200, 200, generator=g).cuda()])
+blk, bodies, boxes, tiles = X.matvec(70, 100, 16)
+sp.exec_block(blk, bodies, [torch.randn(70, generator=g).cuda(), torch.randn(70, 100, generator=g).cuda(),
+                            torch.randn(100, generator=g).cuda()], tile_params=tiles, tiles_per_cta=7, hoist=True)
 mark("sp.jacobi1d_untiled")
 sp.jacobi1d_untiled(a, 3)
 fr = torch.from_numpy(sp_inputs.me_sequence(3, 352, 288, 16)).cuda()
