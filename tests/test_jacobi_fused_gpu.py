@@ -76,6 +76,22 @@ def test_J3_size_sampled():
     _check(got[idx], oracle.jacobi1d_points(a, steps, idx))
 
 
+def test_J3_every_cell_device_and_host_paths():
+    """BASELINE config 3 in full: all 2^26 cells after T = 1024 steps, from the bench's
+    launch (persistent, Tt = 64, device-resident) and from the end-to-end host-buffer call
+    (wavefront order, pinned in / out), against the untiled oracle (about 10 s of host time
+    on 16 cores)."""
+    n, steps, tt = 1 << 26, 1024, 64
+    a = sp_inputs.jacobi_input(n, seed=2008)
+    got = _run(a, steps, tt)
+    h = torch.from_numpy(a.copy()).pin_memory()
+    sp.Jacobi1DHost(n, steps, tt, 0).run(h)
+    torch.cuda.synchronize()
+    want = oracle.jacobi1d(a, steps)
+    _check(got, want)
+    _check(h.numpy(), want)
+
+
 def test_repeated_calls_reuse_flags():
     n = 100003
     a = sp_inputs.jacobi_input(n, seed=11)

@@ -102,6 +102,26 @@ def test_M4_1080p_sampled():
         assert np.array_equal(sad[p].reshape(-1)[mbs], osad), p
 
 
+def test_M4_1080p_every_macroblock_device_and_host_paths():
+    """BASELINE config 4 in full: every macroblock of all 64 pairs (2,107,814,400 valid
+    candidate SADs) from the bench's launch (device-resident frames) and from the end-to-end
+    host-buffer call (streamed frames, outputs in pinned memory), against the oracle on all
+    of them (about 2 s of host time on 16 cores)."""
+    W, H, R, F = 1920, 1080, 32, 65
+    fr = sp_inputs.me_sequence(F, W, H, R)
+    mv, sad, _ = _gpu(fr, W, H, R)
+    ctx = sp.MESearchHost(F, W, H, fr.shape[2], R)
+    hmv, hsad = ctx.run(torch.from_numpy(fr).pin_memory())
+    torch.cuda.synchronize()
+    hmv, hsad = hmv.numpy(), hsad.numpy().view(np.uint32)
+    for p in range(F - 1):
+        omv, osad, _ = _oracle_pair(fr, p, W, H, R, surface=False)
+        assert np.array_equal(mv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(sad[p].reshape(-1), osad), p
+        assert np.array_equal(hmv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(hsad[p].reshape(-1), osad), p
+
+
 def test_host_api_end_to_end():
     W, H, R = 352, 288, 16
     fr = sp_inputs.me_sequence(4, W, H, R)
