@@ -44,6 +44,11 @@ int sp_last_cuda_error(void);
 int sp_last_nccl_error(void);
 /* Library version, major*10000 + minor*100 + patch. */
 int sp_version(void);
+/* sizeof of every ABI struct, in this order: sp_domain, sp_ref, sp_block, sp_plan_opts,
+ * sp_buffer, sp_jacobi_plan, sp_peer_links, sp_tile_problem, sp_tile_result, sp_op,
+ * sp_stmt_body, sp_array_desc, sp_exec_opts, sp_exec_stats.  Writes min(n, 14) entries and
+ * returns 14 — lets a binding check its struct layouts against the library's. */
+int sp_abi_struct_sizes(int64_t* out, int32_t n);
 
 /* =====================================================================================
  * 1. Planner — the paper's data-management framework for one program block
@@ -101,13 +106,20 @@ typedef struct {
                               buffers' total size exceeds it: SP_ERR_SMEM_LIMIT */
     int64_t max_points;    /* enumeration budget (integer points over all statements);
                               0 = default 2^27; exceeding it: SP_ERR_UNSUPPORTED */
+    int32_t compress;      /* 0: the local array keeps every dimension of the global array
+                              (reading R-P5).  1: §3.1.2 literally — a dimension
+                              that is an affine function of the earlier dimensions on the
+                              partition's data spaces (their affine hull) does not appear in
+                              the local array: n = dim of the hull, size = prod over the kept
+                              dimensions, F' drops the rows of the others (reading R-P8) */
+    int32_t reserved;      /* must be 0 */
 } sp_plan_opts;
 
 /* One local-memory buffer = one partition of an array's data spaces (Alg. 2 output). */
 typedef struct {
     int32_t array;       /* array id */
-    int32_t rank;        /* dimensionality n of the local array (= that of the global
-                            array: every dimension is kept, reading R-P5) */
+    int32_t rank;        /* rank m of the global array; lb / ub / in_* / out_* and the
+                            local access rows are given for all m dimensions (n_dims below) */
     int32_t beneficial;  /* Alg. 1 verdict */
     int32_t n_refs;      /* references in the partition */
     int64_t lb[SP_MAX_RANK]; /* lower bound per dimension = offset g */
@@ -124,6 +136,13 @@ typedef struct {
     int32_t out_dense;       /* out_count == volume of the out bbox */
     int64_t overlap;         /* sum over reference pairs of |D_r ∩ D_r'| (Alg. 1 line 7) */
     int64_t union_count;     /* |union of the partition's data spaces| */
+    int32_t n_dims;          /* dimensionality n of the local array: = rank, or
+                                with compress the dimension of the data spaces' affine hull */
+    int32_t kept_mask;       /* bit k set: global dimension k is a dimension of the local
+                                array.  Dropped dimensions have local extent 1 and local
+                                index 0 (their lb / ub still report the bounding box); the
+                                local array is row-major over the kept dimensions in global
+                                order, size = prod over kept k of (ub_k - lb_k + 1) */
 } sp_buffer;
 
 /* Plan the local buffers of one program block.
@@ -133,7 +152,8 @@ typedef struct {
  *   ref_buf[n_refs] : buffer index of each reference, -1 if not staged (nullable).
  *   local_rows      : sum over refs of rank x (depth + n_params + 1) int64, in ref order:
  *                     the local access function F' - g; unchanged F for
- *                     unstaged refs (nullable).
+ *                     unstaged refs (nullable).  Rows of dimensions a buffer does not keep
+ *                     (compress) are all zero: local index 0 along an extent-1 axis.
  * Empty statement domains are not errors: they yield empty (size-0) data spaces. */
 int sp_plan_buffers(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, int32_t cap_bufs,
                     int32_t* n_bufs, int32_t* ref_buf, int64_t* local_rows);
@@ -492,6 +512,9 @@ typedef struct {
     const int32_t* live_out;     /* [n_arrays] (nullable = all 1): SP_MOVE_DATAFLOW writes back
                                     a final value only for live-out arrays */
     int64_t* move_counts;        /* nullable [n_tiles][n_arrays][2]: elements moved in / out */
+    int32_t compress;            /* planner option (sp_plan_opts.compress): local buffers drop
+                                    affinely dependent dimensions (§3.1.2) */
+    int32_t reserved;            /* must be 0 */
 } sp_exec_opts;
 /* Data movement of a tile (P:L397-405 default; §3.1.4 P:L450-482 optimised):
  *   SP_MOVE_ALL      every element of the read data spaces in, of the write data spaces out;

@@ -25,6 +25,13 @@ points (the method reaches exactly this result, so the plain definition is the o
 6. Algorithm 1 (Cond. (1) P:L333-334, delta P:L344-345): beneficial iff some
    ref has rank(F restricted to iterator columns) < depth of its statement; otherwise
    iff sum over pairs of |D_r ∩ D_r'| > delta * |∪ D_r|      (readings R-P3, R-P4)
+7. compress (§3.1.2; reading R-P8): the local array has the dimensions of the
+   convex hull of the partition's data spaces.  Dimension k is left out when, on the set
+   of points, it is an affine function of the dimensions before it — i.e. when the
+   difference vectors p - p0 (p0 the first point) have the same rank restricted to the
+   first k+1 coordinates as to the first k.  size = prod over the kept k of
+   (ub_k - lb_k + 1); the local access function F' drops the other rows (given as zero
+   rows: local index 0 along an extent-1 axis).
 
 Buffers are listed ordered by (array id, smallest ref index in the partition).
 With reuse_filter, partitions that are not beneficial are not staged: they are not
@@ -140,8 +147,26 @@ def _volume(lb, ub) -> int:
     return v
 
 
+def kept_dims(points: set, rank: int) -> list[int]:
+    """Step 7: the dimensions k whose prefix rank of the difference vectors increases."""
+    pts = sorted(points)
+    if not pts:
+        return []
+    p0 = pts[0]
+    diffs = [[c - c0 for c, c0 in zip(p, p0)] for p in pts[1:]]
+    if not diffs:
+        return []
+    kept, prev = [], 0
+    for k in range(rank):
+        rk = exact_rank([row[:k + 1] for row in diffs])
+        if rk > prev:
+            kept.append(k)
+        prev = rk
+    return kept
+
+
 def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_filter: bool = False,
-                 mup_elems: int = 0) -> dict:
+                 mup_elems: int = 0, compress: bool = False) -> dict:
     """Oracle plan.  block = {"params": [...], "stmts": [{"depth", "rows", "box"}],
     "refs": [{"stmt", "array", "is_write", "rank", "rows"}]}.  Returns
     {"status", "buffers": [...], "ref_buf": [...], "local_rows": [[...]...]}."""
@@ -171,6 +196,11 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
         union = set().union(*[sets[k] for k in ids])
         lb, ub = _bbox(union, rank)
         size = _volume(lb, ub)
+        kept = list(range(rank))
+        if compress:
+            kept = kept_dims(union, rank)
+            if union:
+                size = _volume([lb[k] for k in kept], [ub[k] for k in kept])
         rd = [k for k in ids if not refs[k]["is_write"]]
         wr = [k for k in ids if refs[k]["is_write"]]
         in_set = set().union(*[sets[k] for k in rd]) if rd else set()
@@ -201,6 +231,7 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
             "out_lb": out_lb, "out_ub": out_ub, "out_count": len(out_set),
             "out_dense": int(len(out_set) == _volume(out_lb, out_ub) and len(out_set) > 0),
             "overlap": overlap, "union_count": len(union), "refs": ids,
+            "n_dims": len(kept) if (union or not compress) else 0, "kept": kept,
         }
         if reuse_filter and not beneficial:
             continue
@@ -223,5 +254,7 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
             g = buffers[ref_buf[k]]["lb"]
             for d in range(r["rank"]):
                 F[d][-1] -= g[d]
+                if d not in buffers[ref_buf[k]]["kept"]:
+                    F[d] = [0] * len(F[d])
         local_rows.append(F)
     return {"status": OK, "buffers": buffers, "ref_buf": ref_buf, "local_rows": local_rows}

@@ -68,7 +68,8 @@ class sp_block(ctypes.Structure):
 
 
 class sp_plan_opts(ctypes.Structure):
-    _fields_ = [("mode", i32), ("reuse_filter", i32), ("delta", f64), ("mup_elems", i64), ("max_points", i64)]
+    _fields_ = [("mode", i32), ("reuse_filter", i32), ("delta", f64), ("mup_elems", i64), ("max_points", i64),
+                ("compress", i32), ("reserved", i32)]
 
 
 class sp_buffer(ctypes.Structure):
@@ -76,7 +77,8 @@ class sp_buffer(ctypes.Structure):
                 ("lb", i64 * MAX_RANK), ("ub", i64 * MAX_RANK), ("size", i64), ("v_in_ub", i64), ("v_out_ub", i64),
                 ("in_lb", i64 * MAX_RANK), ("in_ub", i64 * MAX_RANK), ("in_count", i64),
                 ("out_lb", i64 * MAX_RANK), ("out_ub", i64 * MAX_RANK), ("out_count", i64),
-                ("in_dense", i32), ("out_dense", i32), ("overlap", i64), ("union_count", i64)]
+                ("in_dense", i32), ("out_dense", i32), ("overlap", i64), ("union_count", i64),
+                ("n_dims", i32), ("kept_mask", i32)]
 
 
 class sp_jacobi_plan(ctypes.Structure):
@@ -104,7 +106,8 @@ class sp_array_desc(ctypes.Structure):
 class sp_exec_opts(ctypes.Structure):
     _fields_ = [("n_tiles", i32), ("tiles_per_cta", i32), ("tile_params", ctypes.POINTER(i64)), ("hoist", i32),
                 ("reuse_filter", i32), ("max_points", i64), ("movement", i32), ("dry_run", i32),
-                ("live_out", ctypes.POINTER(i32)), ("move_counts", ctypes.POINTER(i64))]
+                ("live_out", ctypes.POINTER(i32)), ("move_counts", ctypes.POINTER(i64)), ("compress", i32),
+                ("reserved", i32)]
 
 
 class sp_exec_stats(ctypes.Structure):
@@ -128,6 +131,7 @@ SYMBOLS = {
     "sp_last_cuda_error": (ctypes.c_int, []),
     "sp_last_nccl_error": (ctypes.c_int, []),
     "sp_version": (ctypes.c_int, []),
+    "sp_abi_struct_sizes": (ctypes.c_int, [ctypes.POINTER(i64), i32]),
     "sp_plan_buffers": (ctypes.c_int, [ctypes.POINTER(sp_block), ctypes.POINTER(sp_plan_opts), ctypes.POINTER(sp_buffer),
                                        i32, ctypes.POINTER(i32), ctypes.POINTER(i32), ctypes.POINTER(i64)]),
     "sp_jacobi1d_plan": (ctypes.c_int, [i64, i32, i32, i32, ctypes.POINTER(sp_jacobi_plan)]),
@@ -246,13 +250,14 @@ def _marshal_block(block: dict, P: int | None = None):
 
 
 def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_filter: bool = False,
-                 mup_elems: int = 0, max_points: int = 0, cap: int = 64) -> dict:
+                 mup_elems: int = 0, max_points: int = 0, cap: int = 64, compress: bool = False) -> dict:
     """sp_plan_buffers on a block given as {"params": [...], "stmts": [{"depth", "rows"}],
     "refs": [{"stmt", "array", "is_write", "rank", "rows"}]} (extra keys ignored)."""
     params = [int(p) for p in block.get("params", [])]
     P = len(params)
     blk, keep = _marshal_block(block)
-    opts = sp_plan_opts(int(mode), int(bool(reuse_filter)), float(delta), int(mup_elems), int(max_points))
+    opts = sp_plan_opts(int(mode), int(bool(reuse_filter)), float(delta), int(mup_elems), int(max_points),
+                        int(bool(compress)), 0)
     n_refs = len(block["refs"])
     ref_buf = (i32 * max(1, n_refs))()
     width = sum(int(r["rank"]) * (int(block["stmts"][int(r["stmt"])]["depth"]) + P + 1) for r in block["refs"])
@@ -276,6 +281,7 @@ def plan_buffers(block: dict, mode: int = PER_ARRAY, delta: float = 0.30, reuse_
             "in_lb": list(b.in_lb[:rk]), "in_ub": list(b.in_ub[:rk]), "in_count": b.in_count, "in_dense": b.in_dense,
             "out_lb": list(b.out_lb[:rk]), "out_ub": list(b.out_ub[:rk]), "out_count": b.out_count,
             "out_dense": b.out_dense, "overlap": b.overlap, "union_count": b.union_count,
+            "n_dims": b.n_dims, "kept": [k for k in range(rk) if (b.kept_mask >> k) & 1],
         })
     if st != 0:
         return out
@@ -298,7 +304,7 @@ MOVE_ALL, MOVE_DATAFLOW = 0, 1
 
 def exec_block(block: dict, bodies: list, arrays: list, tile_params=None, tiles_per_cta: int = 1,
                hoist: bool = True, reuse_filter: bool = False, max_points: int = 0, movement: int = MOVE_ALL,
-               live_out=None, dry_run: bool = False, stream=None) -> dict:
+               live_out=None, dry_run: bool = False, compress: bool = False, stream=None) -> dict:
     """sp_exec_block (staged-tile executor).  arrays: CUDA float32 contiguous
     tensors indexed by array id (updated in place).  bodies[s] = {"write_ref": r, "beta": [...],
     "ops": [(op, arg), ...]} with op in OP_LOAD (arg = ref index), OP_CONST (arg = value),
@@ -331,7 +337,7 @@ def exec_block(block: dict, bodies: list, arrays: list, tile_params=None, tiles_
     lo = None if live_out is None else (i32 * len(arrays))(*[int(bool(v)) for v in live_out])
     counts = (i64 * (2 * n_tiles * len(arrays)))()
     opts = sp_exec_opts(n_tiles, int(tiles_per_cta), tp, int(bool(hoist)), int(bool(reuse_filter)), int(max_points),
-                        int(movement), int(bool(dry_run)), lo, counts)
+                        int(movement), int(bool(dry_run)), lo, counts, int(bool(compress)), 0)
     stats = sp_exec_stats()
     _check(lib.sp_exec_block(ctypes.byref(blk), bl, ad, len(arrays), ctypes.byref(opts), ctypes.byref(stats),
                              None if dry_run else _stream(stream)), "sp_exec_block")

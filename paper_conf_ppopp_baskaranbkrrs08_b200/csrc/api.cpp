@@ -26,3 +26,12 @@ extern "C" const char* sp_status_string(int status) {
 extern "C" int sp_last_cuda_error(void) { return sp::g_cuda_error; }
 extern "C" int sp_last_nccl_error(void) { return sp::g_nccl_error; }
 extern "C" int sp_version(void) { return 100; }
+extern "C" int sp_abi_struct_sizes(int64_t* out, int32_t n) {
+    const int64_t sz[] = {sizeof(sp_domain),      sizeof(sp_ref),         sizeof(sp_block),      sizeof(sp_plan_opts),
+                          sizeof(sp_buffer),      sizeof(sp_jacobi_plan), sizeof(sp_peer_links), sizeof(sp_tile_problem),
+                          sizeof(sp_tile_result), sizeof(sp_op),          sizeof(sp_stmt_body),  sizeof(sp_array_desc),
+                          sizeof(sp_exec_opts),   sizeof(sp_exec_stats)};
+    const int32_t k = (int32_t)(sizeof(sz) / sizeof(sz[0]));
+    for (int32_t i = 0; out && i < n && i < k; ++i) out[i] = sz[i];
+    return k;
+}

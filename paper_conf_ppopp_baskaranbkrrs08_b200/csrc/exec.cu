@@ -154,7 +154,7 @@ struct Compiler {
     TileInfo plan(const int64_t* params) const {
         sp_block b = blk;
         b.params = params;
-        sp_plan_opts po{SP_PLAN_PER_ARRAY, o.reuse_filter, 0.30, 0, o.max_points};
+        sp_plan_opts po{SP_PLAN_PER_ARRAY, o.reuse_filter, 0.30, 0, o.max_points, o.compress, 0};
         TileInfo t;
         int32_t nb = 0;
         t.bufs.resize(std::max(1, n_arrays));
@@ -324,7 +324,7 @@ struct Compiler {
                             int64_t li = 0;
                             for (int k = 0; k < R.rank; ++k) {
                                 const int64_t lc = dot(&TI.local_rows[lr_at[r] + (size_t)k * (d + P + 1)], x, d, params, P);
-                                const int64_t ext = Bf.ub[k] - Bf.lb[k] + 1;
+                                const int64_t ext = ((Bf.kept_mask >> k) & 1) ? Bf.ub[k] - Bf.lb[k] + 1 : 1;
                                 if (lc < 0 || lc >= ext) throw Error{SP_ERR_UNSUPPORTED};  // planner invariant
                                 li = li * ext + lc;
                             }
@@ -401,7 +401,8 @@ struct Compiler {
                         rem /= A.extent[k];
                     }
                     int64_t li = 0;
-                    for (int k = 0; k < A.rank; ++k) li = li * (Bf->ub[k] - Bf->lb[k] + 1) + (c[k] - Bf->lb[k]);
+                    for (int k = 0; k < A.rank; ++k)  // dropped dimensions (§3.1.2): extent 1, index 0
+                        if ((Bf->kept_mask >> k) & 1) li = li * (Bf->ub[k] - Bf->lb[k] + 1) + (c[k] - Bf->lb[k]);
                     moves.push_back(a);
                     moves.push_back((int32_t)gi);
                     moves.push_back((int32_t)(slot_off[a] + li));
@@ -478,6 +479,7 @@ extern "C" int sp_exec_block(const sp_block* blk, const sp_stmt_body* bodies, co
     if (!blk || !bodies || !arrays || n_arrays < 1 || !opts) return SP_ERR_INVALID_ARG;
     if (opts->n_tiles < 1 || opts->tiles_per_cta < 1) return SP_ERR_INVALID_ARG;
     if (opts->movement != SP_MOVE_ALL && opts->movement != SP_MOVE_DATAFLOW) return SP_ERR_INVALID_ARG;
+    if ((opts->compress != 0 && opts->compress != 1) || opts->reserved != 0) return SP_ERR_INVALID_ARG;
     if (blk->n_params > 0 && !opts->tile_params && !(opts->n_tiles == 1 && blk->params)) return SP_ERR_INVALID_ARG;
     for (int a = 0; a < n_arrays; ++a)
         if (arrays[a].rank < 1 || arrays[a].rank > SP_MAX_RANK) return SP_ERR_INVALID_ARG;

@@ -324,12 +324,69 @@ i64 union_count(const std::vector<RefInfo>& R, const std::vector<int>& ids) {
     return (i64)(std::unique(all.begin(), all.end()) - all.begin());
 }
 
+// §3.1.2: the dimensions of the local array are those of the partition's
+// convex hull; a global dimension that is an affine function of the earlier ones on the
+// data spaces (CLooG scans dimensions in order and emits such a dimension as an expression,
+// not a loop) is dropped.  On the affine hull p0 + span{p - p0}, dimension k is an affine
+// function of dimensions 0..k-1 iff the projection of the span onto the first k+1
+// coordinates has the same rank as onto the first k.  Those ranks are read off an echelon
+// basis with leftmost-nonzero pivots (rank of the first k+1 columns = pivots <= k): the kept
+// dimensions are exactly the pivot columns.  Exact integer arithmetic (gcd-normalised).
+struct Echelon {
+    int rank;
+    int n = 0;
+    i128 v[SP_MAX_RANK][SP_MAX_RANK];
+    int piv[SP_MAX_RANK];
+    explicit Echelon(int r) : rank(r) {}
+    bool full() const { return n == rank; }
+    void insert(const i64* d) {
+        i128 x[SP_MAX_RANK];
+        for (int k = 0; k < rank; ++k) x[k] = d[k];
+        for (int b = 0; b < n; ++b) {  // basis kept sorted by pivot column
+            const int c = piv[b];
+            if (x[c] == 0) continue;
+            const i128 xb = x[c], vb = v[b][c];
+            i128 g = 0;
+            for (int k = 0; k < rank; ++k) {
+                x[k] = x[k] * vb - v[b][k] * xb;
+                i128 a = x[k] < 0 ? -x[k] : x[k];
+                for (i128 t = g; t != 0;) {  // g <- gcd(g, a)
+                    const i128 r = a % t;
+                    a = t;
+                    t = r;
+                }
+                g = a;
+            }
+            if (g > 1)
+                for (int k = 0; k < rank; ++k) x[k] /= g;
+        }
+        int c = 0;
+        while (c < rank && x[c] == 0) ++c;
+        if (c == rank) return;
+        int pos = n;
+        while (pos > 0 && piv[pos - 1] > c) {
+            for (int k = 0; k < rank; ++k) v[pos][k] = v[pos - 1][k];
+            piv[pos] = piv[pos - 1];
+            --pos;
+        }
+        for (int k = 0; k < rank; ++k) v[pos][k] = x[k];
+        piv[pos] = c;
+        ++n;
+    }
+    int32_t mask() const {
+        int32_t m = 0;
+        for (int b = 0; b < n; ++b) m |= 1 << piv[b];
+        return m;
+    }
+};
+
 int plan_impl(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, int32_t cap_bufs, int32_t* n_bufs,
               int32_t* ref_buf, int64_t* local_rows) {
     if (!blk || !n_bufs) return SP_ERR_INVALID_ARG;
-    sp_plan_opts o{SP_PLAN_PER_ARRAY, 0, 0.30, 0, 0};
+    sp_plan_opts o{SP_PLAN_PER_ARRAY, 0, 0.30, 0, 0, 0, 0};
     if (opts) o = *opts;
     if (o.mode != SP_PLAN_PER_ARRAY && o.mode != SP_PLAN_COMPONENTS) return SP_ERR_INVALID_ARG;
+    if ((o.compress != 0 && o.compress != 1) || o.reserved != 0) return SP_ERR_INVALID_ARG;
     if (o.mup_elems < 0 || o.max_points < 0 || !(o.delta >= 0.0)) return SP_ERR_INVALID_ARG;
     const i64 max_points = o.max_points ? o.max_points : kDefaultMaxPoints;
     const int P = blk->n_params, S = blk->n_stmts, NR = blk->n_refs;
@@ -501,6 +558,40 @@ int plan_impl(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, in
         b.n_refs = (int32_t)pt.ids.size();
         bbox_of(R, pt.ids, rank, b.lb, b.ub);
         b.size = volume(b.lb, b.ub, rank);  // Alg. 2 step 9
+        b.n_dims = rank;
+        b.kept_mask = (int32_t)((1u << rank) - 1);
+        if (o.compress) {  // §3.1.2: dimensions of the data spaces' affine hull only
+            const Lin& Ln = lin[pt.array_slot];
+            Echelon E(rank);
+            bool have0 = false;
+            i64 p0[SP_MAX_RANK], c[SP_MAX_RANK], dlt[SP_MAX_RANK];
+            for (int id : pt.ids) {
+                for (i64 key : R[id].keys) {
+                    i64 rem = key;
+                    for (int k = 0; k < rank; ++k) {
+                        c[k] = Ln.lo[k] + rem / Ln.stride[k];
+                        rem %= Ln.stride[k];
+                    }
+                    if (!have0) {
+                        std::memcpy(p0, c, sizeof(i64) * rank);
+                        have0 = true;
+                        continue;
+                    }
+                    for (int k = 0; k < rank; ++k) dlt[k] = c[k] - p0[k];
+                    E.insert(dlt);
+                    if (E.full()) break;
+                }
+                if (E.full()) break;
+            }
+            b.n_dims = have0 ? E.n : 0;
+            b.kept_mask = have0 ? E.mask() : 0;
+            if (have0) {
+                i128 sz = 1;
+                for (int k = 0; k < rank; ++k)
+                    if ((b.kept_mask >> k) & 1) sz *= (i128)b.ub[k] - b.lb[k] + 1;
+                b.size = to_i64(sz);
+            }
+        }
         std::vector<int> rd, wr;
         for (int id : pt.ids) (R[id].is_write ? wr : rd).push_back(id);
         bbox_of(R, rd, rank, b.in_lb, b.in_ub);
@@ -565,6 +656,7 @@ int plan_impl(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, in
             for (int j = 0; j < W; ++j) {
                 i64 v = Rf.rows[(size_t)k * W + j];
                 if (j == W - 1 && rb[r] >= 0) v = to_i64((i128)v - out[rb[r]].lb[k]);
+                if (rb[r] >= 0 && !((out[rb[r]].kept_mask >> k) & 1)) v = 0;  // F' drops the row
                 lr.push_back(v);
             }
     }

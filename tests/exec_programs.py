@@ -85,3 +85,19 @@ def pipeline(n):
     bodies = [{"write_ref": 0, "beta": [0, 0], "ops": [(LOAD, 1), (CONST, 2.0), (MUL, 0)]},
               {"write_ref": 2, "beta": [0, 1], "ops": [(LOAD, 3), (CONST, 1.0), (ADD, 0)]}]
     return blk, bodies, [[(0, n - 1)], [(0, n - 1)]]
+
+
+def diagonal(n, t):
+    """d[i] = A[i][i] * 2 + A[i+1][i+1] (i = 0..n-2), tiles I of t: i in [tI, tI+t).
+    Parameter (I).  Both references of A lie on the diagonal, so with §3.1.2 compression
+    the staged buffer of A is 1-D (t+1 elements) instead of the (t+1) x (t+1) box."""
+    dom = [[1, -t, 0], [-1, t, t - 1], [1, 0, 0], [-1, 0, n - 2]]
+    blk = {"params": [0], "stmts": [{"depth": 1, "rows": dom}], "refs": [
+        {"stmt": 0, "array": 0, "is_write": 1, "rank": 1, "rows": [[1, 0, 0]]},                   # d[i]
+        {"stmt": 0, "array": 1, "is_write": 0, "rank": 2, "rows": [[1, 0, 0], [1, 0, 0]]},        # A[i][i]
+        {"stmt": 0, "array": 1, "is_write": 0, "rank": 2, "rows": [[1, 0, 1], [1, 0, 1]]},        # A[i+1][i+1]
+    ]}
+    bodies = [{"write_ref": 0, "beta": [0, 0], "ops": [(LOAD, 1), (CONST, 2.0), (MUL, 0), (LOAD, 2), (ADD, 0)]}]
+    tiles = [[I] for I in range((n - 1 + t - 1) // t)]
+    boxes = [lambda p: [(t * p[0], t * p[0] + t - 1)]]
+    return blk, bodies, boxes, tiles

@@ -114,3 +114,17 @@ def test_dataflow_temporary_stays_on_chip():
     assert np.array_equal(got[2], want[2])  # b = a * 2 + 1
     assert np.all(got[1] == 7.0)            # t was produced and consumed in shared memory only
     assert st["moved_in"] == n and st["moved_out"] == n
+
+
+@pytest.mark.parametrize("compress", [False, True])
+def test_diagonal_compressed_buffers(compress):
+    """§3.1.2 dimension compression (reading R-P8): the A buffer of the diagonal program is
+    staged 1-D; the result is bit-identical to the untransformed program either way."""
+    n, t = 70, 16
+    blk, bodies, boxes, tiles = X.diagonal(n, t)
+    rng = np.random.default_rng(5)
+    arrs = [rng.standard_normal(n).astype(np.float32), rng.standard_normal((n, n)).astype(np.float32)]
+    want = run_block(blk, bodies, arrs, tile_params=tiles, boxes=boxes)
+    got, st = _gpu(arrs, blk, bodies, tile_params=tiles, compress=compress)
+    assert np.array_equal(got[0], want[0]) and np.array_equal(got[1], want[1])
+    assert st["smem_bytes"] == 4 * (t + ((t + 1) if compress else (t + 1) * (t + 1)))

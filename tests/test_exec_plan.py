@@ -53,3 +53,18 @@ def test_dataflow_never_moves_more_than_default():
         b = sp.exec_block(blk, bodies, arrays, tile_params=tiles, movement=sp.MOVE_DATAFLOW, live_out=live,
                           dry_run=True)["move_counts"]
         assert np.all(b <= a), name
+
+
+def test_compressed_buffers_dry_run():
+    """§3.1.2 compression in the executor's compile (reading R-P8): the diagonal program's
+    A buffer is 1-D (t + 1 elements per tile: A[i][i] and A[i+1][i+1] for i in the tile)
+    instead of the (t + 1)^2 box; moves are unchanged (the same elements cross)."""
+    n, t = 40, 8
+    blk, bodies, boxes, tiles = X.diagonal(n, t)
+    arrays = [torch.zeros(n), torch.zeros(n, n)]
+    full = sp.exec_block(blk, bodies, arrays, tile_params=tiles, dry_run=True)
+    comp = sp.exec_block(blk, bodies, arrays, tile_params=tiles, dry_run=True, compress=True)
+    assert full["smem_bytes"] == 4 * (t + (t + 1) * (t + 1))
+    assert comp["smem_bytes"] == 4 * (t + (t + 1))
+    assert comp["moved_in"] == full["moved_in"] and comp["moved_out"] == full["moved_out"]
+    assert np.array_equal(comp["move_counts"], full["move_counts"])

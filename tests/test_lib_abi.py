@@ -70,3 +70,14 @@ def test_device_entry_points_reject_bad_args_without_gpu():
     assert sp.lib.sp_jacobi1d_timetiled(None, None, 10, 1, 16, 0, None, None) == -1
     assert sp.lib.sp_me_sad_search(None, None, 16, 16, 16, 0, 16, 1, 256, 8, 4, 0, 1, None, None, None, None) == -5
     assert sp.lib.sp_me_sad_search(None, None, 16, 16, 16, 0, 16, 1, 256, 16, 4, 0, 1, None, None, None, None) == -1
+
+
+def test_struct_layouts_match_the_library():
+    """The binding's ctypes structs have the C ABI's sizes (sp_abi_struct_sizes)."""
+    order = [sp.sp_domain, sp.sp_ref, sp.sp_block, sp.sp_plan_opts, sp.sp_buffer, sp.sp_jacobi_plan,
+             sp.sp_peer_links, sp.sp_tile_problem, sp.sp_tile_result, sp.sp_op, sp.sp_stmt_body, sp.sp_array_desc,
+             sp.sp_exec_opts, sp.sp_exec_stats]
+    out = (ctypes.c_int64 * len(order))()
+    assert sp.lib.sp_abi_struct_sizes(out, len(order)) == len(order)
+    for cls, n in zip(order, out):
+        assert ctypes.sizeof(cls) == n, (cls.__name__, ctypes.sizeof(cls), n)

@@ -200,3 +200,73 @@ def test_jacobi_tile_footprint_closed_form():
             assert a["lb"] == [max(0, x0 - h)] and a["ub"] == [min(N - 1, x0 + S - 1 + h)], (N, S, h, x0)
             assert b["lb"] == [lo_i] and b["ub"] == [hi_i]
             assert a["beneficial"] == 1  # rank([0,1]) = 1 < depth 2
+
+
+# ---- §3.1.2 dimension compression (reading R-P8), hand-derived -------------
+def _block1(ref_rows, lo=0, hi=9, rank=2, depth=1, extra_refs=()):
+    """One statement over i in [lo, hi] (or (i, j) in [lo, hi]^2 for depth 2), one read ref
+    (plus extra_refs) of array 0."""
+    rows = []
+    for k in range(depth):
+        r = [0] * (depth + 1)
+        r[k], r[-1] = 1, -lo
+        rows.append(r)
+        r = [0] * (depth + 1)
+        r[k], r[-1] = -1, hi
+        rows.append(r)
+    refs = [{"stmt": 0, "array": 0, "is_write": 0, "rank": rank, "rows": ref_rows}]
+    refs += [{"stmt": 0, "array": 0, "is_write": 0, "rank": rank, "rows": rr} for rr in extra_refs]
+    return {"params": [], "stmts": [{"depth": depth, "rows": rows, "box": [[lo, hi]] * depth}], "refs": refs}
+
+
+def test_compress_diagonal():
+    # A[i][i], i = 0..9: the data space is a segment of the diagonal; the second subscript
+    # equals the first, so the local array is 1-D with 10 elements instead of the 10 x 10 box
+    b = P.plan_buffers(_block1([[1, 0], [1, 0]]), compress=True)
+    buf = b["buffers"][0]
+    assert buf["kept"] == [0] and buf["n_dims"] == 1 and buf["size"] == 10
+    assert buf["lb"] == [0, 0] and buf["ub"] == [9, 9]  # the bounding box is still reported
+    assert b["local_rows"][0] == [[1, 0], [0, 0]]  # F' = first row only; g = (0, ...)
+    assert P.plan_buffers(_block1([[1, 0], [1, 0]]))["buffers"][0]["size"] == 100  # R-P5 default
+
+
+def test_compress_affine_second_subscript_and_holes():
+    # A[i][2i + 1]: second subscript an affine function of the first -> 1-D, 10 elements
+    buf = P.plan_buffers(_block1([[1, 0], [2, 1]]), compress=True)["buffers"][0]
+    assert buf["kept"] == [0] and buf["size"] == 10
+    # A[2i][i]: the first subscript runs over 0, 2, ..., 18 and determines the second: kept
+    # dimension 0 with bounds [0, 18] -> 19 elements (the paper's size is the hull's extent,
+    # holes included, P:L364-366)
+    buf = P.plan_buffers(_block1([[2, 0], [1, 0]]), compress=True)["buffers"][0]
+    assert buf["kept"] == [0] and buf["lb"] == [0, 0] and buf["ub"] == [18, 9] and buf["size"] == 19
+
+
+def test_compress_plane_in_3d_and_constant_dimension():
+    # A[i][j][i + j], 0 <= i, j <= 3: a 2-D plane in 3-D; the third subscript is dropped:
+    # 4 x 4 = 16 elements instead of 4 x 4 x 7
+    blk = _block1([[1, 0, 0], [0, 1, 0], [1, 1, 0]], lo=0, hi=3, rank=3, depth=2)
+    buf = P.plan_buffers(blk, compress=True)["buffers"][0]
+    assert buf["kept"] == [0, 1] and buf["n_dims"] == 2 and buf["size"] == 16
+    assert P.plan_buffers(blk)["buffers"][0]["size"] == 4 * 4 * 7
+    # A[5][i]: the constant first subscript is dropped (it is an affine function of no
+    # dimension); the size is the same as the box's (extent 1): 10
+    buf = P.plan_buffers(_block1([[0, 5], [1, 0]]), compress=True)["buffers"][0]
+    assert buf["kept"] == [1] and buf["size"] == 10
+
+
+def test_compress_union_of_two_lines_is_not_compressed():
+    # A[i][i] and A[i][i + 1]: two parallel segments; their affine hull is the plane, so
+    # both dimensions stay: box [0, 9] x [0, 10] = 110 elements
+    blk = _block1([[1, 0], [1, 0]], extra_refs=[[[1, 0], [1, 1]]])
+    buf = P.plan_buffers(blk, compress=True)["buffers"][0]
+    assert buf["kept"] == [0, 1] and buf["size"] == 110
+
+
+def test_compress_single_point_and_dimension_order():
+    # A[3][4] for every i: one point, a 0-dimensional hull -> size 1 (empty product)
+    buf = P.plan_buffers(_block1([[0, 3], [0, 4]]), compress=True)["buffers"][0]
+    assert buf["kept"] == [] and buf["n_dims"] == 0 and buf["size"] == 1
+    # A[i][9 - i]: dimensions are kept in global order, so the FIRST one stays (CLooG scans
+    # the hull's dimensions in order and expresses the later one through it)
+    buf = P.plan_buffers(_block1([[1, 0], [-1, 9]]), compress=True)["buffers"][0]
+    assert buf["kept"] == [0] and buf["size"] == 10

@@ -14,7 +14,8 @@ from oracle import planner as O
 
 GOLD = os.path.join(os.path.dirname(__file__), "golden", "figure1.json")
 FIELDS = ["array", "rank", "beneficial", "n_refs", "lb", "ub", "size", "v_in_ub", "v_out_ub", "in_lb", "in_ub",
-          "in_count", "in_dense", "out_lb", "out_ub", "out_count", "out_dense", "overlap", "union_count"]
+          "in_count", "in_dense", "out_lb", "out_ub", "out_count", "out_dense", "overlap", "union_count",
+          "n_dims", "kept"]
 
 
 def _compare(block, **kw):
@@ -83,7 +84,8 @@ def test_random_blocks(seed):
     for _ in range(25):
         blk = _rand_block(rng)
         mode = rng.choice([O.PER_ARRAY, O.COMPONENTS])
-        _compare(blk, mode=mode, reuse_filter=rng.random() < 0.3, delta=rng.choice([0.3, 0.1, 0.6]))
+        _compare(blk, mode=mode, reuse_filter=rng.random() < 0.3, delta=rng.choice([0.3, 0.1, 0.6]),
+                 compress=rng.random() < 0.5)
 
 
 def test_jacobi_tile_blocks_match_kernel_closed_form():
@@ -183,3 +185,18 @@ def test_capacity_raw_abi():
     assert sp.lib.sp_plan_buffers(None, None, None, 0, ctypes.byref(n), None, None) == -1
     b.reserved = 1
     assert sp.lib.sp_plan_buffers(ctypes.byref(b), None, None, 0, ctypes.byref(n), None, None) == -1
+
+
+@pytest.mark.parametrize("seed", range(12))
+def test_random_blocks_compressed(seed):
+    """§3.1.2 compression on random blocks (rank-deficient accesses are frequent: subscript
+    coefficients in {-1, 0, 1, 2}): kept dimensions, sizes and F' rows equal the oracle's."""
+    rng = random.Random(1000 + seed)
+    dropped = 0
+    for _ in range(25):
+        blk = _rand_block(rng)
+        for mode in (O.PER_ARRAY, O.COMPONENTS):
+            o, _ = _compare(blk, mode=mode, compress=True)
+            if o["status"] == 0:
+                dropped += sum(b["n_dims"] < b["rank"] for b in o["buffers"])
+    assert dropped > 0  # the case is exercised
