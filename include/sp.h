@@ -400,6 +400,11 @@ int sp_ipc_get_handle(const void* ptr, uint8_t out_handle[64]);
 int sp_ipc_open_handle(const uint8_t handle[64], void** ptr);
 int sp_ipc_close_handle(void* ptr);
 
+/* Failure detection: the communicator's asynchronous NCCL state
+ * (ncclCommGetAsyncError; ncclSuccess = 0, ncclInProgress = 7, anything else = the
+ * communicator failed and must be destroyed).  Host call, does not synchronize. */
+int sp_comm_async_error(sp_comm* c, int32_t* nccl_result);
+
 /* ncclAllGather of `bytes` per rank (device buffers) — used for the ME results. */
 int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream);
 

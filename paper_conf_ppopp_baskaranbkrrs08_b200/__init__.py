@@ -153,6 +153,7 @@ SYMBOLS = {
     "sp_jacobi1d_timetiled_loopback": (ctypes.c_int, [ctypes.POINTER(vp), ctypes.POINTER(vp), i32, i64,
                                                       ctypes.POINTER(i64), ctypes.POINTER(i64), i32, i32, i32, vp]),
     "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
+    "sp_comm_async_error": (ctypes.c_int, [vp, ctypes.POINTER(i32)]),
     "sp_jacobi1d_untiled": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_tile_search": (ctypes.c_int, [ctypes.POINTER(sp_tile_problem), ctypes.POINTER(sp_tile_result)]),
     "sp_me_sad_search_unrestricted": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i64, i32, i32, vp, vp, vp, vp]),
@@ -703,6 +704,12 @@ class Comm:
     def allgather(self, send, recv, stream=None):
         nbytes = send.numel() * send.element_size()
         _check(lib.sp_allgather(self.handle, _ptr(send), _ptr(recv), nbytes, _stream(stream)), "sp_allgather")
+
+    def async_error(self) -> int:
+        """ncclCommGetAsyncError of this communicator (0 = healthy, 7 = in progress)."""
+        r = i32(0)
+        _check(lib.sp_comm_async_error(self.handle, ctypes.byref(r)), "sp_comm_async_error")
+        return r.value
 
 
 # ---------------------------------------------------------------------------------------

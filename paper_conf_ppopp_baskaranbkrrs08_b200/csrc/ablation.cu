@@ -91,6 +91,7 @@ __global__ void __launch_bounds__(128) me_direct_kernel(const uint8_t* __restric
 }  // namespace
 
 extern "C" int sp_jacobi1d_untiled(float* a, float* work, int64_t n, int32_t steps, void* stream) {
+    SP_NVTX("sp_jacobi1d_untiled");
     if (!a || !work || a == work || n < 3 || steps < 0) return SP_ERR_INVALID_ARG;
     const cudaStream_t s = (cudaStream_t)stream;
     float* cur = a;
@@ -113,6 +114,7 @@ extern "C" int sp_me_sad_search_direct(const uint8_t* ref, const uint8_t* cur, i
                                        int32_t n_pairs, int64_t pair_stride, int32_t block, int32_t range,
                                        int32_t mb_row_begin, int32_t mb_row_end, int16_t* mv, uint32_t* best_sad,
                                        uint32_t* surface, void* stream) {
+    SP_NVTX("sp_me_sad_search_direct");
     if (block != 16) return SP_ERR_UNSUPPORTED;
     if (!ref || !cur || !mv || !best_sad || range < 0 || range > 63 || width < 16 || frame_height < 16 ||
         n_pairs < 0 || rows_in_buffer < 1 || (pitch & 3) || pitch < width || (reinterpret_cast<uintptr_t>(ref) & 3) ||

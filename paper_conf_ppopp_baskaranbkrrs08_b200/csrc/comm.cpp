@@ -41,6 +41,7 @@ struct Nccl {
     ncclResult_t (*GroupStart)() = nullptr;
     ncclResult_t (*GroupEnd)() = nullptr;
     ncclResult_t (*AllGather)(const void*, void*, size_t, ncclDataType_t, ncclComm_t, cudaStream_t) = nullptr;
+    ncclResult_t (*CommGetAsyncError)(ncclComm_t, ncclResult_t*) = nullptr;
 };
 
 Nccl& nccl() {
@@ -61,6 +62,7 @@ Nccl& nccl() {
         SP_SYM(GroupStart, "ncclGroupStart");
         SP_SYM(GroupEnd, "ncclGroupEnd");
         SP_SYM(AllGather, "ncclAllGather");
+        SP_SYM(CommGetAsyncError, "ncclCommGetAsyncError");
 #undef SP_SYM
         n.ok = n.GetUniqueId && n.CommInitRank && n.CommDestroy && n.Send && n.Recv && n.GroupStart && n.GroupEnd &&
                n.AllGather;
@@ -100,7 +102,10 @@ int pass_loop(std::vector<Slab>& slabs, int64_t n_global, int32_t steps, int32_t
     int st;
     for (int32_t done = 0; done < steps; done += tt) {
         const int32_t h = steps - done < tt ? steps - done : tt;
-        if ((st = exchange(cur))) return st;
+        {
+            SP_NVTX("halo exchange");
+            if ((st = exchange(cur))) return st;
+        }
         for (size_t r = 0; r < slabs.size(); ++r) {
             const Slab& s = slabs[r];
             const int64_t g0 = s.x_begin - H;
@@ -184,6 +189,7 @@ extern "C" int sp_comm_destroy(sp_comm* c) {
 extern "C" int sp_jacobi1d_timetiled_dist(sp_comm* c, float* a_local, float* work_local, int64_t n_global,
                                           int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
                                           int32_t space_tile, void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled_dist");
     if (!c) return SP_ERR_INVALID_ARG;
     int st = check_slab(n_global, x_begin, n_local, time_tile, a_local, work_local);
     if (st) return st;
@@ -213,7 +219,21 @@ extern "C" int sp_jacobi1d_timetiled_dist(sp_comm* c, float* a_local, float* wor
     });
 }
 
+extern "C" int sp_comm_async_error(sp_comm* c, int32_t* nccl_result) {
+    if (!c || !nccl_result) return SP_ERR_INVALID_ARG;
+    Nccl& n = nccl();
+    if (!n.ok || !n.CommGetAsyncError) {
+        sp::set_nccl_error((int)ncclSystemError);
+        return SP_ERR_NCCL;
+    }
+    ncclResult_t r = ncclSuccess;
+    SP_NCCL_TRY(n.CommGetAsyncError(c->comm, &r));
+    *nccl_result = (int32_t)r;
+    return SP_OK;
+}
+
 extern "C" int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream) {
+    SP_NVTX("sp_allgather");
     if (!c || !send || !recv || bytes < 0) return SP_ERR_INVALID_ARG;
     Nccl& n = nccl();
     SP_NCCL_TRY(n.AllGather(send, recv, (size_t)bytes, ncclUint8, c->comm, (cudaStream_t)stream));
@@ -226,6 +246,7 @@ extern "C" int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t by
 extern "C" int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_locals, int32_t nranks, int64_t n_global,
                                               const int64_t* x_begins, const int64_t* n_locals, int32_t steps,
                                               int32_t time_tile, int32_t space_tile, void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled_loopback");
     if (!a_locals || !work_locals || !x_begins || !n_locals || nranks < 1) return SP_ERR_INVALID_ARG;
     const int32_t H = halo_of(time_tile);
     std::vector<Slab> slabs;

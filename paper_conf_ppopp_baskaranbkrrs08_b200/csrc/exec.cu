@@ -476,6 +476,7 @@ int upload(const std::vector<T>& v, void** dev, cudaStream_t s) {
 
 extern "C" int sp_exec_block(const sp_block* blk, const sp_stmt_body* bodies, const sp_array_desc* arrays,
                              int32_t n_arrays, const sp_exec_opts* opts, sp_exec_stats* stats, void* stream) {
+    SP_NVTX("sp_exec_block");
     if (!blk || !bodies || !arrays || n_arrays < 1 || !opts) return SP_ERR_INVALID_ARG;
     if (opts->n_tiles < 1 || opts->tiles_per_cta < 1) return SP_ERR_INVALID_ARG;
     if (opts->movement != SP_MOVE_ALL && opts->movement != SP_MOVE_DATAFLOW) return SP_ERR_INVALID_ARG;

@@ -1028,6 +1028,7 @@ extern "C" int sp_jacobi1d_pass_segment(const float* src, float* dst, int64_t n_
 
 extern "C" int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32_t time_tile,
                                      int32_t space_tile, int64_t* footprint_log, void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled");
     if (!a || !work || n < 3 || steps < 0 || a == work) return SP_ERR_INVALID_ARG;
     if ((reinterpret_cast<uintptr_t>(a) & 15) || (reinterpret_cast<uintptr_t>(work) & 15)) return SP_ERR_INVALID_ARG;
     int64_t S;
@@ -1092,6 +1093,7 @@ int device_view(const void* p, const void** out) {
 extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float* buf1, int32_t* flags,
                                             int64_t flags_len, int64_t n, int32_t steps, int32_t time_tile,
                                             int32_t space_tile, int64_t skew, int64_t* footprint_log, void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled_stream");
     if (!in || !out || !buf0 || !buf1 || !flags || n < 3 || steps < 0 || buf0 == buf1 || in == buf1)
         return SP_ERR_INVALID_ARG;
     for (const void* q : {(const void*)in, (const void*)out, (const void*)buf0, (const void*)buf1})
@@ -1171,6 +1173,7 @@ __global__ void peer_done_kernel(unsigned long long* left_done, unsigned long lo
 extern "C" int sp_jacobi1d_timetiled_peer(const sp_peer_links* L, float* a_local, float* work_local, int64_t n_global,
                                           int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
                                           int32_t space_tile, void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled_peer");
     if (!L || !a_local || !work_local || a_local == work_local || n_global < 3 || x_begin < 0 || n_local < 1 ||
         x_begin + n_local > n_global || steps < 0 || (x_begin & 3) || !L->my_flags)
         return SP_ERR_INVALID_ARG;
@@ -1328,6 +1331,7 @@ extern "C" int sp_jacobi1d_resident_capacity(int64_t* max_cells) {
 }
 
 extern "C" int sp_jacobi1d_resident(const float* in, float* out, int64_t n, int32_t steps, void* stream) {
+    SP_NVTX("sp_jacobi1d_resident");
     if (!in || !out || n < 3 || steps < 0) return SP_ERR_INVALID_ARG;
     cudaError_t e = cudaSuccess;
     const int64_t cap_s = ResidentSmall::capacity(e);

@@ -731,6 +731,7 @@ extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t 
                                 int32_t rows_in_buffer, int32_t row0_global, int32_t frame_height, int32_t n_pairs,
                                 int64_t pair_stride, int32_t block, int32_t range, int32_t mb_row_begin,
                                 int32_t mb_row_end, int16_t* mv, uint32_t* best_sad, uint32_t* surface, void* stream) {
+    SP_NVTX("sp_me_sad_search");
     return me_search_impl(ref, cur, pitch, width, rows_in_buffer, row0_global, frame_height, n_pairs, pair_stride,
                           block, range, mb_row_begin, mb_row_end, mv, best_sad, surface, stream, 0);
 }
@@ -739,6 +740,7 @@ extern "C" int sp_me_sad_search_unrestricted(const uint8_t* ref_padded, const ui
                                              int32_t width, int32_t height, int32_t pad, int32_t n_pairs,
                                              int64_t pair_stride, int32_t block, int32_t range, int16_t* mv,
                                              uint32_t* best_sad, uint32_t* surface, void* stream) {
+    SP_NVTX("sp_me_sad_search_unrestricted");
     if (range < 0 || pad < range || (fast_range(range) && (pad % 16)) || pad < 1) return SP_ERR_INVALID_ARG;
     return me_search_impl(ref_padded, cur_padded, pitch, width, height + 2 * pad, 0, height, n_pairs, pair_stride,
                           block, range, 0, height / kMB, mv, best_sad, surface, stream, pad);
@@ -789,6 +791,7 @@ cudaStream_t own_copy_stream() {  // per process; used when the caller passes no
 extern "C" int sp_me_search_host(const uint8_t* frames_host, int64_t pitch, int32_t width, int32_t height,
                                  int32_t n_frames, int32_t range, uint8_t* frames_dev, int32_t* ready, int16_t* mv,
                                  uint32_t* best_sad, void* stream, void* copy_stream) {
+    SP_NVTX("sp_me_search_host");
     if (!frames_host || !frames_dev || !ready || !mv || !best_sad || n_frames < 1 || height < kMB || width < kMB)
         return SP_ERR_INVALID_ARG;
     if (!fast_range(range)) return SP_ERR_UNSUPPORTED;

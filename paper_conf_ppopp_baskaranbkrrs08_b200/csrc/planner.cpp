@@ -671,6 +671,7 @@ int plan_impl(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, in
 
 extern "C" int sp_plan_buffers(const sp_block* blk, const sp_plan_opts* opts, sp_buffer* bufs, int32_t cap_bufs,
                                int32_t* n_bufs, int32_t* ref_buf, int64_t* local_rows) {
+    SP_NVTX("sp_plan_buffers");
     try {
         return plan_impl(blk, opts, bufs, cap_bufs, n_bufs, ref_buf, local_rows);
     } catch (const PlanError& e) {
@@ -786,6 +787,7 @@ int tile_search_impl(const sp_tile_problem* pb, sp_tile_result* out) {
 }  // namespace
 
 extern "C" int sp_tile_search(const sp_tile_problem* prob, sp_tile_result* out) {
+    SP_NVTX("sp_tile_search");
     try {
         return tile_search_impl(prob, out);
     } catch (const PlanError& e) {

@@ -3,6 +3,8 @@
 #include <cstdint>
 #include <vector>
 
+#include <nvtx3/nvToolsExt.h>
+
 #include "../../include/sp.h"
 
 namespace sp {
@@ -24,3 +26,15 @@ void set_nccl_error(int e);
             return SP_ERR_CUDA;                           \
         }                                                 \
     } while (0)
+
+// NVTX range over an entry point (SURVEY §5 tracing): visible to ncu (--nvtx) and nsys;
+// header-only NVTX v3, a no-op unless a tool is attached.
+namespace sp {
+struct NvtxRange {
+    explicit NvtxRange(const char* name) { nvtxRangePushA(name); }
+    ~NvtxRange() { nvtxRangePop(); }
+    NvtxRange(const NvtxRange&) = delete;
+    NvtxRange& operator=(const NvtxRange&) = delete;
+};
+}  // namespace sp
+#define SP_NVTX(name) const sp::NvtxRange sp_nvtx_range_(name)

@@ -222,5 +222,6 @@ def test_dist_path_single_rank_nccl():
         comm.allgather(src, dst)
         torch.cuda.synchronize()
         assert torch.equal(src, dst)
+        assert comm.async_error() == 0  # failure detection: a healthy communicator
     finally:
         comm.destroy()

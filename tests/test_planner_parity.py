@@ -78,7 +78,7 @@ def _rand_block(rng: random.Random):
     return {"params": params, "stmts": stmts, "refs": refs}
 
 
-@pytest.mark.parametrize("seed", range(12))
+@pytest.mark.parametrize("seed", range(40))
 def test_random_blocks(seed):
     rng = random.Random(1000 + seed)
     for _ in range(25):
