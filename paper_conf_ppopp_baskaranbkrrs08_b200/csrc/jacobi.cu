@@ -799,7 +799,7 @@ Variant make_variant() {
 
 constexpr int kNumVariants = 11;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
-constexpr int64_t kDefaultSkew = 1024;  // wavefront order: tiles between consecutive passes (host path sweep: 256 -> 9.6 ms, 1024 -> 8.9, 2048 -> 10.3 on J3)
+constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
 Variant* variants() {
     static Variant v[kNumVariants] = {
