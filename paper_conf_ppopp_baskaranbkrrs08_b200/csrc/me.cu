@@ -306,7 +306,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         if (tid == 0) mbS[s ^ 1] = atomicAdd(A.counter, 1u) + Gs;
         mbar_wait(&full[s], (it >> 1) & 1);
         PMARK(0);
-        {   // byte-phase copies (word q of copy p = bytes [4q+p, 4q+p+4) of the row):
+        if (!(SP_ME_EXP & 128)) {  // (128: timing-only build without the phase build)
+            // byte-phase copies (word q of copy p = bytes [4q+p, 4q+p+4) of the row):
             // (row, phase) units spread over the CTA, one window row loaded per unit
             constexpr int v4_per_row = win / 16;
             const uint8_t* raw = smem + s * G::kCopy;
