@@ -392,6 +392,18 @@ typedef struct {
 int sp_jacobi1d_timetiled_peer(const sp_peer_links* links, float* a_local, float* work_local, int64_t n_global,
                                int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
                                int32_t space_tile, void* stream);
+/* The same computation in ONE persistent launch per call (no kernel boundary between
+ * passes; B200-native form of §8(e)): tiles are ordered by completion flags as in
+ * sp_jacobi1d_timetiled_fused, and the halo exchange happens at tile granularity — a slab's
+ * edge tiles of pass p wait for the neighbour's epoch (epoch0 + 1 + p) and the last edge
+ * tile of each side pushes the new edge cells into the neighbour's buffer and raises its
+ * flag, while the interior tiles run on.  flags: device int32 [flags_len >= tiles + 1 +
+ * 2 * passes] (tiles = ceil(n_local / space tile)), zeroed by the call; same links, buffer
+ * layout and epoch protocol as sp_jacobi1d_timetiled_peer (advance epoch0 by the pass count
+ * between calls).  All ranks of a run must use the same entry point. */
+int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* links, float* a_local, float* work_local, int32_t* flags,
+                                     int64_t flags_len, int64_t n_global, int64_t x_begin, int64_t n_local,
+                                     int32_t steps, int32_t time_tile, int32_t space_tile, void* stream);
 
 /* Exportable device allocations and CUDA-IPC handles (64 bytes) for the peer path. */
 int sp_device_alloc(void** ptr, int64_t bytes); /* cudaMalloc + zero fill */

@@ -160,6 +160,8 @@ SYMBOLS = {
     "sp_me_pad_frames": (ctypes.c_int, [vp, i64, i64, i32, i32, i32, i32, vp, i64, i64, vp]),
     "sp_jacobi1d_timetiled_peer": (ctypes.c_int, [ctypes.POINTER(sp_peer_links), vp, vp, i64, i64, i64, i32, i32, i32,
                                                   vp]),
+    "sp_jacobi1d_timetiled_peer_fused": (ctypes.c_int, [ctypes.POINTER(sp_peer_links), vp, vp, vp, i64, i64, i64, i64,
+                                                        i32, i32, i32, vp]),
     "sp_device_alloc": (ctypes.c_int, [ctypes.POINTER(vp), i64]),
     "sp_device_free": (ctypes.c_int, [vp]),
     "sp_ipc_get_handle": (ctypes.c_int, [vp, ctypes.POINTER(ctypes.c_uint8)]),
@@ -731,11 +733,15 @@ class PeerSlab:
     GPUs; the same code runs between processes sharing one GPU).  `a` is a torch view of the
     rank's [x_begin - H, x_end + H) buffer."""
 
-    def __init__(self, n_global: int, x_begin: int, n_local: int, time_tile: int, space_tile: int = 0):
+    def __init__(self, n_global: int, x_begin: int, n_local: int, time_tile: int, space_tile: int = 0,
+                 fused: bool = False):
+        """fused: one persistent launch per call with tile-granular halo exchange
+        (sp_jacobi1d_timetiled_peer_fused); every rank of a run must pass the same value."""
         import torch
         import torch.distributed as dist
         self.n_global, self.x_begin, self.n_local = int(n_global), int(x_begin), int(n_local)
-        self.time_tile, self.space_tile = int(time_tile), int(space_tile)
+        self.time_tile, self.space_tile, self.fused = int(time_tile), int(space_tile), bool(fused)
+        self._flags = None
         self.H = halo_of(time_tile)
         cells = self.n_local + 2 * self.H
         self._own = []
@@ -781,11 +787,25 @@ class PeerSlab:
         dist.barrier()
 
     def run(self, steps: int, stream=None):
-        """sp_jacobi1d_timetiled_peer over this slab; advances the epoch base."""
-        _check(lib.sp_jacobi1d_timetiled_peer(ctypes.byref(self.links), vp(self.a_ptr), vp(self.w_ptr),
-                                              self.n_global, self.x_begin, self.n_local, int(steps), self.time_tile,
-                                              self.space_tile, _stream(stream)), "sp_jacobi1d_timetiled_peer")
-        self.links.epoch0 += (int(steps) + self.time_tile - 1) // self.time_tile
+        """sp_jacobi1d_timetiled_peer(_fused) over this slab; advances the epoch base."""
+        import torch
+        passes = (int(steps) + self.time_tile - 1) // self.time_tile
+        if self.fused:
+            tiles = jacobi1d_plan(self.n_local, max(1, int(steps)), self.time_tile, self.space_tile)["tiles"]
+            need = tiles + 1 + 2 * passes
+            if self._flags is None or self._flags.numel() < need:
+                self._flags = torch.empty(need, dtype=torch.int32, device="cuda")
+            _check(lib.sp_jacobi1d_timetiled_peer_fused(ctypes.byref(self.links), vp(self.a_ptr), vp(self.w_ptr),
+                                                        _ptr(self._flags), self._flags.numel(), self.n_global,
+                                                        self.x_begin, self.n_local, int(steps), self.time_tile,
+                                                        self.space_tile, _stream(stream)),
+                   "sp_jacobi1d_timetiled_peer_fused")
+        else:
+            _check(lib.sp_jacobi1d_timetiled_peer(ctypes.byref(self.links), vp(self.a_ptr), vp(self.w_ptr),
+                                                  self.n_global, self.x_begin, self.n_local, int(steps),
+                                                  self.time_tile, self.space_tile, _stream(stream)),
+                   "sp_jacobi1d_timetiled_peer")
+        self.links.epoch0 += passes
 
     def close(self):
         import torch

@@ -110,6 +110,19 @@ struct PassArgs {
     const float* in0;
     float* outL;
     int64_t skew;
+    // Persistent mode across GPUs (sp_jacobi1d_timetiled_peer_fused; null otherwise): the
+    // halo of pass p arrives in bufs[p & 1] with epoch `epoch + p` on wait_left / wait_right
+    // (pass 0: the push at kernel start above).  Edge tiles (those that produce one of the
+    // first / last H owned cells — exactly the tiles that read the halo) count their
+    // completion per side and pass in edge_cnt; the last one of pass p pushes the new edge
+    // cells (bufs[(p + 1) & 1]) into pushL / pushR[(p + 1) & 1] and raises the neighbour's
+    // flag to epoch + p + 1.  The neighbour read the halo it overwrites in its pass p - 1
+    // edge tiles, which finished before its own push that this rank's pass p edge tiles
+    // waited for, so no extra handshake is needed.
+    float* pushL[2];
+    float* pushR[2];
+    int* edge_cnt;  // [2][passes]
+    int32_t nE_left, nE_right;
 };
 
 // Spin (acquire, system scope) until *flag >= e.  A peer that never arrives (crashed rank,
@@ -429,7 +442,10 @@ __device__ __forceinline__ void run_steps_se(uint64_t (&P)[kK], int h, int lane,
 //   move-out (H7): owned cells [x0, x0+S) registers -> shared -> 1-D TMA bulk store.
 // No CTA-wide barrier anywhere: warps drift freely, so one warp's transfers overlap the
 // other warps' arithmetic.
-template <class Cfg>
+// kPeer: the instantiation with the persistent multi-GPU halo exchange (PassArgs::pushL);
+// the single-GPU launches use the one without it (its code would cost the common path
+// registers: 6.89 -> 6.96 ms on J3 when compiled in).
+template <class Cfg, bool kPeer = false>
 __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_kernel(PassArgs A) {
     constexpr int kK = Cfg::K, kStrip = Cfg::kStrip;
     extern __shared__ __align__(128) float smem[];
@@ -469,7 +485,22 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     const int64_t reach = (A.H + A.S - 1) / A.S;
     // Warp-uniform (every lane calls it): lane-divergent polling loops would leave the warp
     // split through the step loop that follows (measured: 1.7x the instructions issued).
+    // persistent multi-GPU mode: the neighbour's halo for this pass has arrived (every lane
+    // loads the same flag: warp-uniform)
+    const bool peer = kPeer && pers && (A.wait_left || A.wait_right);
+    auto peer_ready = [&](int64_t t, int pass) -> bool {
+        if (!peer) return true;
+        int64_t x0, st, lo, hi;
+        tile_range(t, x0, st, lo, hi);
+        const unsigned long long e = A.epoch + (unsigned long long)pass;
+        if (A.wait_left && lo < A.own_begin && ld_acquire_sys(A.wait_left) < e) return false;
+        if (A.wait_right && hi > A.own_end && ld_acquire_sys(A.wait_right) < e) return false;
+        return true;
+    };
     auto deps_ready = [&](int64_t t, int pass) -> bool {
+        if constexpr (kPeer) {
+            if (pers && !peer_ready(t, pass)) return false;
+        }
         if (!pers || pass == 0) return true;
         bool ok = true;
         for (int64_t q0 = t - reach; q0 <= t + reach; q0 += 32) {
@@ -495,12 +526,13 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         int64_t x0, st, lo, hi;
         tile_range(t, x0, st, lo, hi);
         if (pers) fence_proxy_async_global();  // observed flags -> the async-proxy read below
+        const unsigned long long ep = kPeer && pers ? A.epoch + (unsigned long long)pass : A.epoch;
         if (A.wait_left && lo < A.own_begin) {   // halo from the left neighbour (peer store)
-            wait_epoch(A.wait_left, A.epoch);
+            wait_epoch(A.wait_left, ep);
             fence_proxy_async_global();
         }
         if (A.wait_right && hi > A.own_end) {
-            wait_epoch(A.wait_right, A.epoch);
+            wait_epoch(A.wait_right, ep);
             fence_proxy_async_global();
         }
         const uint32_t bytes = (uint32_t)(((hi - lo) & ~int64_t(3)) * 4);
@@ -678,7 +710,9 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         // for and published at once.
         if (lane == 0 && pers) publish(A.skew != 0);
         if (u_next < total) {
-            pending = (pers && pn > 0 && 2 * reach < 32) ? !__all_sync(0xffffffffu, next_flag >= pn) : !deps_ready(tn, pn);
+            pending = (pers && pn > 0 && 2 * reach < 32)
+                          ? (!__all_sync(0xffffffffu, next_flag >= pn) || (kPeer && !peer_ready(tn, pn)))
+                          : !deps_ready(tn, pn);
             if (lane == 0) {
                 bulk_wait_read0();
                 if (!pending) issue(tn, pn, s ^ 1);
@@ -769,6 +803,32 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             pub_t[k] = t;
             pub_pass[k] = pass;
         }
+        if constexpr (kPeer) if (pers && (A.pushL[0] || A.pushR[0]) && pass + 1 < A.passes) {
+            // multi-GPU: the last edge tile of this pass on a side pushes the new edge cells
+            const bool eL = A.pushL[0] && x0 < A.own_begin + A.H;
+            const bool eR = A.pushR[0] && x0 + st > A.own_end - A.H;
+            if (eL || eR) {  // warp-uniform
+                if (lane == 0) {
+                    bulk_wait0();  // this tile's cells are in global memory ...
+                    fence_proxy_async_global();  // ... and ordered before the release below
+                }
+                __syncwarp();
+                for (int side = 0; side < 2; ++side) {
+                    if (!(side == 0 ? eL : eR)) continue;
+                    int c = 0;
+                    if (lane == 0) c = atom_add_acq_rel_gpu(A.edge_cnt + (int64_t)side * A.passes + pass, 1) + 1;
+                    c = __shfl_sync(0xffffffffu, c, 0);
+                    if (c != (side == 0 ? A.nE_left : A.nE_right)) continue;
+                    const float* sb = A.bufs[(pass + 1) & 1];
+                    float* db = side == 0 ? A.pushL[(pass + 1) & 1] : A.pushR[(pass + 1) & 1];
+                    const int64_t first = side == 0 ? A.own_begin : A.own_end - A.H;
+                    for (int i = lane; i < A.H; i += 32) db[i] = __ldcg(sb + (first + i - A.g0));
+                    __threadfence_system();
+                    __syncwarp();
+                    if (lane == 0) st_release_sys(side == 0 ? A.signal_left : A.signal_right, A.epoch + pass + 1);
+                }
+            }
+        }
         u = u_next;
     }
     if (lane == 0) {
@@ -781,7 +841,8 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 struct Variant {
     int K, warps, threads, strip, stage_floats;
     void (*kernel)(PassArgs);
-    int sms = 0, occ = 0;
+    void (*kernel_peer)(PassArgs) = nullptr;  // kPeer instantiation (default variant only)
+    int sms = 0, occ = 0, occ_peer = 0;
     bool ok = false;
 };
 
@@ -796,6 +857,12 @@ Variant make_variant() {
     v.kernel = jacobi1d_pass_kernel<Cfg>;
     return v;
 }
+template <class Cfg>
+Variant make_variant_peer() {
+    Variant v = make_variant<Cfg>();
+    v.kernel_peer = jacobi1d_pass_kernel<Cfg, true>;
+    return v;
+}
 
 constexpr int kNumVariants = 11;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
@@ -808,7 +875,7 @@ Variant* variants() {
         make_variant<JCfg<20, 4, 4>>(),  // 2: 40 cells/lane, <= 128 regs
         make_variant<JCfg<28, 4, 4>>(),  // 3: 56 cells/lane, <= 128 regs
         make_variant<JCfg<20, 2, 8>>(),  // 4: 40 cells/lane, 2 warps/CTA, <= 128 regs
-        make_variant<JCfg<28, 8, 2>>(),  // 5: 56 cells/lane, 8 warps/CTA (224 KB of stages per SM)
+        make_variant_peer<JCfg<28, 8, 2>>(),  // 5: 56 cells/lane, 8 warps/CTA (224 KB of stages per SM)
         make_variant<JCfg<28, 8, 2, true>>(),  // 6: as 5, scalar edge cells
         make_variant<JCfg<52, 8, 1, true>>(),  // 7: 104 cells/lane, scalar edges, 8 warps/SM (208 KB of stages)
         make_variant<JCfg<44, 8, 1, true>>(),  // 8: 88 cells/lane, scalar edges, 8 warps/SM
@@ -844,6 +911,12 @@ int device_info(Variant& out) {
         SP_CUDA_TRY(cudaFuncSetAttribute(d.kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes(d)));
         SP_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&d.occ, d.kernel, d.threads, smem_bytes(d)));
         if (d.occ < 1) d.occ = 1;
+        if (d.kernel_peer) {
+            SP_CUDA_TRY(cudaFuncSetAttribute(d.kernel_peer, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes(d)));
+            SP_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&d.occ_peer, d.kernel_peer, d.threads,
+                                                                      smem_bytes(d)));
+            if (d.occ_peer < 1) d.occ_peer = 1;
+        }
         d.ok = true;
     }
     out = d;
@@ -869,7 +942,8 @@ int geometry(int32_t time_tile, int32_t space_tile, int64_t& S, int32_t& wo) {
     return SP_OK;
 }
 
-int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v) {
+int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v, bool peer = false) {
+    if (peer && !v.kernel_peer) return SP_ERR_UNSUPPORTED;  // (SP_JACOBI_VARIANT other than the default)
     if (a.tiles <= 0) return SP_OK;
     // SP_JACOBI_GRID_CAP (sanitizer runs): a few CTAs then take many tiles per warp, so
     // racecheck sees both stages of every warp's double buffer in use
@@ -877,10 +951,10 @@ int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v) {
         const char* e = std::getenv("SP_JACOBI_GRID_CAP");
         return e ? (int64_t)std::atoll(e) : (int64_t)0;
     }();
-    int64_t cap = (int64_t)v.sms * v.occ;
+    int64_t cap = (int64_t)v.sms * (peer ? v.occ_peer : v.occ);
     if (env_cap > 0 && env_cap < cap) cap = env_cap;
     const int grid = (int)(a.tiles < cap ? a.tiles : cap);
-    v.kernel<<<grid, v.threads, smem_bytes(v), stream>>>(a);
+    (peer ? v.kernel_peer : v.kernel)<<<grid, v.threads, smem_bytes(v), stream>>>(a);
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }
@@ -1218,6 +1292,78 @@ extern "C" int sp_jacobi1d_timetiled_peer(const sp_peer_links* L, float* a_local
     // tell the neighbours this rank is done with every buffer of this call
     peer_done_kernel<<<1, 1, 0, s>>>(has_left ? L->left_flags + 3 : nullptr, has_right ? L->right_flags + 2 : nullptr,
                                      (unsigned long long)(L->epoch0 + (uint64_t)pass));
+    SP_CUDA_TRY(cudaGetLastError());
+    return SP_OK;
+}
+
+// Multi-GPU time-tiled Jacobi in ONE persistent launch per call: the pass loop of
+// sp_jacobi1d_timetiled_peer without kernel boundaries.  Tiles are ordered by the per-tile
+// completion flags as in sp_jacobi1d_timetiled_fused; the halo exchange happens at tile
+// granularity (see PassArgs::pushL): a slab's edge tiles of pass p wait for the neighbour's
+// pass p - 1 edge cells, and push their own as soon as the last of them completes, while the
+// interior tiles run on.  flags: tiles + 1 + 2 * passes int32 (device; zeroed here).
+extern "C" int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* L, float* a_local, float* work_local,
+                                                int32_t* flags, int64_t flags_len, int64_t n_global, int64_t x_begin,
+                                                int64_t n_local, int32_t steps, int32_t time_tile, int32_t space_tile,
+                                                void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled_peer_fused");
+    if (!L || !a_local || !work_local || !flags || a_local == work_local || n_global < 3 || x_begin < 0 ||
+        n_local < 1 || x_begin + n_local > n_global || steps < 0 || (x_begin & 3) || !L->my_flags)
+        return SP_ERR_INVALID_ARG;
+    if ((reinterpret_cast<uintptr_t>(a_local) & 15) || (reinterpret_cast<uintptr_t>(work_local) & 15))
+        return SP_ERR_INVALID_ARG;
+    const bool has_left = x_begin > 0, has_right = x_begin + n_local < n_global;
+    if ((has_left && (!L->left_bufs[0] || !L->left_bufs[1] || !L->left_flags)) ||
+        (has_right && (!L->right_bufs[0] || !L->right_bufs[1] || !L->right_flags)))
+        return SP_ERR_INVALID_ARG;
+    int64_t S;
+    int32_t wo;
+    int st = geometry(time_tile, space_tile, S, wo);
+    if (st) return st;
+    const int32_t H = halo_of(time_tile);
+    if ((has_left || has_right) && n_local < H) return SP_ERR_INVALID_ARG;
+    if (steps == 0) return SP_OK;
+    const int32_t passes = (steps + time_tile - 1) / time_tile;
+    const int64_t tiles = (n_local + S - 1) / S;
+    if (flags_len < tiles + 1 + 2 * (int64_t)passes) return SP_ERR_INVALID_ARG;
+    if ((int64_t)passes * tiles + (int64_t(1) << 20) > INT32_MAX) return SP_ERR_UNSUPPORTED;
+    Variant di;
+    if ((st = device_info(di))) return st;
+    const cudaStream_t s = (cudaStream_t)stream;
+    SP_CUDA_TRY(cudaMemsetAsync(flags, 0, (size_t)(tiles + 1 + 2 * (int64_t)passes) * sizeof(int32_t), s));
+    // edge tiles per side: tile t (owned [x0, x0 + st)) produces one of the first / last H
+    // owned cells iff x0 < x_begin + H / x0 + st > x_end - H (= it reads that halo)
+    const int64_t x_end = x_begin + n_local;
+    int32_t nL = 0, nR = 0;
+    for (int64_t t = 0; t < tiles && x_begin + t * S < x_begin + H; ++t) ++nL;
+    for (int64_t t = tiles - 1; t >= 0; --t) {
+        const int64_t x0 = x_begin + t * S, e = x0 + S < x_end ? x0 + S : x_end;
+        if (e > x_end - H) ++nR;
+        else break;
+    }
+    const uint64_t e0 = L->epoch0 + 1;  // pass p's halo epoch = e0 + p
+    PassArgs p{a_local, nullptr, n_global, x_begin - H, n_local + 2 * H, x_begin, x_end, S, tiles, time_tile, H, wo,
+               nullptr, kNegZero2,
+               has_left ? L->left_bufs[0] + L->left_n_local + H : nullptr,
+               has_right ? L->right_bufs[0] : nullptr,
+               has_left ? L->left_flags + 1 : nullptr,
+               has_right ? L->right_flags + 0 : nullptr,
+               has_left ? L->my_flags + 0 : nullptr,
+               has_right ? L->my_flags + 1 : nullptr,
+               (unsigned long long)e0,
+               has_left ? L->my_flags + 2 : nullptr,
+               has_right ? L->my_flags + 3 : nullptr,
+               flags, {a_local, work_local}, passes, steps, time_tile, nullptr, nullptr, 0,
+               {has_left ? L->left_bufs[0] + L->left_n_local + H : nullptr,
+                has_left ? L->left_bufs[1] + L->left_n_local + H : nullptr},
+               {has_right ? L->right_bufs[0] : nullptr, has_right ? L->right_bufs[1] : nullptr},
+               flags + tiles + 1, has_left ? nL : 0, has_right ? nR : 0};
+    if ((st = launch_pass(p, s, di, true))) return st;
+    if (passes & 1)
+        SP_CUDA_TRY(cudaMemcpyAsync(a_local + H, work_local + H, (size_t)n_local * sizeof(float),
+                                    cudaMemcpyDeviceToDevice, s));
+    peer_done_kernel<<<1, 1, 0, s>>>(has_left ? L->left_flags + 3 : nullptr, has_right ? L->right_flags + 2 : nullptr,
+                                     (unsigned long long)(L->epoch0 + (uint64_t)passes));
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }

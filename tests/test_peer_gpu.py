@@ -1,4 +1,5 @@
-"""Fused peer-memory halo exchange (sp_jacobi1d_timetiled_peer) across processes.
+"""Fused peer-memory halo exchange (sp_jacobi1d_timetiled_peer, and its persistent form
+sp_jacobi1d_timetiled_peer_fused) across processes.
 
 The box has one GPU, so the ranks are processes sharing it: buffers and flags are exported
 with CUDA IPC and the pass kernels store halos straight into the neighbours' buffers — the
@@ -24,7 +25,7 @@ def _free_port():
     return p
 
 
-def _worker(rank, world, port, n, steps_list, tt, out_dir):
+def _worker(rank, world, port, n, steps_list, tt, out_dir, fused=False, space_tile=256):
     import sys
     sys.path.insert(0, ROOT)
     import torch
@@ -38,7 +39,7 @@ def _worker(rank, world, port, n, steps_list, tt, out_dir):
     dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank, world_size=world)
     H = sp.halo_of(tt)
     xb, nl = jacobi_slabs(n, world, H)[rank]
-    slab = sp.PeerSlab(n, xb, nl, tt, space_tile=256)
+    slab = sp.PeerSlab(n, xb, nl, tt, space_tile=space_tile, fused=fused)
     slab.a[H:H + nl] = torch.from_numpy(sp_inputs.jacobi_input(nl, seed=31, begin=xb)).cuda()
     torch.cuda.synchronize()
     dist.barrier()
@@ -57,6 +58,22 @@ def test_peer_fused_halo_equals_oracle(world, tmp_path):
     import sp_inputs
     n, tt, steps_list = 12011, 16, [37, 16]
     mp.spawn(_worker, args=(world, _free_port(), n, steps_list, tt, str(tmp_path)), nprocs=world, join=True)
+    got = np.concatenate([np.load(tmp_path / f"r{r}.npy") for r in range(world)])
+    want = oracle.jacobi1d(sp_inputs.jacobi_input(n, seed=31), sum(steps_list))
+    assert np.array_equal(got.view(np.uint32), want.view(np.uint32))
+
+
+@pytest.mark.timeout(600)
+@pytest.mark.parametrize("world,space_tile", [(2, 256), (3, 256), (2, 8)])
+def test_peer_persistent_halo_equals_oracle(world, space_tile, tmp_path):
+    """sp_jacobi1d_timetiled_peer_fused: every pass of a call in one persistent launch per
+    rank, halos pushed by the last edge tile of each side (space tile 8 < halo 16: two edge
+    tiles per side).  Three calls (37, 16, 5 steps) exercise the call-boundary handshake."""
+    import oracle
+    import sp_inputs
+    n, tt, steps_list = 12011, 16, [37, 16, 5]
+    mp.spawn(_worker, args=(world, _free_port(), n, steps_list, tt, str(tmp_path), True, space_tile), nprocs=world,
+             join=True)
     got = np.concatenate([np.load(tmp_path / f"r{r}.npy") for r in range(world)])
     want = oracle.jacobi1d(sp_inputs.jacobi_input(n, seed=31), sum(steps_list))
     assert np.array_equal(got.view(np.uint32), want.view(np.uint32))
