@@ -311,8 +311,12 @@ def run_ours(args, rank, world, local_rank):
         clk.mark()
         barrier()
     total_ms = e_start.elapsed_time(e_end)
-    jac_ms = sum(ev[k][0].elapsed_time(ev[k][1]) for k in range(K))
-    me_ms = sum(ev[k][1].elapsed_time(ev[k][2]) for k in range(K))
+    jac_steps = [ev[k][0].elapsed_time(ev[k][1]) for k in range(K)]
+    me_steps = [ev[k][1].elapsed_time(ev[k][2]) for k in range(K)]
+    jac_ms, me_ms = sum(jac_steps), sum(me_steps)
+    # the median and the best step beside the mean (this rank's events)
+    step_stats = {"jacobi_ms": {"median": round(float(np.median(jac_steps)), 4), "best": round(min(jac_steps), 4)},
+                  "me_ms": {"median": round(float(np.median(me_steps)), 4), "best": round(min(me_steps), 4)}}
 
     def max_over_ranks(x):
         if world == 1:
@@ -457,6 +461,7 @@ def run_ours(args, rank, world, local_rank):
         "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
                "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},
         "roofline": dominant, "roofline_jacobi": roof_jac, "roofline_jacobi_hbm_regime": roof_hbm,
+        "step_stats": step_stats,
         "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches_per_step * K, "clocks": clk.summary(),
     }
     if rank == 0:
