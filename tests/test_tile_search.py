@@ -61,3 +61,37 @@ def test_model_properties():
     assert not none["feasible"]
     with pytest.raises(sp.SPError):
         sp.tile_search(ext, _jacobi_like(), [[64], [8]], procs=8)  # t > N
+
+
+def test_cost_hand_derived_jacobi_band():
+    """Pin of the §4.3 objective computed by hand for one tile of the Jacobi
+    band (extent T = 32, N = 256; tile t = (8, 64); P = 8, S = 20, L = 1):
+    array a is read (a[i-1], a[i], a[i+1]) -> one move-in per tile of the box [-1, 64]:
+    V_in = 66;  array b is written (b[i]) -> one move-out per tile: V_out = 64.  Both depend
+    on loop 1, so neither movement is hoisted: 4 x 4 = 16 tiles each.
+    C = 16 (8*20 + 66/8) + 16 (8*20 + 64/8) = 2692 + 2688 = 5380;  local footprint 66 + 64."""
+    for f in (sp.tile_search, OT.tile_search):
+        r = f([32, 256], _jacobi_like(), [[8], [64]], procs=8, sync_cost=20.0, elem_cost=1.0)
+        best = r if "tile" in r else r["best"]
+        assert list(best["tile"]) == [8, 64]
+        assert best["cost"] == pytest.approx(5380.0)
+        assert best["local_elems"] == 130
+
+
+def test_cost_hand_derived_matvec_hoisting():
+    """Hoisting above a redundant tiling loop (reading R-T2), by hand: y[i] +=
+    A[i][j] * x[j] over (i, j) with extent (64, 128), tile (16, 32), P = 4, S = 10, L = 2.
+    y depends only on loop 0: moved in and out once per i-tile (4 times, 16 elements each);
+    A (16 x 32) and x (32) depend on loop 1: moved in per tile (4 x 4 = 16 times).
+    C = 4 (40 + 16*2/4) * 2 + 16 (40 + 512*2/4) + 16 (40 + 32*2/4) = 384 + 4736 + 896 = 6016."""
+    refs = [
+        {"array": 0, "is_write": 1, "rank": 1, "rows": [[1, 0, 0]]},             # y[i] (write)
+        {"array": 0, "is_write": 0, "rank": 1, "rows": [[1, 0, 0]]},             # y[i] (read)
+        {"array": 1, "is_write": 0, "rank": 2, "rows": [[1, 0, 0], [0, 1, 0]]},  # A[i][j]
+        {"array": 2, "is_write": 0, "rank": 1, "rows": [[0, 1, 0]]},             # x[j]
+    ]
+    for f in (sp.tile_search, OT.tile_search):
+        r = f([64, 128], refs, [[16], [32]], procs=4, sync_cost=10.0, elem_cost=2.0)
+        best = r if "tile" in r else r["best"]
+        assert best["cost"] == pytest.approx(6016.0)
+        assert best["local_elems"] == 16 + 512 + 32
