@@ -81,3 +81,26 @@ def test_struct_layouts_match_the_library():
     assert sp.lib.sp_abi_struct_sizes(out, len(order)) == len(order)
     for cls, n in zip(order, out):
         assert ctypes.sizeof(cls) == n, (cls.__name__, ctypes.sizeof(cls), n)
+
+
+def test_peer_entry_points_validate_before_cuda():
+    """sp_jacobi1d_timetiled_peer(_fused): argument errors return SP_ERR_INVALID_ARG before any
+    CUDA call (fake, never dereferenced, 16-byte-aligned pointers)."""
+    L = sp.sp_peer_links()
+    L.my_flags = 0x10000
+    a, w, f = 0x20000, 0x40000, 0x60000
+    fused = sp.lib.sp_jacobi1d_timetiled_peer_fused
+    # no links / a == work / misaligned slab start / x range outside the domain
+    assert fused(None, a, w, f, 100, 1000, 0, 1000, 10, 16, 0, None) == -1
+    assert fused(ctypes.byref(L), a, a, f, 100, 1000, 0, 1000, 10, 16, 0, None) == -1
+    assert fused(ctypes.byref(L), a, w, f, 100, 1000, 2, 900, 10, 16, 0, None) == -1
+    assert fused(ctypes.byref(L), a, w, f, 100, 1000, 0, 1001, 10, 16, 0, None) == -1
+    # a slab with a left neighbour but no mapped neighbour buffers
+    assert fused(ctypes.byref(L), a, w, f, 100, 1000, 500, 500, 10, 16, 0, None) == -1
+    # flags too short: tiles + 1 + 2 * passes entries are needed (one tile, 1 pass -> 4)
+    assert fused(ctypes.byref(L), a, w, f, 3, 1000, 0, 1000, 10, 16, 0, None) == -1
+    # zero steps is the identity (no launch)
+    assert fused(ctypes.byref(L), a, w, f, 1, 1000, 0, 1000, 0, 16, 0, None) == 0
+    per_pass = sp.lib.sp_jacobi1d_timetiled_peer
+    assert per_pass(None, a, w, 1000, 0, 1000, 10, 16, 0, None) == -1
+    assert per_pass(ctypes.byref(L), a, w, 1000, 500, 500, 10, 16, 0, None) == -1
