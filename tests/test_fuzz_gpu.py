@@ -31,7 +31,7 @@ def _jacobi_cases(seed, count):
         yield n, steps, tt, S, H
 
 
-@pytest.mark.parametrize("seed", range(4))
+@pytest.mark.parametrize("seed", range(8))
 def test_jacobi_random_shapes_all_entry_points(seed):
     checked = 0
     for n, steps, tt, S, H in _jacobi_cases(100 + seed, 6):
@@ -67,7 +67,7 @@ def test_jacobi_random_shapes_all_entry_points(seed):
     assert checked == 6
 
 
-@pytest.mark.parametrize("seed", range(3))
+@pytest.mark.parametrize("seed", range(6))
 def test_me_random_frames_surfaces(seed):
     rng = np.random.default_rng(200 + seed)
     pairs_checked = 0
