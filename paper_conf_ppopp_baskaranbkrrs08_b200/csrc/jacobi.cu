@@ -772,6 +772,10 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         if (lane == 0) atomicAdd(&g_jac_dbg[6 + (pass > 0)], (unsigned long long)(clock64() - tp1));
         if (lane == 0) atomicAdd(&g_jac_dbg[8 + (pass > 0)], 1ull);
 #endif
+#ifdef SP_JAC_STRESS  // schedule stress (tests run against a build with it): one tile in eight, picked by
+        // a hash of (tile, pass), finishes 20 us late, so dependent tiles really wait
+        if ((((uint32_t)t * 2654435761u) ^ (uint32_t)(pass * 40503u)) % 8u == 0u) __nanosleep(20000);
+#endif
         // ---- owned cells -> staged buffer -> TMA bulk store ------------------------------
         {
             const int own_hi = A.H + (int)st;  // strip offsets [H, H + st) are owned
