@@ -370,7 +370,7 @@ def run_ours(args, rank, world, local_rank):
     roof_jac = {"kernel": "jacobi1d_pass_kernel", "bound": "alu", "achieved": round(jac_tflops, 2),
                 "peak": round(fp32_peak, 2), "unit": "TFLOP/s (fp32)", "frac": round(jac_tflops / fp32_peak, 4),
                 "traffic": tr.get("jacobi1d_pass_kernel"),
-                "peak_source": "148 SM x 128 fp32 flop/clk (guide unit counts; microbenchmark-confirmed) x sm_max_mhz",
+                "peak_source": "148 SM x 128 fp32 lanes/clk x 1 op (the update is FADD, FADD, FMUL: no FMA to count twice; guide unit counts, microbenchmark-confirmed) x sm_max_mhz",
                 "per_launch_ms": round(jac_launch_ms, 4), "algorithmic_flops_per_launch": jac_flops,
                 "hbm": {"achieved": round(jac_gbs, 1), "peak": pk["hbm_gbs"], "unit": "GB/s",
                         "frac": round(jac_gbs / pk["hbm_gbs"], 4), "algorithmic_bytes_per_launch": jac_bytes,
