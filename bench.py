@@ -1,24 +1,33 @@
 """Benchmark of the staged multi-level-tiled hot path (Baskaran et al., PPoPP'08) on B200.
 
 One step = one pass of the whole hot path over one batch:
-  * Jacobi (BASELINE config 3): T = 1024 steps of the fp32 1-D Jacobi stencil over
-    n_local = 2^26 cells per GPU, time-tiled (N = 1: every pass in one persistent launch with
-    per-tile dependence flags; N > 1: one launch per time tile);
-  * ME (BASELINE config 4): full-search SAD motion estimation of a 64-pair batch of
-    1920x1080 uint8 frames, +-32, 16x16 macroblocks, per GPU.
-Multi-GPU (torchrun, one process per GPU): weak scaling.  Jacobi's global domain is the
-concatenation of the ranks' slabs with a halo exchange once per time tile, fused into the
-pass kernel as peer-memory stores (default) or as NCCL send/recv (--halo nccl); ME ranks search their own 64-pair shard of a 64*N-pair batch (no data-path
-collective).  `value` = Jacobi point-updates of all ranks / max-over-ranks device time;
-ME's throughput is reported in the `me` object with its own roofline.
+  * N = 1 (BASELINE configs 3 + 4):
+      - Jacobi J3: T = 1024 steps of the fp32 1-D Jacobi stencil over 2^26 cells, time-tiled,
+        every pass in one persistent launch with per-tile dependence flags;
+      - ME M4: full-search SAD motion estimation of a 64-pair batch of 1920x1080 uint8 frames,
+        +-32, 16x16 macroblocks.
+  * N > 1 (BASELINE configs 5 + 4, strong scaling: the total problem is fixed):
+      - Jacobi J5: 2^30 cells, T = 4096, split into N contiguous slabs; the halo exchange
+        once per time tile is fused into each rank's persistent kernel as peer-memory stores
+        over NVLink (default) or done by NCCL send/recv per pass (--halo nccl);
+      - ME M4: the same 64-pair batch, its (pair, MB row) space split over the ranks by valid-
+        candidate count; each rank holds only its band rows and the results are all-gathered
+        by the search kernel itself over peer memory (default) or by grouped NCCL broadcasts
+        (--gather nccl).
+`value` = Jacobi point-updates of the whole job / max-over-ranks device time; ME's throughput
+is reported in the `me` object with its own roofline.
 
   python bench.py [--gpus N] [--steps K] [--warmup W] [--impl ours|reference] [--time-tile Tt]
+
+With --gpus N > 1 and no torchrun environment, bench.py launches itself under
+torch.distributed.run (one process per GPU, rendezvous on 127.0.0.1).
 """
 from __future__ import annotations
 
 import argparse
 import json
 import os
+import socket
 import statistics
 import subprocess
 import sys
@@ -31,32 +40,50 @@ ROOT = os.path.dirname(os.path.abspath(__file__))
 sys.path.insert(0, ROOT)
 
 METRIC = "Jacobi GPoint-updates/s & ME SAD/s; %HBM roofline at 1/2/4/8 B200"
-JAC_N_LOCAL = 1 << 26
-JAC_T = 1024
+JAC3_N, JAC3_T = 1 << 26, 1024    # BASELINE config 3 (N = 1)
+JAC5_N, JAC5_T = 1 << 30, 4096    # BASELINE config 5 (N > 1, strong scaling)
 ME_W, ME_H, ME_R, ME_PAIRS = 1920, 1080, 32, 64
 VABSDIFF4_PER_CLK_SM = 64  # measured issue rate (profiles/r01_ubench_issue_rates.txt)
 
 
-def me_valid_sads(width, height, r, pairs):
-    tot = 0
-    for by in range(height // 16):
+def me_valid_sads(width, height, r, pairs, rows=None):
+    """Valid 16x16 candidates (restricted vectors) of `pairs` pairs, or of the flat (pair, MB
+    row) rows `rows` = (begin, end) of the batch."""
+    mby = height // 16
+
+    def row_count(by):
         y0 = 16 * by
         ny = min(r, height - 16 - y0) - max(-r, -y0) + 1
-        for bx in range(width // 16):
-            x0 = 16 * bx
-            tot += (min(r, width - 16 - x0) - max(-r, -x0) + 1) * ny
-    return tot * pairs
+        return ny * sum(min(r, width - 16 - 16 * bx) - max(-r, -16 * bx) + 1 for bx in range(width // 16))
+    per_row = [row_count(by) for by in range(mby)]
+    if rows is None:
+        return sum(per_row) * pairs
+    return sum(per_row[k % mby] for k in range(rows[0], rows[1]))
 
 
-def bench_config(world, tt):
+def workload(world, tt):
+    if world == 1:
+        return {"name": "J3+M4", "jac_n": JAC3_N, "jac_t": JAC3_T}
+    return {"name": "J5+M4", "jac_n": JAC5_N, "jac_t": JAC5_T}
+
+
+def bench_config(world, tt, halo="peer", gather="peer"):
     h = (tt + 3) & ~3
-    return {"workload": f"J3: Jacobi fp32 N=2^26 cells/GPU, T={JAC_T}, time tile {tt} (halo {h}) + "
-                        f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs/GPU",
-            "jacobi_global_n": JAC_N_LOCAL * world, "time_tile": tt, "me_pairs_global": ME_PAIRS * world,
-            "l2": "inputs larger than L2 (256 MiB Jacobi state per GPU, 135 MB frame batch); no flush",
-            "parallelism": f"weak scaling over {world} GPU(s); Jacobi halo exchange per time tile, fused "
-                           "into the persistent kernel (edge tiles store halos into the neighbours' buffers "
-                           "over peer memory)"}
+    if world == 1:
+        return {"workload": f"J3: Jacobi fp32 N=2^26, T={JAC3_T}, time tile {tt} (halo {h}) + "
+                            f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs",
+                "jacobi_global_n": JAC3_N, "jacobi_steps": JAC3_T, "time_tile": tt, "me_pairs_global": ME_PAIRS,
+                "l2": "inputs larger than L2 (256 MiB Jacobi state, 135 MB frame batch); no flush",
+                "parallelism": "1 GPU"}
+    return {"workload": f"J5: Jacobi fp32 N=2^30, T={JAC5_T}, time tile {tt} (halo {h}), {world} slabs + "
+                        f"M4: ME {ME_W}x{ME_H} uint8 +-{ME_R}, {ME_PAIRS} pairs sharded by MB rows",
+            "jacobi_global_n": JAC5_N, "jacobi_steps": JAC5_T, "time_tile": tt, "me_pairs_global": ME_PAIRS,
+            "l2": "inputs larger than L2 (4 GiB / N of Jacobi state per GPU); no flush",
+            "parallelism": f"strong scaling over {world} GPUs; Jacobi halo exchange per time tile "
+                           + ("fused into the persistent kernel (peer-memory stores over NVLink)" if halo == "peer"
+                              else "by NCCL send/recv between per-pass launches")
+                           + "; ME results all-gathered "
+                           + ("by the search kernel (peer stores)" if gather == "peer" else "by NCCL broadcasts")}
 
 
 def peaks():
@@ -151,33 +178,47 @@ def traffic_from_profiles():
 
 
 # ---------------------------------------------------------------------------------------
-# reference arm: the CPU oracle, as it stands, on the host cores
+# the CPU oracle, as it stands, on the host cores (reference arm and cpu_baseline)
 # ---------------------------------------------------------------------------------------
-def oracle_samples(rng_seed=0):
-    """Bounded samples of the bench workload for the oracle (~2-4 s of CPU per call)."""
+def oracle_samples():
+    """Bounded samples of the bench workload for the oracle: all host threads (~10-20 cpu-s)
+    and one thread (~1 s)."""
     import oracle
     import sp_inputs
     cores = len(os.sched_getaffinity(0))
-    oracle.set_threads(cores)
-    # Jacobi: the full 2^26-cell state, 16 of the 1024 steps
-    a = sp_inputs.jacobi_input(JAC_N_LOCAL, seed=sp_inputs.JACOBI_BENCH_SEED)
-    js = 16
-    t0 = time.perf_counter()
-    oracle.jacobi1d(a, js)
-    tj = time.perf_counter() - t0
-    jac = (JAC_N_LOCAL - 2) * js / tj
-    # ME: 2 macroblock rows (interior) of one 1080p pair at +-32
+    a = sp_inputs.jacobi_input(JAC3_N, seed=sp_inputs.JACOBI_BENCH_SEED)
     fr0 = sp_inputs.me_frame(0, ME_W, ME_H, ME_R)
     fr1 = sp_inputs.me_frame(1, ME_W, ME_H, ME_R)
-    mbx = ME_W // 16
-    mbs = np.arange(30 * mbx, 32 * mbx, dtype=np.int32)
-    t0 = time.perf_counter()
-    oracle.me_search(fr0, fr1, ME_W, ME_H, ME_R, mbs=mbs)
-    tm = time.perf_counter() - t0
-    me = len(mbs) * (2 * ME_R + 1) ** 2 / tm
-    return {"jacobi_ups": jac, "me_sads": me, "cores": oracle.get_threads(), "jacobi_s": tj, "me_s": tm,
-            "sample": f"Jacobi: N=2^26 cells x {js} steps (of T=1024); ME: {len(mbs)} interior macroblocks "
-                      f"(2 MB rows) of one 1920x1080 pair at +-32"}
+    mbx, mby = ME_W // 16, ME_H // 16
+    out = {}
+    for tag, threads, js, me_rows in (("all", cores, 32, (0, mby)), ("one", 1, 4, (30, 32))):
+        oracle.set_threads(threads)
+        t0 = time.perf_counter()
+        oracle.jacobi1d(a, js)
+        tj = time.perf_counter() - t0
+        mbs = np.arange(me_rows[0] * mbx, me_rows[1] * mbx, dtype=np.int32)
+        t0 = time.perf_counter()
+        oracle.me_search(fr0, fr1, ME_W, ME_H, ME_R, mbs=mbs)
+        tm = time.perf_counter() - t0
+        out[tag] = {"jacobi_ups": (JAC3_N - 2) * js / tj, "me_sads": me_valid_sads(ME_W, ME_H, ME_R, 1, me_rows) / tm,
+                    "threads": oracle.get_threads(), "jacobi_steps": js, "me_mb_rows": me_rows,
+                    "seconds": tj + tm}
+    oracle.set_threads(cores)
+    a_ = out["all"]
+    o_ = out["one"]
+    return {"jacobi_ups": a_["jacobi_ups"], "me_sads": a_["me_sads"], "cores": a_["threads"],
+            "jacobi_ups_1t": o_["jacobi_ups"], "me_sads_1t": o_["me_sads"], "cpu_model": oracle.cpu_model(),
+            "sample": (f"all {a_['threads']} threads: Jacobi N=2^26 x {a_['jacobi_steps']} steps (of T=1024), "
+                       f"ME one whole 1920x1080 pair at +-32 (M4 has 64); 1 thread: Jacobi N=2^26 x "
+                       f"{o_['jacobi_steps']} steps, ME 2 interior MB rows"),
+            "build": "gcc " + " ".join(oracle.CFLAGS)}
+
+
+def cpu_baseline_obj(s, value_key="jacobi_ups"):
+    return {"value": s[value_key] / 1e9, "unit": "GPoint-updates/s", "cores": s["cores"], "kind": "oracle",
+            "sample": s["sample"], "value_1thread": s["jacobi_ups_1t"] / 1e9, "cpu_model": s["cpu_model"],
+            "me_value": s["me_sads"] / 1e9, "me_value_1thread": s["me_sads_1t"] / 1e9, "me_unit": "GSAD/s",
+            "build": s["build"]}
 
 
 def run_reference(args, rank, world):
@@ -185,7 +226,7 @@ def run_reference(args, rank, world):
         return 0
     for _ in range(args.warmup):
         oracle_samples()
-    js, ms, tot = [], [], 0.0
+    js, ms = [], []
     t_start = time.perf_counter()
     last = None
     for _ in range(args.steps):
@@ -194,15 +235,17 @@ def run_reference(args, rank, world):
         ms.append(last["me_sads"])
     tot = time.perf_counter() - t_start
     val = statistics.median(js) / 1e9
+    cb = cpu_baseline_obj(last)
+    cb["value"] = val
     line = {
         "impl": "reference", "metric": METRIC, "value": val, "unit": "GPoint-updates/s", "n_gpus": args.gpus,
         "steps": args.steps, "warmup": args.warmup, "ms_per_step": tot / max(1, args.steps) * 1e3,
-        "higher_is_better": True, "scaling": "weak", "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
-        "config": dict(bench_config(world, args.time_tile),
+        "higher_is_better": True, "scaling": "weak" if args.gpus == 1 else "strong", "vs_baseline": None,
+        "dtype": "f32/u8", "data": "synthetic",
+        "config": dict(bench_config(args.gpus, args.time_tile),
                        note="oracle timed on bounded samples of the workload (see cpu_baseline.sample)"),
         "me": {"value": statistics.median(ms) / 1e9, "unit": "GSAD/s"},
-        "cpu_baseline": {"value": val, "unit": "GPoint-updates/s", "cores": last["cores"], "kind": "oracle",
-                         "sample": last["sample"], "me_value": statistics.median(ms) / 1e9, "me_unit": "GSAD/s"},
+        "cpu_baseline": cb,
         "e2e": {"value": val, "unit": "GPoint-updates/s", "h2d_bytes_per_step": 0, "d2h_bytes_per_step": 0},
     }
     print(json.dumps(line), flush=True)
@@ -218,6 +261,7 @@ def run_ours(args, rank, world, local_rank):
 
     import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
     import sp_inputs
+    from paper_conf_ppopp_baskaranbkrrs08_b200 import partition
 
     dev = torch.device("cuda", local_rank)
     torch.cuda.set_device(dev)
@@ -225,11 +269,11 @@ def run_ours(args, rank, world, local_rank):
     tt = args.time_tile
     H = sp.halo_of(tt)
     pk = peaks()
+    wl = workload(world, tt)
+    n_global, T = wl["jac_n"], wl["jac_t"]
 
     # ---- Jacobi state: this rank's slab [x_begin, x_begin + n_local) of the global domain
-    n_local = JAC_N_LOCAL
-    n_global = n_local * world
-    x_begin = rank * n_local
+    x_begin, n_local = partition.jacobi_slabs(n_global, world, H)[rank]
     comm = None
     slab = None
     flags = None
@@ -238,7 +282,7 @@ def run_ours(args, rank, world, local_rank):
         a = torch.from_numpy(a_host).to(dev)
         work = torch.empty_like(a)
         # all passes in one persistent launch (per-tile completion flags + unit counter)
-        flags = torch.empty(sp.jacobi1d_plan(n_local, JAC_T, tt, 0)["tiles"] + 1, dtype=torch.int32, device=dev)
+        flags = torch.empty(sp.jacobi1d_plan(n_local, T, tt, 0)["tiles"] + 1, dtype=torch.int32, device=dev)
     elif args.halo == "peer":
         # fused halo exchange: ONE persistent launch per step on every rank; the edge tiles
         # store their halos into the neighbours' buffers as soon as they complete
@@ -252,33 +296,45 @@ def run_ours(args, rank, world, local_rank):
         a[lo - (x_begin - H): hi - (x_begin - H)] = torch.from_numpy(
             sp_inputs.jacobi_input(hi - lo, seed=sp_inputs.JACOBI_BENCH_SEED, begin=lo)).to(dev)
         work = torch.empty_like(a)
-        uid = torch.zeros(128, dtype=torch.uint8, device=dev)
-        if rank == 0:
-            uid.copy_(torch.frombuffer(bytearray(sp.get_unique_id()), dtype=torch.uint8))
-        dist.broadcast(uid, 0)
-        comm = sp.Comm(bytes(uid.cpu().numpy().tobytes()), world, rank, local_rank)
+    if world > 1 and (args.halo == "nccl" or args.gather == "nccl"):
+        uid = [sp.get_unique_id() if rank == 0 else None]
+        dist.broadcast_object_list(uid, 0)
+        comm = sp.Comm(uid[0], world, rank, local_rank)
 
     def jacobi_run(steps):
         if slab is not None:
             slab.run(steps)
-        elif comm is not None:
+        elif world > 1:
             comm.jacobi1d_timetiled_dist(a, work, n_global, x_begin, n_local, steps, tt, 0)
         else:
             sp.jacobi1d_timetiled_fused(a, steps, tt, 0, work=work, flags=flags)
 
     def jacobi_step():
-        jacobi_run(JAC_T)
+        jacobi_run(T)
 
-    # ---- ME batch: this rank's 64 pairs = frames [64 r, 64 r + 65) of the sequence
-    f0 = ME_PAIRS * rank
-    frames_host = np.ascontiguousarray(np.stack([sp_inputs.me_frame(f0 + f, ME_W, ME_H, ME_R) for f in range(ME_PAIRS + 1)]))
-    frames = torch.from_numpy(frames_host).to(dev)
+    # ---- ME batch: 64 pairs = frames [0, 65) of the sequence; N > 1: this rank's MB-row range
     mbx, mby = ME_W // 16, ME_H // 16
-    me_out = (torch.empty((ME_PAIRS, mby, mbx, 2), dtype=torch.int16, device=dev),
-              torch.empty((ME_PAIRS, mby, mbx), dtype=torch.int32, device=dev), None)
+    me_shard = None
+    frames_host = None
+    if world == 1:
+        frames_host = np.ascontiguousarray(np.stack([sp_inputs.me_frame(f, ME_W, ME_H, ME_R)
+                                                     for f in range(ME_PAIRS + 1)]))
+        frames = torch.from_numpy(frames_host).to(dev)
+        me_out = (torch.empty((ME_PAIRS, mby, mbx, 2), dtype=torch.int16, device=dev),
+                  torch.empty((ME_PAIRS, mby, mbx), dtype=torch.int32, device=dev), None)
 
-    def me_step():
-        sp.me_search_sequence(frames, ME_W, ME_H, ME_R, out=me_out)
+        def me_step():
+            sp.me_search_sequence(frames, ME_W, ME_H, ME_R, out=me_out)
+    else:
+        me_shard = sp.MEShard(ME_PAIRS, ME_W, ME_H, ME_R)
+        me_shard.load_frames(lambda f: sp_inputs.me_frame(f, ME_W, ME_H, ME_R))
+        if args.gather == "peer":
+            def me_step():
+                me_shard.run()
+        else:
+            def me_step():
+                comm.me_sad_search_dist(me_shard.frames, ME_W, ME_H, ME_R, me_shard.ranges, me_shard.pair_base,
+                                        me_shard.mv, me_shard.sad)
 
     def barrier():
         if world > 1:
@@ -326,23 +382,27 @@ def run_ours(args, rank, world, local_rank):
         return float(t.item())
 
     total_ms, jac_ms, me_ms = max_over_ranks(total_ms), max_over_ranks(jac_ms), max_over_ranks(me_ms)
-    updates = (n_global - 2) * JAC_T * K
-    sads = me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * world * K
+    updates = (n_global - 2) * T * K
+    sads = me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * K
     jac_val = updates / (jac_ms * 1e-3) / 1e9
     me_val = sads / (me_ms * 1e-3) / 1e9
 
     # ---- per-launch kernel durations (CUDA events on the launching stream) for the roofline
-    plan = sp.jacobi1d_plan(n_local, JAC_T, tt, 0)
     e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
     torch.cuda.synchronize()
-    if flags is not None or slab is not None:  # one persistent launch = all T steps (flag memset inside, ~us)
-        reps, steps_per_launch = 3, JAC_T
+    persistent = flags is not None or slab is not None
+    if persistent:  # one persistent launch = all T steps
+        reps, steps_per_launch = (3 if world == 1 else 1), T
+        if world > 1:
+            dist.barrier()
         e0.record(stream)
         for _ in range(reps):
-            jacobi_run(JAC_T)
+            jacobi_run(T)
         e1.record(stream)
-    else:  # one launch per pass: time full-height passes
-        reps, steps_per_launch = 8, tt
+    else:  # one launch per pass (NCCL halo baseline): time full-height passes, exchange included
+        reps, steps_per_launch = 4, tt
+        if world > 1:
+            dist.barrier()
         e0.record(stream)
         for _ in range(reps):
             jacobi_run(2 * tt)
@@ -351,32 +411,39 @@ def run_ours(args, rank, world, local_rank):
     torch.cuda.synchronize()
     jac_launch_ms = e0.elapsed_time(e1) / reps
     jac_bytes = 8.0 * n_local * (steps_per_launch // tt)  # algorithmic: each cell read + written once per pass
-    jac_flops = 3.0 * (n_local - 2) * steps_per_launch  # algorithmic: 3 flops per point-update
+    upd_local = n_local - (x_begin == 0) - (x_begin + n_local == n_global)  # this rank's updated cells
+    jac_flops = 3.0 * upd_local * steps_per_launch  # algorithmic: 3 flops per point-update
     jac_gbs = jac_bytes / (jac_launch_ms * 1e-3) / 1e9
     jac_tflops = jac_flops / (jac_launch_ms * 1e-3) / 1e12
     fp32_peak = 148 * 128 * pk["sm_max_mhz"] * 1e6 / 1e12  # FADD/FMUL (and f32x2 forms) retire 128 flop/clk/SM
+    if world > 1:
+        dist.barrier()
     e0.record(stream)
     for _ in range(3):
         me_step()
     e1.record(stream)
     torch.cuda.synchronize()
     me_launch_ms = e0.elapsed_time(e1) / 3
-    me_ops = me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * 256.0
+    me_ops = (me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) if world == 1 else
+              me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS, (me_shard.flat_begin, me_shard.flat_end))) * 256.0
     me_achieved = me_ops / (me_launch_ms * 1e-3) / 1e12
     alu_peak = 148 * VABSDIFF4_PER_CLK_SM * 4 * pk["sm_max_mhz"] * 1e6 / 1e12
     tr = traffic_from_profiles()
     # Jacobi at Tt >= 16 is bound by the FP32 pipe (3 flops per update; HBM bytes per update
     # fall as 8/Tt): the binding roof is reported, with the HBM view beside it (north_star)
-    roof_jac = {"kernel": "jacobi1d_pass_kernel", "bound": "alu", "achieved": round(jac_tflops, 2),
+    kname = "jacobi1d_pass_kernel" + ("<kPeer>" if slab is not None else "")
+    roof_jac = {"kernel": kname, "bound": "alu", "achieved": round(jac_tflops, 2),
                 "peak": round(fp32_peak, 2), "unit": "TFLOP/s (fp32)", "frac": round(jac_tflops / fp32_peak, 4),
-                "traffic": tr.get("jacobi1d_pass_kernel"),
+                "traffic": tr.get("jacobi1d_pass_kernel") if world == 1 else None,
                 "peak_source": "148 SM x 128 fp32 lanes/clk x 1 op (the update is FADD, FADD, FMUL: no FMA to count twice; guide unit counts, microbenchmark-confirmed) x sm_max_mhz",
                 "per_launch_ms": round(jac_launch_ms, 4), "algorithmic_flops_per_launch": jac_flops,
                 "hbm": {"achieved": round(jac_gbs, 1), "peak": pk["hbm_gbs"], "unit": "GB/s",
                         "frac": round(jac_gbs / pk["hbm_gbs"], 4), "algorithmic_bytes_per_launch": jac_bytes,
                         "peak_source": pk["source"]}}
-    roof_me = {"kernel": "me_sad_kernel", "bound": "alu", "achieved": round(me_achieved, 2), "peak": round(alu_peak, 2),
-               "unit": "Tabsdiff/s", "frac": round(me_achieved / alu_peak, 4), "traffic": tr.get("me_sad_kernel"),
+    roof_me = {"kernel": "me_sad_kernel" + ("<kGather>" if (me_shard is not None and args.gather == "peer") else ""),
+               "bound": "alu", "achieved": round(me_achieved, 2), "peak": round(alu_peak, 2),
+               "unit": "Tabsdiff/s", "frac": round(me_achieved / alu_peak, 4),
+               "traffic": tr.get("me_sad_kernel") if world == 1 else None,
                "peak_source": f"148 SM x {VABSDIFF4_PER_CLK_SM} VABSDIFF4/clk (measured) x 4 x sm_max_mhz",
                "per_launch_ms": round(me_launch_ms, 4), "algorithmic_ops_per_launch": me_ops}
     dominant = roof_jac if jac_ms >= me_ms else roof_me
@@ -405,7 +472,7 @@ def run_ours(args, rank, world, local_rank):
                     "peak_source": pk["source"]}
         del b, wb
 
-    # ---- end-to-end through the public API with host buffers (N = 1: pinned H2D/D2H in the timed region)
+    # ---- end-to-end through the public API with host buffers (pinned H2D / D2H in the timed region)
     e2e = None
     me_e2e = None
     if world == 1:
@@ -413,13 +480,12 @@ def run_ours(args, rank, world, local_rank):
         f_pin = torch.from_numpy(frames_host).pin_memory()
         # host-buffer Jacobi: the kernel reads a_pin and writes the result back over PCIe itself
         # (sp_jacobi1d_host, wavefront order), in place: every call advances the state T steps
-        jac_host = sp.Jacobi1DHost(n_local, JAC_T, tt)
+        jac_host = sp.Jacobi1DHost(n_local, T, tt)
         # host-buffer ME: frames streamed frame by frame while the search runs, MV / SAD stored
         # into pinned host memory by the kernel (sp_me_search_host)
         me_host = sp.MESearchHost(ME_PAIRS + 1, ME_W, ME_H, frames_host.shape[2], ME_R)
-        for _ in range(1):
-            jac_host.run(a_pin)
-            me_host.run(f_pin)
+        jac_host.run(a_pin)
+        me_host.run(f_pin)
         torch.cuda.synchronize()
         ke = max(1, min(K, 3))
         tj = tm = 0.0
@@ -434,35 +500,55 @@ def run_ours(args, rank, world, local_rank):
             tj += t1 - t0
             tm += t2 - t1
         # Jacobi's own bytes: the state read from and written back to pinned host memory
-        e2e = {"value": (n_local - 2) * JAC_T * ke / tj / 1e9, "unit": "GPoint-updates/s",
+        e2e = {"value": (n_local - 2) * T * ke / tj / 1e9, "unit": "GPoint-updates/s",
                "h2d_bytes_per_step": 4 * n_local, "d2h_bytes_per_step": 4 * n_local,
                "api": "sp_jacobi1d_host (kernel move-in/out over PCIe, wavefront order)"}
         me_e2e = {"value": me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * ke / tm / 1e9, "unit": "GSAD/s",
                   "h2d_bytes_per_step": frames_host.nbytes, "d2h_bytes_per_step": ME_PAIRS * mby * mbx * 8,
                   "api": "sp_me_search_host (per-frame H2D overlapped with the search, outputs stored to pinned host)"}
+    else:
+        # every rank: its slab from pinned host memory -> the fused multi-GPU call -> back to
+        # pinned host memory; wall clock per step, max over ranks
+        slab_pin = torch.from_numpy(sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED,
+                                                           begin=x_begin)).pin_memory()
+        ke = max(1, min(K, 2))
+        walls = []
+        for _ in range(ke + 1):  # (the first round is a warm-up)
+            dist.barrier()
+            t0 = time.perf_counter()
+            a[H:H + n_local].copy_(slab_pin, non_blocking=True)
+            jacobi_run(T)
+            slab_pin.copy_(a[H:H + n_local], non_blocking=True)
+            torch.cuda.synchronize()
+            walls.append(time.perf_counter() - t0)
+        tj = max_over_ranks(sum(walls[1:]))
+        e2e = {"value": (n_global - 2) * T * ke / tj / 1e9, "unit": "GPoint-updates/s",
+               "h2d_bytes_per_step": 4 * n_global, "d2h_bytes_per_step": 4 * n_global,
+               "api": "pinned slab H2D + PeerSlab.run (sp_jacobi1d_timetiled_peer_fused) + D2H on every rank"
+                      if slab is not None else "pinned slab H2D + Comm.jacobi1d_timetiled_dist + D2H on every rank"}
 
     # ---- CPU baseline: the oracle on a bounded sample (rank 0, N = 1 only)
     cpu = None
     if world == 1 and not args.no_cpu_baseline:
-        s = oracle_samples()
-        cpu = {"value": s["jacobi_ups"] / 1e9, "unit": "GPoint-updates/s", "cores": s["cores"], "kind": "oracle",
-               "sample": s["sample"], "me_value": s["me_sads"] / 1e9, "me_unit": "GSAD/s"}
+        cpu = cpu_baseline_obj(oracle_samples())
 
-    # our kernels per step: Jacobi (1 persistent launch at N = 1, else one per pass) + ME (+ peer done signal)
-    launches_per_step = (1 if (flags is not None or slab is not None) else plan["passes"]) + 1 + \
-        (1 if slab is not None else 0)
+    # our kernels per step: Jacobi (1 persistent launch, or one per pass) (+ peer done signal)
+    # + ME (1 launch; + the gather wait kernel)
+    jac_l = (1 if persistent else -(-T // tt)) + (1 if slab is not None else 0)
+    me_l = 1 + (1 if (me_shard is not None and args.gather == "peer") else 0)
     line = {
         "metric": METRIC, "value": round(jac_val, 2), "unit": "GPoint-updates/s", "n_gpus": world, "steps": K,
-        "warmup": args.warmup, "ms_per_step": round(total_ms / K, 4), "higher_is_better": True, "scaling": "weak",
+        "warmup": args.warmup, "ms_per_step": round(total_ms / K, 4), "higher_is_better": True,
+        "scaling": "weak" if world == 1 else "strong",
         "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
-        "config": bench_config(world, tt),
+        "config": bench_config(world, tt, args.halo, args.gather),
         "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4),
-                   "space_tile": plan["space_tile"], "passes_per_step": plan["passes"]},
+                   "n_local": n_local, "passes_per_step": -(-T // tt)},
         "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
                "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},
         "roofline": dominant, "roofline_jacobi": roof_jac, "roofline_jacobi_hbm_regime": roof_hbm,
         "step_stats": step_stats,
-        "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": launches_per_step * K, "clocks": clk.summary(),
+        "cpu_baseline": cpu, "e2e": e2e, "gpu_launches": (jac_l + me_l) * K, "clocks": clk.summary(),
     }
     if rank == 0:
         print(json.dumps(line), flush=True)
@@ -470,10 +556,28 @@ def run_ours(args, rank, world, local_rank):
         comm.destroy()
     if slab is not None:
         slab.close()
+    if me_shard is not None:
+        me_shard.close()
     return 0
 
 
-def main():
+def _free_port():
+    s = socket.socket()
+    s.bind(("127.0.0.1", 0))
+    p = s.getsockname()[1]
+    s.close()
+    return p
+
+
+def launch_cmd(argv, gpus, port=None):
+    """The torchrun command bench.py runs itself under for --gpus N > 1 (one process per GPU
+    of this node, rendezvous on 127.0.0.1)."""
+    return [sys.executable, "-m", "torch.distributed.run", "--nnodes=1", f"--nproc-per-node={gpus}",
+            "--master-addr=127.0.0.1", f"--master-port={port or _free_port()}", os.path.abspath(__file__), *argv]
+
+
+def main(argv=None):
+    argv = sys.argv[1:] if argv is None else argv
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=10)
@@ -483,17 +587,23 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--halo", choices=["peer", "nccl"], default="peer",
                     help="multi-GPU Jacobi halo exchange: fused peer stores in the pass kernel, or NCCL send/recv")
-    args = ap.parse_args()
+    ap.add_argument("--gather", choices=["peer", "nccl"], default="peer",
+                    help="multi-GPU ME result all-gather: fused peer stores in the search kernel, or NCCL broadcasts")
+    args = ap.parse_args(argv)
+    if args.impl == "ours" and args.gpus > 1 and "WORLD_SIZE" not in os.environ:
+        return subprocess.call(launch_cmd(argv, args.gpus))
     world = int(os.environ.get("WORLD_SIZE", "1"))
     rank = int(os.environ.get("RANK", "0"))
     local_rank = int(os.environ.get("LOCAL_RANK", "0"))
+    if args.impl == "reference":
+        return run_reference(args, rank, world)
+    if world != args.gpus:
+        raise SystemExit(f"--gpus {args.gpus} but WORLD_SIZE={world}: launch one process per GPU")
     # test hook: SP_BENCH_SHARE_GPU=1 runs every rank on cuda:0 with a gloo process group, to
     # exercise the multi-rank path on a one-GPU box (timings are then meaningless)
     share = os.environ.get("SP_BENCH_SHARE_GPU") == "1"
     if share:
         local_rank = 0
-    if args.impl == "reference":
-        return run_reference(args, rank, world)
     if world > 1:
         import torch
         import torch.distributed as dist

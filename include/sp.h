@@ -222,15 +222,17 @@ int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t f
  *               Pass 0's move-in reads `in` and the last pass's move-out writes `out`
  *               directly (TMA bulk copies; over PCIe for host memory), so host<->device
  *               transfer is part of the staged movement, overlapped with the other passes.
- *               in and out may alias each other and buf0 (not buf1).
+ *               in may alias out and buf0 (not buf1: pass 0 writes buf1 while later tiles
+ *               of pass 0 still read in); out may alias in, buf0 or buf1 (when out is the
+ *               array the last pass reads, see below).
  *   buf0, buf1: device scratch of n fp32 each (distinct), ping-pong between passes.
  *   skew      : unit order.  0 = pass-major (all tiles of pass p, then pass p+1);
  *               D > 0 = wavefront: tile t of pass p is scheduled at key t + D p (D a power
  *               of two exceeding ceil(H/S)), so pass p runs D tiles behind pass p-1 — the passes of a
  *               band of tiles follow each other while its data is still in L2, and pass 0's
  *               reads / the last pass's writes stream concurrently with the middle passes;
- *               < 0 = library default (wavefront, D = the least power of two >= 1024
- *               exceeding ceil(H/S)).
+ *               < 0 = library default (wavefront, D = 512, doubled until it exceeds
+ *               ceil(H/S); $SP_JACOBI_SKEW overrides 512).
  *   flags as for sp_jacobi1d_timetiled_fused; passes x tiles < 2^31.
  * If out is the array the last pass reads (e.g. passes == 1 and out == in), the last pass
  * writes buf[passes & 1] and the result is copied to out (stream-ordered). */
@@ -404,6 +406,62 @@ int sp_jacobi1d_timetiled_peer(const sp_peer_links* links, float* a_local, float
 int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* links, float* a_local, float* work_local, int32_t* flags,
                                      int64_t flags_len, int64_t n_global, int64_t x_begin, int64_t n_local,
                                      int32_t steps, int32_t time_tile, int32_t space_tile, void* stream);
+
+/* Motion estimation sharded over ranks (§8(e) ME row): the batch's flattened (pair, MB row)
+ * space [0, n_pairs * mby) is split into contiguous ranges (partition.me_row_ranges, balanced
+ * by valid-candidate count); macroblocks are independent FORALL iterations (Fig. 2,
+ * P:L860-861 "requiring no synchronization across thread blocks"), so a rank searches its
+ * range without any exchange and the results are all-gathered once per batch.
+ *
+ * sp_me_sad_search_range: the search of one range on this device.
+ *   ref, cur       : FULL frames (rows [0, frame_height)), pair p at + (p - pair_base) *
+ *                    pair_stride, p in [pair_base, pair_base + n_pairs_buffer); only the rows
+ *                    the range reads need to be valid: cur rows [16 r0, 16 r1) and ref rows
+ *                    [16 r0 - R, 16 r1 + R) ∩ [0, frame_height) of each pair's MB rows [r0, r1)
+ *                    (partition.me_band_rows: the R-row reference halo).
+ *   flat_begin/end : the range, pair_base * mby <= flat_begin <= flat_end <= (pair_base +
+ *                    n_pairs_buffer) * mby, mby = floor(frame_height / 16).
+ *   mv, best_sad   : GLOBAL outputs [n_pairs][mby][mbx](2) as in sp_me_sad_search (mb_row_begin
+ *                    = 0): only the range's entries are written.
+ * Other arguments and errors as for sp_me_sad_search (any 0 <= range <= 63). */
+int sp_me_sad_search_range(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                           int32_t frame_height, int32_t n_pairs_buffer, int64_t pair_stride, int32_t pair_base,
+                           int32_t range, int64_t flat_begin, int64_t flat_end, int16_t* mv, uint32_t* best_sad,
+                           void* stream);
+
+/* sp_me_sad_search_gather: sp_me_sad_search_range with the all-gather FUSED into the search
+ * kernel over peer memory (NVLink P2P / CUDA-IPC mapped pointers): the thread that finishes a
+ * macroblock stores its (MV, SAD) into every rank's output arrays, so the gather overlaps the
+ * search macroblock by macroblock; the kernel's last CTA then raises done[rank] = epoch in
+ * every rank's flags (release, system scope) and a one-CTA wait kernel holds `stream` until
+ * this rank's done[q] >= epoch for all q.  At kernel start rank r announces ready[r] = epoch
+ * to every rank (its outputs of the previous call are no longer read, by stream order); a
+ * macroblock's peer stores wait for every rank's ready.  R must be 16 or 32.
+ *   links->mv[q], sad[q]: rank q's global output arrays (mapped; q == rank: own, device);
+ *   links->flags[q]     : rank q's u64 flags[2 * nranks] = ready[nranks], done[nranks]
+ *                         (zero-initialised, monotone);
+ *   links->epoch        : >= 1, strictly increasing per call, the same on every rank.
+ * Every rank must call it once per epoch (an empty range included).  A rank that never
+ * arrives makes the others trap after ~20 s instead of hanging. */
+#define SP_ME_MAX_RANKS 8
+typedef struct {
+    int32_t nranks, rank;
+    int16_t* mv[SP_ME_MAX_RANKS];
+    uint32_t* sad[SP_ME_MAX_RANKS];
+    unsigned long long* flags[SP_ME_MAX_RANKS];
+    uint64_t epoch;
+} sp_me_gather_links;
+int sp_me_sad_search_gather(const sp_me_gather_links* links, const uint8_t* ref, const uint8_t* cur, int64_t pitch,
+                            int32_t width, int32_t frame_height, int32_t n_pairs_buffer, int64_t pair_stride,
+                            int32_t pair_base, int32_t range, int64_t flat_begin, int64_t flat_end, void* stream);
+
+/* NCCL baseline of the same gather: the rank's range by sp_me_sad_search_range, then one
+ * grouped ncclBroadcast per rank and output array (root q sends its range in place: an
+ * all-gather-v into the global arrays) on `stream`.
+ *   flat_ranges : host int64 [nranks][2], every rank's [flat_begin, flat_end) (contiguous). */
+int sp_me_sad_search_dist(sp_comm* c, const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                          int32_t frame_height, int32_t n_pairs_buffer, int64_t pair_stride, int32_t pair_base,
+                          int32_t range, const int64_t* flat_ranges, int16_t* mv, uint32_t* best_sad, void* stream);
 
 /* Exportable device allocations and CUDA-IPC handles (64 bytes) for the peer path. */
 int sp_device_alloc(void** ptr, int64_t bytes); /* cudaMalloc + zero fill */

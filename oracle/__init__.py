@@ -31,13 +31,44 @@ from . import planner  # noqa: F401  (re-export)
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
 _SRC = os.path.join(_HERE, "oracle.c")
-_LIB = os.path.join(_HERE, "liboracle.so")
 
-CFLAGS = ["-O2", "-fopenmp", "-ffp-contract=off", "-fno-fast-math", "-fPIC", "-shared", "-std=c11"]
+# -O3 -march=native -ffp-contract=off, no -ffast-math (every fp32 op of the
+# definition rounded as written; vectorisation keeps the op order).  -march=native ties the
+# binary to the host CPU, so the library name carries a tag of the CPU model and flags: a box
+# with another CPU builds its own copy instead of loading one it cannot execute.
+CFLAGS = ["-O3", "-march=native", "-fopenmp", "-ffp-contract=off", "-fno-fast-math", "-fPIC", "-shared", "-std=c11"]
+
+
+def cpu_model() -> str:
+    try:
+        with open("/proc/cpuinfo") as f:
+            for ln in f:
+                if ln.startswith("model name"):
+                    return ln.split(":", 1)[1].strip()
+    except OSError:
+        pass
+    return "unknown"
+
+
+def _cpu_tag() -> str:
+    import hashlib
+    flags = ""
+    try:
+        with open("/proc/cpuinfo") as f:
+            for ln in f:
+                if ln.startswith("flags"):
+                    flags = ln
+                    break
+    except OSError:
+        pass
+    return hashlib.sha1((cpu_model() + flags + " ".join(CFLAGS)).encode()).hexdigest()[:12]
+
+
+_LIB = os.path.join(_HERE, f"liboracle.{_cpu_tag()}.so")
 
 
 def build(force: bool = False) -> str:
-    """Compile oracle.c into liboracle.so (gcc; no FMA contraction)."""
+    """Compile oracle.c into liboracle.<cpu tag>.so (gcc -O3 -march=native; no FMA contraction)."""
     if force or not os.path.exists(_LIB) or os.path.getmtime(_LIB) < os.path.getmtime(_SRC):
         tmp = _LIB + f".tmp{os.getpid()}"
         subprocess.check_call(["gcc", *CFLAGS, "-o", tmp, _SRC])

@@ -26,6 +26,9 @@ C entry point -> Python name (same names, `sp_` prefix dropped):
   sp_me_sad_search            -> me_sad_search(ref, cur, ...)          (device tensors)
   sp_me_ref_window            -> me_ref_window(...)
   sp_me_search_host           -> MESearchHost(F, W, H, pitch, R).run(frames_pinned)  (the e2e public call)
+  sp_me_sad_search_range      -> me_sad_search_range(frames, ...)      (one rank's range of a batch)
+  sp_me_sad_search_gather     -> MEShard(...).run()                    (sharded batch, fused peer all-gather)
+  sp_me_sad_search_dist       -> Comm.me_sad_search_dist(...)          (same, NCCL broadcast baseline)
   sp_get_unique_id / sp_comm_init / sp_comm_destroy / sp_allgather -> Comm
 Host-buffer convenience (the end-to-end public API used for bench.py's `e2e`):
   jacobi1d(host_array, steps, ...), me_search(host_frames, ...)
@@ -40,7 +43,7 @@ import numpy as np
 __all__ = [
     "SPError", "lib", "plan_buffers", "jacobi1d_plan", "jacobi1d_tile_footprint", "jacobi1d_timetiled",
     "jacobi1d_pass_segment", "jacobi1d_timetiled_loopback", "me_sad_search", "me_ref_window", "me_search_sequence",
-    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "jacobi1d_resident", "get_unique_id", "PER_ARRAY", "COMPONENTS", "halo_of",
+    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "jacobi1d_resident", "get_unique_id", "MEShard", "me_sad_search_range", "PER_ARRAY", "COMPONENTS", "halo_of",
 ]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
@@ -89,6 +92,14 @@ class sp_jacobi_plan(ctypes.Structure):
 class sp_peer_links(ctypes.Structure):
     _fields_ = [("left_bufs", vp * 2), ("right_bufs", vp * 2), ("left_n_local", i64), ("right_n_local", i64),
                 ("left_flags", vp), ("right_flags", vp), ("my_flags", vp), ("epoch0", ctypes.c_uint64)]
+
+
+ME_MAX_RANKS = 8
+
+
+class sp_me_gather_links(ctypes.Structure):
+    _fields_ = [("nranks", i32), ("rank", i32), ("mv", vp * ME_MAX_RANKS), ("sad", vp * ME_MAX_RANKS),
+                ("flags", vp * ME_MAX_RANKS), ("epoch", ctypes.c_uint64)]
 
 
 class sp_op(ctypes.Structure):
@@ -144,6 +155,11 @@ SYMBOLS = {
     "sp_jacobi1d_resident_capacity": (ctypes.c_int, [ctypes.POINTER(i64)]),
     "sp_jacobi1d_resident": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
+    "sp_me_sad_search_range": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i64, i32, i32, i64, i64, vp, vp, vp]),
+    "sp_me_sad_search_gather": (ctypes.c_int, [ctypes.POINTER(sp_me_gather_links), vp, vp, i64, i32, i32, i32, i64, i32,
+                                               i32, i64, i64, vp]),
+    "sp_me_sad_search_dist": (ctypes.c_int, [vp, vp, vp, i64, i32, i32, i32, i64, i32, i32, ctypes.POINTER(i64), vp, vp,
+                                             vp]),
     "sp_me_search_host": (ctypes.c_int, [vp, i64, i32, i32, i32, i32, vp, vp, vp, vp, vp, vp]),
     "sp_me_ref_window": (ctypes.c_int, [i32, i32, i32, i32, i32, ctypes.POINTER(i64), ctypes.POINTER(i64)]),
     "sp_get_unique_id": (ctypes.c_int, [ctypes.POINTER(ctypes.c_uint8)]),
@@ -219,6 +235,19 @@ def _stream(stream):
 
 def _ptr(t):
     return vp(t.data_ptr()) if t is not None else None
+
+
+def _scratch(shape, dtype, device, stream):
+    """Library scratch allocated for one call.  When the call runs on a stream other than the
+    current one, the caching allocator is told so (record_stream): the block is then not handed
+    out again before the work queued on that stream has finished with it."""
+    import torch
+    t = torch.empty(shape, dtype=dtype, device=device)
+    if stream is not None and not isinstance(stream, int):
+        t.record_stream(stream)
+    elif isinstance(stream, int):
+        t.record_stream(torch.cuda.ExternalStream(stream, device=t.device))
+    return t
 
 
 def halo_of(time_tile: int) -> int:
@@ -395,7 +424,7 @@ def jacobi1d_timetiled(a, steps: int, time_tile: int = 16, space_tile: int = 0, 
     import torch
     assert a.is_cuda and a.dtype == torch.float32 and a.is_contiguous()
     if work is None:
-        work = torch.empty_like(a)
+        work = _scratch(a.shape, a.dtype, a.device, stream)
     _check(lib.sp_jacobi1d_timetiled(_ptr(a), _ptr(work), a.numel(), int(steps), int(time_tile), int(space_tile),
                                      _ptr(footprint_log), _stream(stream)), "sp_jacobi1d_timetiled")
     return a
@@ -408,10 +437,10 @@ def jacobi1d_timetiled_fused(a, steps: int, time_tile: int = 64, space_tile: int
     import torch
     assert a.is_cuda and a.dtype == torch.float32 and a.is_contiguous()
     if work is None:
-        work = torch.empty_like(a)
+        work = _scratch(a.shape, a.dtype, a.device, stream)
     if flags is None:
-        flags = torch.empty(jacobi1d_plan(a.numel(), steps, time_tile, space_tile)["tiles"] + 1, dtype=torch.int32,
-                            device=a.device)
+        flags = _scratch(jacobi1d_plan(a.numel(), steps, time_tile, space_tile)["tiles"] + 1, torch.int32, a.device,
+                         stream)
     _check(lib.sp_jacobi1d_timetiled_fused(_ptr(a), _ptr(work), _ptr(flags), flags.numel(), a.numel(), int(steps),
                                            int(time_tile), int(space_tile), _ptr(footprint_log), _stream(stream)),
            "sp_jacobi1d_timetiled_fused")
@@ -428,11 +457,11 @@ def jacobi1d_timetiled_stream(inp, out, steps: int, time_tile: int = 64, space_t
     assert inp.dtype == torch.float32 and out.dtype == torch.float32 and out.numel() == n
     dev = inp.device if inp.is_cuda else (out.device if out.is_cuda else torch.device("cuda"))
     if buf0 is None:
-        buf0 = torch.empty(n, dtype=torch.float32, device=dev)
+        buf0 = _scratch(n, torch.float32, dev, stream)
     if buf1 is None:
-        buf1 = torch.empty(n, dtype=torch.float32, device=dev)
+        buf1 = _scratch(n, torch.float32, dev, stream)
     if flags is None:
-        flags = torch.empty(jacobi1d_plan(n, steps, time_tile, space_tile)["tiles"] + 1, dtype=torch.int32, device=dev)
+        flags = _scratch(jacobi1d_plan(n, steps, time_tile, space_tile)["tiles"] + 1, torch.int32, dev, stream)
     _check(lib.sp_jacobi1d_timetiled_stream(_ptr(inp), _ptr(out), _ptr(buf0), _ptr(buf1), _ptr(flags), flags.numel(), n,
                                             int(steps), int(time_tile), int(space_tile), int(skew), _ptr(footprint_log),
                                             _stream(stream)), "sp_jacobi1d_timetiled_stream")
@@ -482,7 +511,7 @@ def jacobi1d_untiled(a, steps: int, work=None, stream=None):
     """N1 ablation: no staging, no time tiling (one launch per step).  In place on a[n]."""
     import torch
     if work is None:
-        work = torch.empty_like(a)
+        work = _scratch(a.shape, a.dtype, a.device, stream)
     _check(lib.sp_jacobi1d_untiled(_ptr(a), _ptr(work), a.numel(), int(steps), _stream(stream)), "sp_jacobi1d_untiled")
     return a
 
@@ -620,6 +649,144 @@ def me_search_sequence(frames, width: int, frame_height: int, search_range: int,
     return me_sad_search(frames[:-1], frames[1:], width, frame_height, search_range, **kw)
 
 
+def me_sad_search_range(frames, width: int, frame_height: int, search_range: int, flat_begin: int, flat_end: int,
+                        pair_base: int = 0, out=None, n_pairs_total: int | None = None, stream=None):
+    """sp_me_sad_search_range: the macroblocks of flat (pair, MB row) rows [flat_begin, flat_end)
+    of a batch.  frames: CUDA uint8 [F, H, pitch] holding frames pair_base .. pair_base + F - 1
+    (pair p = (frame p, frame p + 1)); out = (mv [P, mby, mbx, 2] int16, sad [P, mby, mbx] int32)
+    global arrays (allocated for n_pairs_total pairs if None); only the range's entries are written."""
+    import torch
+    assert frames.is_cuda and frames.dtype == torch.uint8 and frames.dim() == 3 and frames.stride(2) == 1
+    mbx, mby = width // 16, frame_height // 16
+    if out is None:
+        P = n_pairs_total if n_pairs_total is not None else pair_base + frames.shape[0] - 1
+        out = (torch.zeros((P, mby, mbx, 2), dtype=torch.int16, device=frames.device),
+               torch.zeros((P, mby, mbx), dtype=torch.int32, device=frames.device))
+    mv, sad = out
+    ref, cur = frames[:-1], frames[1:]
+    _check(lib.sp_me_sad_search_range(_ptr(ref), _ptr(cur), frames.stride(1), int(width), int(frame_height),
+                                      ref.shape[0], frames.stride(0), int(pair_base), int(search_range), int(flat_begin),
+                                      int(flat_end), _ptr(mv), _ptr(sad), _stream(stream)), "sp_me_sad_search_range")
+    return mv, sad
+
+
+class MEShard:
+    """One rank's share of a sharded ME batch (SURVEY §8(e) ME row) with the all-gather fused
+    into the search kernel over peer memory (sp_me_sad_search_gather).
+
+    The batch's n_pairs x mby (pair, MB row) space is split by partition.me_row_ranges over the
+    ranks of the default process group; this rank holds the frames of the pairs its range
+    touches (`frames`, [F, H, pitch] uint8, frames pair_base .. pair_base + F - 1), of which only
+    the rows `needed_rows(f)` are read (the current blocks plus the R-row reference halo,
+    partition.me_band_rows).  Outputs mv / sad are libsp-owned, CUDA-IPC-exported global arrays
+    [n_pairs, mby, mbx](, 2) on every rank; after run() (stream-ordered) every rank's arrays
+    hold the whole batch's results.  Handles are exchanged through torch.distributed (any
+    backend); the data path uses no collective library."""
+
+    def __init__(self, n_pairs: int, width: int, height: int, search_range: int, pitch: int | None = None):
+        import torch
+        import torch.distributed as dist
+        from . import partition
+        self.n_pairs, self.width, self.height, self.range = int(n_pairs), int(width), int(height), int(search_range)
+        self.pitch = int(pitch) if pitch else (self.width + 15) // 16 * 16
+        self.rank, self.world = dist.get_rank(), dist.get_world_size()
+        if self.world > ME_MAX_RANKS:
+            raise ValueError(f"at most {ME_MAX_RANKS} ranks")
+        self.mbx, self.mby = self.width // 16, self.height // 16
+        self.ranges = partition.me_row_ranges(self.n_pairs, self.height, self.range, self.world)
+        self.flat_begin, self.flat_end = self.ranges[self.rank]
+        self.pieces = partition.split_flat_range(self.flat_begin, self.flat_end, self.mby)
+        if self.pieces:
+            self.pair_base = self.pieces[0][0]
+            n_frames = self.pieces[-1][0] - self.pair_base + 2
+        else:
+            self.pair_base, n_frames = 0, 2
+        self.frames = torch.zeros((n_frames, self.height, self.pitch), dtype=torch.uint8, device="cuda")
+        cells = self.n_pairs * self.mby * self.mbx
+        self._own = []
+        ptrs = []
+        for nbytes in (4 * cells, 4 * cells, 16 * self.world):
+            p = vp()
+            _check(lib.sp_device_alloc(ctypes.byref(p), max(16, nbytes)), "sp_device_alloc")
+            self._own.append(p.value)
+            ptrs.append(p.value)
+        self.mv_ptr, self.sad_ptr, self.flags_ptr = ptrs
+        handles = []
+        for q in ptrs:
+            h = (ctypes.c_uint8 * 64)()
+            _check(lib.sp_ipc_get_handle(vp(q), h), "sp_ipc_get_handle")
+            handles.append(bytes(h))
+        info = [None] * self.world
+        dist.all_gather_object(info, handles)
+        L = sp_me_gather_links()
+        L.nranks, L.rank, L.epoch = self.world, self.rank, 0
+        self._mapped = []
+        for q in range(self.world):
+            if q == self.rank:
+                L.mv[q], L.sad[q], L.flags[q] = self.mv_ptr, self.sad_ptr, self.flags_ptr
+                continue
+            got = []
+            for hb in info[q]:
+                m = vp()
+                _check(lib.sp_ipc_open_handle((ctypes.c_uint8 * 64)(*hb), ctypes.byref(m)), "sp_ipc_open_handle")
+                self._mapped.append(m.value)
+                got.append(m.value)
+            L.mv[q], L.sad[q], L.flags[q] = got
+        self.links = L
+        self.mv = torch.as_tensor(_DevView(self.mv_ptr, cells * 2, "<i2"), device="cuda").view(
+            self.n_pairs, self.mby, self.mbx, 2)
+        self.sad = torch.as_tensor(_DevView(self.sad_ptr, cells, "<i4"), device="cuda").view(
+            self.n_pairs, self.mby, self.mbx)
+        dist.barrier()
+
+    def needed_rows(self, f: int) -> tuple[int, int]:
+        """Rows [r0, r1) of global frame f this rank's range reads (empty: (0, 0)): as the
+        reference of pair f (band rows with the R-row halo) and as the current frame of pair f - 1."""
+        from . import partition
+        lo, hi = self.height, 0
+        for p, r0, r1 in self.pieces:
+            if p == f:  # ref
+                a, b = partition.me_band_rows(r0, r1, self.height, self.range)
+                lo, hi = min(lo, a), max(hi, b)
+            if p + 1 == f:  # cur
+                lo, hi = min(lo, 16 * r0), max(hi, 16 * r1)
+        return (lo, hi) if lo < hi else (0, 0)
+
+    def load_frames(self, frame_fn):
+        """Fill the needed rows of this rank's frames from frame_fn(f) -> host uint8 [H, >= W]."""
+        import torch
+        for k in range(self.frames.shape[0]):
+            f = self.pair_base + k
+            r0, r1 = self.needed_rows(f)
+            if r1 > r0:
+                fr = np.ascontiguousarray(np.asarray(frame_fn(f))[r0:r1, : self.width])
+                self.frames[k, r0:r1, : self.width].copy_(torch.from_numpy(fr))
+
+    def run(self, stream=None):
+        """Search this rank's range; every rank's results land in every rank's mv / sad
+        (stream-ordered: the stream waits for all ranks).  Returns (mv, sad)."""
+        self.links.epoch += 1
+        ref, cur = self.frames[:-1], self.frames[1:]
+        _check(lib.sp_me_sad_search_gather(ctypes.byref(self.links), _ptr(ref), _ptr(cur), self.frames.stride(1),
+                                           self.width, self.height, ref.shape[0], self.frames.stride(0),
+                                           self.pair_base, self.range, self.flat_begin, self.flat_end,
+                                           _stream(stream)), "sp_me_sad_search_gather")
+        return self.mv, self.sad
+
+    def close(self):
+        import torch
+        import torch.distributed as dist
+        torch.cuda.synchronize()
+        dist.barrier()
+        for q in self._mapped:
+            lib.sp_ipc_close_handle(vp(q))
+        self._mapped = []
+        dist.barrier()
+        for q in self._own:
+            lib.sp_device_free(vp(q))
+        self._own = []
+
+
 class MESearchHost:
     """Reusable device staging for the end-to-end host-buffer search (sp_me_search_host): the
     frame buffer and ready flags on the device, the outputs in pinned host memory (the kernel
@@ -706,6 +873,18 @@ class Comm:
     def allgather(self, send, recv, stream=None):
         nbytes = send.numel() * send.element_size()
         _check(lib.sp_allgather(self.handle, _ptr(send), _ptr(recv), nbytes, _stream(stream)), "sp_allgather")
+
+    def me_sad_search_dist(self, frames, width: int, frame_height: int, search_range: int, ranges, pair_base: int,
+                           mv, sad, stream=None):
+        """NCCL baseline of MEShard.run: this rank's range (ranges[rank]) searched into the
+        global mv / sad, then grouped ncclBroadcasts (every rank roots its range)."""
+        ref, cur = frames[:-1], frames[1:]
+        fr = (i64 * (2 * len(ranges)))(*[int(v) for r in ranges for v in r])
+        _check(lib.sp_me_sad_search_dist(self.handle, _ptr(ref), _ptr(cur), frames.stride(1), int(width),
+                                         int(frame_height), ref.shape[0], frames.stride(0), int(pair_base),
+                                         int(search_range), fr, _ptr(mv), _ptr(sad), _stream(stream)),
+               "sp_me_sad_search_dist")
+        return mv, sad
 
     def async_error(self) -> int:
         """ncclCommGetAsyncError of this communicator (0 = healthy, 7 = in progress)."""
@@ -794,6 +973,8 @@ class PeerSlab:
             tiles = jacobi1d_plan(self.n_local, max(1, int(steps)), self.time_tile, self.space_tile)["tiles"]
             need = tiles + 1 + 2 * passes
             if self._flags is None or self._flags.numel() < need:
+                if self._flags is not None and stream is not None:  # the old block may still be in use there
+                    self._flags.record_stream(stream if not isinstance(stream, int) else torch.cuda.ExternalStream(stream))
                 self._flags = torch.empty(need, dtype=torch.int32, device="cuda")
             _check(lib.sp_jacobi1d_timetiled_peer_fused(ctypes.byref(self.links), vp(self.a_ptr), vp(self.w_ptr),
                                                         _ptr(self._flags), self._flags.numel(), self.n_global,

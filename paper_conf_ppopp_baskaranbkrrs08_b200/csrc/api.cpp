@@ -30,7 +30,7 @@ extern "C" int sp_abi_struct_sizes(int64_t* out, int32_t n) {
     const int64_t sz[] = {sizeof(sp_domain),      sizeof(sp_ref),         sizeof(sp_block),      sizeof(sp_plan_opts),
                           sizeof(sp_buffer),      sizeof(sp_jacobi_plan), sizeof(sp_peer_links), sizeof(sp_tile_problem),
                           sizeof(sp_tile_result), sizeof(sp_op),          sizeof(sp_stmt_body),  sizeof(sp_array_desc),
-                          sizeof(sp_exec_opts),   sizeof(sp_exec_stats)};
+                          sizeof(sp_exec_opts),   sizeof(sp_exec_stats), sizeof(sp_me_gather_links)};
     const int32_t k = (int32_t)(sizeof(sz) / sizeof(sz[0]));
     for (int32_t i = 0; out && i < n && i < k; ++i) out[i] = sz[i];
     return k;

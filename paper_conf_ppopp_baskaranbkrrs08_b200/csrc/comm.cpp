@@ -42,6 +42,7 @@ struct Nccl {
     ncclResult_t (*GroupEnd)() = nullptr;
     ncclResult_t (*AllGather)(const void*, void*, size_t, ncclDataType_t, ncclComm_t, cudaStream_t) = nullptr;
     ncclResult_t (*CommGetAsyncError)(ncclComm_t, ncclResult_t*) = nullptr;
+    ncclResult_t (*Broadcast)(const void*, void*, size_t, ncclDataType_t, int, ncclComm_t, cudaStream_t) = nullptr;
 };
 
 Nccl& nccl() {
@@ -63,6 +64,7 @@ Nccl& nccl() {
         SP_SYM(GroupEnd, "ncclGroupEnd");
         SP_SYM(AllGather, "ncclAllGather");
         SP_SYM(CommGetAsyncError, "ncclCommGetAsyncError");
+        SP_SYM(Broadcast, "ncclBroadcast");
 #undef SP_SYM
         n.ok = n.GetUniqueId && n.CommInitRank && n.CommDestroy && n.Send && n.Recv && n.GroupStart && n.GroupEnd &&
                n.AllGather;
@@ -273,4 +275,35 @@ extern "C" int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_loc
         }
         return SP_OK;
     });
+}
+
+extern "C" int sp_me_sad_search_dist(sp_comm* c, const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                                     int32_t frame_height, int32_t n_pairs_buffer, int64_t pair_stride,
+                                     int32_t pair_base, int32_t range, const int64_t* flat_ranges, int16_t* mv,
+                                     uint32_t* best_sad, void* stream) {
+    SP_NVTX("sp_me_sad_search_dist");
+    if (!c || !flat_ranges || !mv || !best_sad) return SP_ERR_INVALID_ARG;
+    for (int q = 0; q < c->nranks; ++q)
+        if (flat_ranges[2 * q] > flat_ranges[2 * q + 1] || (q > 0 && flat_ranges[2 * q] != flat_ranges[2 * q - 1]))
+            return SP_ERR_INVALID_ARG;
+    int st = sp_me_sad_search_range(ref, cur, pitch, width, frame_height, n_pairs_buffer, pair_stride, pair_base, range,
+                                    flat_ranges[2 * c->rank], flat_ranges[2 * c->rank + 1], mv, best_sad, stream);
+    if (st) return st;
+    if (c->nranks == 1) return SP_OK;
+    Nccl& n = nccl();
+    if (!n.Broadcast) {
+        sp::set_nccl_error((int)ncclSystemError);
+        return SP_ERR_NCCL;
+    }
+    const int64_t mbx = width / 16;
+    const cudaStream_t s = (cudaStream_t)stream;
+    SP_NCCL_TRY(n.GroupStart());
+    for (int q = 0; q < c->nranks; ++q) {
+        const int64_t off = flat_ranges[2 * q] * mbx, cnt = (flat_ranges[2 * q + 1] - flat_ranges[2 * q]) * mbx;
+        if (cnt == 0) continue;
+        SP_NCCL_TRY(n.Broadcast(mv + 2 * off, mv + 2 * off, (size_t)(4 * cnt), ncclUint8, q, c->comm, s));
+        SP_NCCL_TRY(n.Broadcast(best_sad + off, best_sad + off, (size_t)(4 * cnt), ncclUint8, q, c->comm, s));
+    }
+    SP_NCCL_TRY(n.GroupEnd());
+    return SP_OK;
 }

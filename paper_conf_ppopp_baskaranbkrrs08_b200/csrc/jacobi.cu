@@ -525,7 +525,15 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     auto issue = [&](int64_t t, int pass, int s) {  // lane 0 only
         int64_t x0, st, lo, hi;
         tile_range(t, x0, st, lo, hi);
-        if (pers) fence_proxy_async_global();  // observed flags -> the async-proxy read below
+        if (pers) {
+#ifndef SP_JAC_NO_ACQ
+            // the dependence flags were observed by relaxed loads (cheap polling); one
+            // acquire fence per tile turns that observation into synchronisation with the
+            // producers' release stores before the move-in reads their cells
+            if (pass > 0) fence_acq_rel_gpu();
+#endif
+            fence_proxy_async_global();  // observed flags -> the async-proxy read below
+        }
         const unsigned long long ep = kPeer && pers ? A.epoch + (unsigned long long)pass : A.epoch;
         if (A.wait_left && lo < A.own_begin) {   // halo from the left neighbour (peer store)
             wait_epoch(A.wait_left, ep);
@@ -794,8 +802,12 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         __syncwarp();
         {
             const int64_t n16 = st & ~int64_t(3);
-            if (lane == 0 && n16 > 0) {
-                tma_store_1d(dst + (x0 - A.g0), buf + A.H, (uint32_t)(n16 * 4));
+            // one bulk group per tile, empty when the tile owns < 4 cells: publish() counts
+            // groups (wait_group 1 = every tile but the newest has landed), so a tile without
+            // a store must still close a group or the previous tile's store would be taken
+            // for the newest one and published before it completed
+            if (lane == 0) {
+                if (n16 > 0) tma_store_1d(dst + (x0 - A.g0), buf + A.H, (uint32_t)(n16 * 4));
                 bulk_commit();
             }
             if (lane < st - n16) dst[x0 - A.g0 + n16 + lane] = buf[A.H + n16 + lane];

@@ -26,8 +26,10 @@
 #include <cuda_runtime.h>
 
 #include <cstdint>
+#include <algorithm>
 #include <cstdlib>
 #include <mutex>
+#include <unordered_map>
 
 #include "../../include/sp.h"
 #include "sm100_ptx.cuh"
@@ -80,10 +82,31 @@ struct MeArgs {
     // move-in of a macroblock waits for its pair's flag
     const int32_t* ready;
     // dynamic macroblock distribution: CTA c takes macroblock c first, then the next index
-    // from this counter (zeroed before the launch) + gridDim.x.  Co-resident CTAs progress at
+    // from this counter (zero at launch, reset by the last CTA) + gridDim.x.  Co-resident CTAs progress at
     // very different rates (measured: the first of four CTAs on an SM finished after 2.8 ms,
     // the last after 8.8 ms under a static assignment), so static shares left SMs idle.
     uint32_t* counter;
+    // Range mode (sp_me_sad_search_range / _gather; 0 otherwise): macroblock mb of the launch is
+    // global macroblock mb + flat_mb0 of the (pair, MB row, MB column) space of the whole
+    // batch (mb_rows = all MB rows of a frame), outputs are indexed globally, and the tensor
+    // maps address pair `pair - pair_base` (the buffer holds frames from pair_base on).
+    uint32_t flat_mb0;
+    int32_t pair_base;
+    uint32_t total_mb;  // macroblocks of this launch (fast kernel)
+};
+
+// Fused all-gather of the results over peer memory (sp_me_sad_search_gather): every
+// macroblock's (MV, SAD) is stored into the output arrays of every rank (NVLink / CUDA-IPC
+// mapped pointers) by the thread that computes it.  Flags: each rank owns u64 flags[2 * nranks]
+// = ready[q] (rank q may write into this rank's outputs for epoch e) and done[q] (rank q's
+// results of epoch e have all landed here).
+constexpr int kMaxGatherRanks = 8;
+struct GatherArgs {
+    int16_t* mv[kMaxGatherRanks];                 // [q]: rank q's mv array (own one included)
+    uint32_t* sad[kMaxGatherRanks];
+    unsigned long long* flags[kMaxGatherRanks];  // [q]: rank q's flags (mapped)
+    int32_t nranks, rank;
+    unsigned long long epoch;
 };
 
 __device__ __forceinline__ uint64_t make_key(uint32_t s, int dx, int dy, int R) {
@@ -165,10 +188,17 @@ __device__ __noinline__ void wait_ready(const int32_t* flag) {
     fence_proxy_async_global();
 }
 
-template <int R, bool kStream>
+// kMode: kPlain (device-resident frames), kStream (frames still streaming in: ready flags),
+// kGather (results all-gathered into every rank's outputs over peer memory).  Separate
+// instantiations keep the common path's register and uniform-datapath layout untouched.
+enum { kPlain = 0, kStreamed = 1, kGather = 2 };
+
+template <int R, int kMode>
 __global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
-me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A) {
+me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A,
+              const __grid_constant__ GatherArgs X) {
     using G = MeGeom<R>;
+    constexpr bool kStream = kMode == kStreamed;
     constexpr int win = G::kWin;
     constexpr int side = 2 * R + 1;
     constexpr int nwarps = G::kWarps;
@@ -182,7 +212,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
     const uint32_t mbx = (uint32_t)A.mbx;
     const uint32_t per_pair = (uint32_t)A.mb_rows * mbx;
-    const uint32_t total = per_pair * (uint32_t)A.n_pairs;  // host guarantees < 2^31
+    const uint32_t total = A.total_mb;  // host guarantees < 2^31
     const uint32_t Gs = gridDim.x;
     const int W = A.width, Hf = A.frame_height;
     // byte phase ph of stage st (ph = 0: the TMA'd window).  Copy ph starts 32*ph bytes past
@@ -194,6 +224,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         int pair, byr, bx;
     };
     auto locate = [&](uint32_t mb) -> Pos {
+        mb += A.flat_mb0;
         const uint32_t pair = mb / per_pair, rem = mb - pair * per_pair;
         const uint32_t byr = rem / mbx;
         return Pos{(int)pair, (int)byr, (int)(rem - byr * mbx)};
@@ -203,9 +234,12 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         if (kStream) wait_ready(A.ready + q.pair);
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         mbar_arrive_expect_tx(&full[st], (uint32_t)(G::kCopy + kMB * kMB));
-        tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair, &full[st]);
-        tma_load_3d(smem + G::kOffCur + st * 256, &cur_map, x0 + A.pad, y0 - A.row0 + A.pad, q.pair, &full[st]);
+        tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair - A.pair_base,
+                    &full[st]);
+        tma_load_3d(smem + G::kOffCur + st * 256, &cur_map, x0 + A.pad, y0 - A.row0 + A.pad, q.pair - A.pair_base,
+                    &full[st]);
     };
+    bool gather_armed = false;  // (kGather, finalizing thread) every rank's ready flag seen for this epoch
     // publish macroblock mbp's argmin from stage sp (every warp's key + the corner candidate)
     auto finalize = [&](uint32_t mbp, int sp) {
         uint32_t b = red32[sp][0];
@@ -221,8 +255,27 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const int dy = (int)((tie >> 1) & 127) - R;
         const int adx = (int)((tie >> 8) & 127) - abs(dy);
         // (dx, dy) as one 32-bit store (the outputs may be mapped host memory: fewer PCIe writes)
-        *reinterpret_cast<uint32_t*>(A.mv + 2 * idx) = (uint32_t)(uint16_t)((tie & 1) ? adx : -adx) | ((uint32_t)(uint16_t)dy << 16);
+        const uint32_t mvw = (uint32_t)(uint16_t)((tie & 1) ? adx : -adx) | ((uint32_t)(uint16_t)dy << 16);
+        *reinterpret_cast<uint32_t*>(A.mv + 2 * idx) = mvw;
         A.sad[idx] = sad;
+        if constexpr (kMode == kGather) {
+            // all-gather: the same 8 bytes into every other rank's outputs (peer stores), once
+            // those ranks have announced (ready) that their outputs of the previous epoch are free
+            if (!gather_armed) {
+                const long long t0 = clock64();
+                for (int q = 0; q < X.nranks; ++q)
+                    while (ld_acquire_sys(X.flags[X.rank] + q) < X.epoch) {
+                        __nanosleep(128);
+                        if (clock64() - t0 > (40ll << 30)) __trap();
+                    }
+                gather_armed = true;
+            }
+            for (int q = 0; q < X.nranks; ++q) {
+                if (q == X.rank) continue;
+                *reinterpret_cast<uint32_t*>(X.mv[q] + 2 * idx) = mvw;
+                X.sad[q][idx] = sad;
+            }
+        }
         if (A.surface) A.surface[idx * side * side + (size_t)side * side - 1] = lvalid ? lsad : 0xffffffffu;
     };
 
@@ -234,6 +287,11 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         g_me_cta[blockIdx.x][1] = globaltimer();
     }
 #endif
+    if (kMode == kGather && blockIdx.x == 0 && tid == 0) {
+        // this rank's outputs of the previous epoch are no longer read (stream order): let
+        // every rank write this epoch's results into them
+        for (int q = 0; q < X.nranks; ++q) st_release_sys(X.flags[q] + X.rank, X.epoch);
+    }
     if (tid == 0) {
         prefetch_tmap(&ref_map);
         prefetch_tmap(&cur_map);
@@ -501,6 +559,25 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
 #endif
     __syncthreads();
     if (tid == G::kThreads - 32 && it > 0) finalize(prev_mb, (it - 1) & 1);
+    if (kMode == kGather) __syncthreads();  // the last finalize's peer stores precede the fence below
+    if (tid == 0) {
+        // self-resetting counter: every grab of this CTA precedes its arrival here, so the
+        // last CTA to arrive sees all of them done and zeroes both words for the next launch
+        // on this stream (no per-launch memset)
+        if (kMode == kGather) __threadfence_system();
+        else __threadfence();
+        if (atomicAdd(A.counter + 1, 1u) == Gs - 1) {
+            if (kMode == kGather) {
+                // every CTA's results are out (each fenced before its arrival): tell every rank
+                __threadfence_system();
+                for (int q = 0; q < X.nranks; ++q) st_release_sys(X.flags[q] + X.nranks + X.rank, X.epoch);
+            } else {
+                __threadfence();
+            }
+            A.counter[0] = 0;
+            A.counter[1] = 0;
+        }
+    }
 #if SP_ME_EXP & 32
     if (tid == 0 && blockIdx.x < 4096) g_me_cta[blockIdx.x][2] = globaltimer();
 #endif
@@ -602,54 +679,113 @@ int make_map(CUtensorMap* m, const uint8_t* base, int32_t width, int32_t rows, i
 
 bool fast_range(int R) { return R == 16 || R == 32; }
 
-// The fast kernel's macroblock counter: one slot of a small per-device ring (library-owned,
-// allocated once), zeroed on the launch stream; concurrent launches on different streams
-// take different slots.
+// The fast kernel's macroblock counter: two words (grab counter, CTAs finished) per
+// (device, stream), library-owned, zero between launches (the kernel resets them: see the end
+// of me_sad_kernel), so launches on one stream reuse their slot and launches on different
+// streams never share one.  A stream handle is assumed not to be destroyed and recreated
+// while a launch on it is still running.
+constexpr int kMaxDev = 64;
 int counter_slot(cudaStream_t s, uint32_t** out) {
     constexpr int kSlots = 4096;
     static std::mutex mu;
-    static uint32_t* ring[64] = {};
-    static uint32_t next[64] = {};
+    static uint32_t* pool[kMaxDev] = {};
+    static std::unordered_map<cudaStream_t, uint32_t*>* slots[kMaxDev] = {};
     int dev = 0;
     SP_CUDA_TRY(cudaGetDevice(&dev));
-    uint32_t* slot;
-    {
-        std::lock_guard<std::mutex> lk(mu);
-        if (!ring[dev & 63]) {
-            void* p = nullptr;
-            SP_CUDA_TRY(cudaMalloc(&p, kSlots * sizeof(uint32_t)));
-            ring[dev & 63] = static_cast<uint32_t*>(p);
-        }
-        slot = ring[dev & 63] + (next[dev & 63]++ % kSlots);
+    if (dev < 0 || dev >= kMaxDev) return SP_ERR_UNSUPPORTED;
+    std::lock_guard<std::mutex> lk(mu);
+    if (!pool[dev]) {
+        void* p = nullptr;
+        SP_CUDA_TRY(cudaMalloc(&p, 2 * kSlots * sizeof(uint32_t)));
+        SP_CUDA_TRY(cudaMemset(p, 0, 2 * kSlots * sizeof(uint32_t)));
+        pool[dev] = static_cast<uint32_t*>(p);
+        slots[dev] = new std::unordered_map<cudaStream_t, uint32_t*>();
     }
-    SP_CUDA_TRY(cudaMemsetAsync(slot, 0, sizeof(uint32_t), s));
-    *out = slot;
+    auto it = slots[dev]->find(s);
+    if (it == slots[dev]->end()) {
+        if (slots[dev]->size() >= (size_t)kSlots) return SP_ERR_CAPACITY;  // > 4096 distinct streams
+        it = slots[dev]->emplace(s, pool[dev] + 2 * slots[dev]->size()).first;
+    }
+    *out = it->second;
     return SP_OK;
 }
 
-template <int R, bool kStream>
-int launch_fast(const CUtensorMap& rm, const CUtensorMap& cm, const MeArgs& a, int64_t total, cudaStream_t s) {
+// Per-device launch state of one fast-kernel instantiation: grid cap (occupancy x SMs) and
+// the shared-memory attribute, set once per device (the attribute is per device context).
+template <int R, int kMode>
+int fast_grid_cap(int* cap) {
     using G = MeGeom<R>;
-    static int grid_cap = 0;
-    static std::once_flag once;
-    static cudaError_t err = cudaSuccess;
-    std::call_once(once, [] {
-        int dev = 0, sms = 0, occ = 0;
-        err = cudaGetDevice(&dev);
-        if (err == cudaSuccess) err = cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev);
-        if (err == cudaSuccess)
-            err = cudaFuncSetAttribute(me_sad_kernel<R, kStream>, cudaFuncAttributeMaxDynamicSharedMemorySize, G::kSmem);
-        if (err == cudaSuccess)
-            err = cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, me_sad_kernel<R, kStream>, G::kThreads, G::kSmem);
-        grid_cap = sms * (occ > 0 ? occ : 1);
+    static std::mutex mu;
+    static int caps[kMaxDev] = {};
+    int dev = 0;
+    SP_CUDA_TRY(cudaGetDevice(&dev));
+    if (dev < 0 || dev >= kMaxDev) return SP_ERR_UNSUPPORTED;
+    std::lock_guard<std::mutex> lk(mu);
+    if (!caps[dev]) {
+        int sms = 0, occ = 0;
+        SP_CUDA_TRY(cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, dev));
+        SP_CUDA_TRY(cudaFuncSetAttribute(me_sad_kernel<R, kMode>, cudaFuncAttributeMaxDynamicSharedMemorySize, G::kSmem));
+        SP_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&occ, me_sad_kernel<R, kMode>, G::kThreads, G::kSmem));
+        int c = sms * (occ > 0 ? occ : 1);
         // SP_ME_GRID_CAP (sanitizer runs): a few CTAs then walk many macroblocks each, so
         // racecheck sees both pipeline stages in use within one CTA
         if (const char* e = std::getenv("SP_ME_GRID_CAP"))
-            if (std::atoi(e) > 0 && std::atoi(e) < grid_cap) grid_cap = std::atoi(e);
-    });
-    SP_CUDA_TRY(err);
+            if (std::atoi(e) > 0 && std::atoi(e) < c) c = std::atoi(e);
+        caps[dev] = c;
+    }
+    *cap = caps[dev];
+    return SP_OK;
+}
+
+template <int R, int kMode>
+int launch_fast(const CUtensorMap& rm, const CUtensorMap& cm, const MeArgs& a, const GatherArgs& x, int64_t total,
+                cudaStream_t s) {
+    using G = MeGeom<R>;
+    int grid_cap = 0;
+    int st = fast_grid_cap<R, kMode>(&grid_cap);
+    if (st) return st;
     const int grid = (int)(total < grid_cap ? total : grid_cap);
-    me_sad_kernel<R, kStream><<<grid, G::kThreads, G::kSmem, s>>>(rm, cm, a);
+    me_sad_kernel<R, kMode><<<grid, G::kThreads, G::kSmem, s>>>(rm, cm, a, x);
+    return SP_OK;
+}
+
+// Encoded tensor maps, cached per (device, base, geometry): encoding is pure host work (a few
+// us per map); the map holds only the address and the geometry, so a freed-and-reused address
+// with the same geometry yields the same map — no stale entries are possible.
+struct MapKey {
+    int dev;
+    const void* base;
+    int64_t w, rows, pairs, pitch, stride, bw, bh;
+    bool operator==(const MapKey& o) const {
+        return dev == o.dev && base == o.base && w == o.w && rows == o.rows && pairs == o.pairs && pitch == o.pitch &&
+               stride == o.stride && bw == o.bw && bh == o.bh;
+    }
+};
+int cached_map(CUtensorMap* m, const uint8_t* base, int32_t width, int32_t rows, int32_t n_pairs, int64_t pitch,
+               int64_t pair_stride, uint32_t box_w, uint32_t box_h) {
+    constexpr int kEntries = 32;
+    static std::mutex mu;
+    static MapKey keys[kEntries];
+    static CUtensorMap maps[kEntries];
+    static int used = 0, next = 0;
+    int dev = 0;
+    SP_CUDA_TRY(cudaGetDevice(&dev));
+    const MapKey k{dev, base, width, rows, n_pairs, pitch, pair_stride, box_w, box_h};
+    {
+        std::lock_guard<std::mutex> lk(mu);
+        for (int i = 0; i < used; ++i)
+            if (keys[i] == k) {
+                *m = maps[i];
+                return SP_OK;
+            }
+    }
+    int st = make_map(m, base, width, rows, n_pairs, pitch, pair_stride, box_w, box_h);
+    if (st) return st;
+    std::lock_guard<std::mutex> lk(mu);
+    keys[next] = k;
+    maps[next] = *m;
+    next = (next + 1) % kEntries;
+    if (used < kEntries) ++used;
     return SP_OK;
 }
 
@@ -694,39 +830,164 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
     if (n_pairs == 0 || rows == 0 || mbx == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
     MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, pad,
-             pad > 0 ? 1 : 0, mv, best_sad, surface, ready, nullptr};
+             pad > 0 ? 1 : 0, mv, best_sad, surface, ready, nullptr, 0u, 0, 0u};
+    const GatherArgs nox{};
     if (fast_range(range)) {
         int st0;
         if ((st0 = counter_slot(s, &a.counter))) return st0;
         CUtensorMap rm, cm;
         int st;
         const int64_t ps = n_pairs > 1 ? pair_stride : pitch * rows_in_buffer;
-        if ((st = make_map(&rm, ref, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, (uint32_t)a.win, (uint32_t)a.win)))
+        if ((st = cached_map(&rm, ref, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, (uint32_t)a.win,
+                             (uint32_t)a.win)))
             return st;
-        if ((st = make_map(&cm, cur, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, kMB, kMB))) return st;
+        if ((st = cached_map(&cm, cur, width + 2 * pad, rows_in_buffer, n_pairs, pitch, ps, kMB, kMB))) return st;
         a.n_pairs = n_pairs;
         const int64_t total = (int64_t)mbx * rows * n_pairs;
         if (total >= (int64_t(1) << 31)) return SP_ERR_UNSUPPORTED;  // 32-bit macroblock indices in the kernel
+        a.total_mb = (uint32_t)total;
         // (the streamed-frames variant is a separate instantiation: the flag wait in its move-in
         // costs the device-resident kernel its uniform-datapath index math, 2 % of M4)
-        if (range == 32) st = ready ? launch_fast<32, true>(rm, cm, a, total, s) : launch_fast<32, false>(rm, cm, a, total, s);
-        else st = ready ? launch_fast<16, true>(rm, cm, a, total, s) : launch_fast<16, false>(rm, cm, a, total, s);
+        if (range == 32)
+            st = ready ? launch_fast<32, kStreamed>(rm, cm, a, nox, total, s) : launch_fast<32, kPlain>(rm, cm, a, nox, total, s);
+        else
+            st = ready ? launch_fast<16, kStreamed>(rm, cm, a, nox, total, s) : launch_fast<16, kPlain>(rm, cm, a, nox, total, s);
         if (st) return st;
     } else {
         const int smem = a.win * a.win + kMB * kMB;
-        static std::once_flag once;
-        static cudaError_t attr_err = cudaSuccess;
-        std::call_once(once, [] {
-            attr_err = cudaFuncSetAttribute(me_sad_generic_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 142 * 142 + 256);
-        });
-        SP_CUDA_TRY(attr_err);
+        {  // the shared-memory attribute is per device: set it once on each
+            static std::mutex mu;
+            static bool set[kMaxDev] = {};
+            int dev = 0;
+            SP_CUDA_TRY(cudaGetDevice(&dev));
+            if (dev < 0 || dev >= kMaxDev) return SP_ERR_UNSUPPORTED;
+            std::lock_guard<std::mutex> lk(mu);
+            if (!set[dev]) {
+                SP_CUDA_TRY(cudaFuncSetAttribute(me_sad_generic_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                                                 142 * 142 + 256));
+                set[dev] = true;
+            }
+        }
         me_sad_generic_kernel<<<dim3(mbx, rows, n_pairs), 256, smem, s>>>(ref, cur, pitch, rows_in_buffer, n_pairs > 1 ? pair_stride : 0, a);
     }
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }
 
+// Range mode: the macroblocks of flat (pair, MB row) rows [flat_begin, flat_end) of a batch,
+// full frames in the buffers (pair p at + (p - pair_base) * pair_stride), outputs indexed
+// globally.  gx != nullptr: results also stored into every rank's outputs (fused all-gather).
+int me_range_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width, int32_t frame_height,
+                  int32_t n_pairs_buffer, int64_t pair_stride, int32_t pair_base, int32_t range, int64_t flat_begin,
+                  int64_t flat_end, int16_t* mv, uint32_t* best_sad, void* stream, const GatherArgs* gx) {
+    if (!ref || !cur || !mv || !best_sad || (reinterpret_cast<uintptr_t>(mv) & 3) ||
+        (reinterpret_cast<uintptr_t>(best_sad) & 3))
+        return SP_ERR_INVALID_ARG;
+    if (range < 0 || range > 63 || width < kMB || frame_height < kMB || n_pairs_buffer < 0 || pair_base < 0)
+        return SP_ERR_INVALID_ARG;
+    if (pitch < width || (pitch & 15) || (pair_stride & 15) || (reinterpret_cast<uintptr_t>(ref) & 15) ||
+        (reinterpret_cast<uintptr_t>(cur) & 15))
+        return SP_ERR_INVALID_ARG;
+    if (n_pairs_buffer > 1 && pair_stride < pitch * frame_height) return SP_ERR_INVALID_ARG;
+    const int64_t mbx = width / kMB, mby = frame_height / kMB;
+    if (flat_begin > flat_end ||
+        (flat_end > flat_begin &&
+         (flat_begin < (int64_t)pair_base * mby || flat_end > (int64_t)(pair_base + n_pairs_buffer) * mby)))
+        return SP_ERR_INVALID_ARG;
+    if ((int64_t)(pair_base + n_pairs_buffer) * mby * mbx >= (int64_t(1) << 31)) return SP_ERR_UNSUPPORTED;
+    if (gx && !fast_range(range)) return SP_ERR_UNSUPPORTED;
+    const cudaStream_t s = (cudaStream_t)stream;
+    if (flat_end == flat_begin || mbx == 0) {
+        if (!gx) return SP_OK;  // (an empty range still takes part in the gather protocol)
+    }
+    const int64_t ps = n_pairs_buffer > 1 ? pair_stride : pitch * frame_height;
+    if (!fast_range(range)) {
+        // generic kernel: one launch per (pair, MB-row band) piece of the range
+        for (int64_t f = flat_begin; f < flat_end;) {
+            const int64_t p = f / mby, r0 = f % mby, r1 = std::min<int64_t>(mby, r0 + (flat_end - f));
+            const int64_t o = (p * mby + r0) * mbx;
+            int st = me_search_impl(ref + (p - pair_base) * ps, cur + (p - pair_base) * ps, pitch, width, frame_height,
+                                    0, frame_height, 1, ps, kMB, range, (int32_t)r0, (int32_t)r1, mv + 2 * o,
+                                    best_sad + o, nullptr, stream, 0);
+            if (st) return st;
+            f += r1 - r0;
+        }
+        return SP_OK;
+    }
+    MeArgs a{width, frame_height, 0, range, n_pairs_buffer, (int32_t)mbx, 0, (int32_t)mby, 2 * range + 16, 0, 0,
+             mv, best_sad, nullptr, nullptr, nullptr, (uint32_t)(flat_begin * mbx), pair_base,
+             (uint32_t)((flat_end - flat_begin) * mbx)};
+    int st;
+    if ((st = counter_slot(s, &a.counter))) return st;
+    CUtensorMap rm, cm;
+    const int32_t np = n_pairs_buffer > 0 ? n_pairs_buffer : 1;
+    if ((st = cached_map(&rm, ref, width, frame_height, np, pitch, ps, (uint32_t)a.win, (uint32_t)a.win))) return st;
+    if ((st = cached_map(&cm, cur, width, frame_height, np, pitch, ps, kMB, kMB))) return st;
+    int64_t total = (int64_t)a.total_mb;
+    if (gx) {
+        if (total == 0) {  // nothing to search: a one-CTA launch still arms and signals the gather
+            total = 1;
+            a.total_mb = 0;
+        }
+        st = range == 32 ? launch_fast<32, kGather>(rm, cm, a, *gx, total, s) : launch_fast<16, kGather>(rm, cm, a, *gx, total, s);
+    } else {
+        const GatherArgs nox{};
+        st = range == 32 ? launch_fast<32, kPlain>(rm, cm, a, nox, total, s) : launch_fast<16, kPlain>(rm, cm, a, nox, total, s);
+    }
+    if (st) return st;
+    SP_CUDA_TRY(cudaGetLastError());
+    return SP_OK;
+}
+
+__global__ void me_gather_wait_kernel(const unsigned long long* done, int32_t nranks, unsigned long long epoch) {
+    const int q = threadIdx.x;
+    if (q < nranks) {
+        const long long t0 = clock64();
+        while (ld_acquire_sys(done + q) < epoch) {
+            __nanosleep(256);
+            if (clock64() - t0 > (40ll << 30)) __trap();  // a rank that never arrives: ~20 s
+        }
+    }
+    __syncthreads();
+}
+
 }  // namespace
+
+extern "C" int sp_me_sad_search_range(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
+                                      int32_t frame_height, int32_t n_pairs_buffer, int64_t pair_stride,
+                                      int32_t pair_base, int32_t range, int64_t flat_begin, int64_t flat_end,
+                                      int16_t* mv, uint32_t* best_sad, void* stream) {
+    SP_NVTX("sp_me_sad_search_range");
+    return me_range_impl(ref, cur, pitch, width, frame_height, n_pairs_buffer, pair_stride, pair_base, range,
+                         flat_begin, flat_end, mv, best_sad, stream, nullptr);
+}
+
+extern "C" int sp_me_sad_search_gather(const sp_me_gather_links* L, const uint8_t* ref, const uint8_t* cur,
+                                       int64_t pitch, int32_t width, int32_t frame_height, int32_t n_pairs_buffer,
+                                       int64_t pair_stride, int32_t pair_base, int32_t range, int64_t flat_begin,
+                                       int64_t flat_end, void* stream) {
+    SP_NVTX("sp_me_sad_search_gather");
+    if (!L || L->nranks < 1 || L->nranks > SP_ME_MAX_RANKS || L->rank < 0 || L->rank >= L->nranks || L->epoch < 1)
+        return SP_ERR_INVALID_ARG;
+    static_assert(SP_ME_MAX_RANKS == kMaxGatherRanks, "gather rank limit");
+    GatherArgs x{};
+    for (int q = 0; q < L->nranks; ++q) {
+        if (!L->mv[q] || !L->sad[q] || !L->flags[q]) return SP_ERR_INVALID_ARG;
+        x.mv[q] = L->mv[q];
+        x.sad[q] = L->sad[q];
+        x.flags[q] = L->flags[q];
+    }
+    x.nranks = L->nranks;
+    x.rank = L->rank;
+    x.epoch = (unsigned long long)L->epoch;
+    int st = me_range_impl(ref, cur, pitch, width, frame_height, n_pairs_buffer, pair_stride, pair_base, range,
+                           flat_begin, flat_end, L->mv[L->rank], L->sad[L->rank], stream, &x);
+    if (st) return st;
+    // the stream continues only when every rank's results have landed in this rank's outputs
+    me_gather_wait_kernel<<<1, 32, 0, (cudaStream_t)stream>>>(L->flags[L->rank] + L->nranks, L->nranks, x.epoch);
+    SP_CUDA_TRY(cudaGetLastError());
+    return SP_OK;
+}
 
 extern "C" int sp_me_sad_search(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
                                 int32_t rows_in_buffer, int32_t row0_global, int32_t frame_height, int32_t n_pairs,
@@ -779,13 +1040,14 @@ const int32_t* pinned_one() {
     return one;
 }
 
-cudaStream_t own_copy_stream() {  // per process; used when the caller passes no copy stream
-    static cudaStream_t cs = nullptr;
-    static std::once_flag once;
-    std::call_once(once, [] {
-        if (cudaStreamCreateWithFlags(&cs, cudaStreamNonBlocking) != cudaSuccess) cs = nullptr;
-    });
-    return cs;
+cudaStream_t own_copy_stream() {  // per device (the current one); used when the caller passes no copy stream
+    static std::mutex mu;
+    static cudaStream_t cs[kMaxDev] = {};
+    int dev = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= kMaxDev) return nullptr;
+    std::lock_guard<std::mutex> lk(mu);
+    if (!cs[dev] && cudaStreamCreateWithFlags(&cs[dev], cudaStreamNonBlocking) != cudaSuccess) cs[dev] = nullptr;
+    return cs[dev];
 }
 }  // namespace
 

@@ -76,7 +76,7 @@ def test_struct_layouts_match_the_library():
     """The binding's ctypes structs have the C ABI's sizes (sp_abi_struct_sizes)."""
     order = [sp.sp_domain, sp.sp_ref, sp.sp_block, sp.sp_plan_opts, sp.sp_buffer, sp.sp_jacobi_plan,
              sp.sp_peer_links, sp.sp_tile_problem, sp.sp_tile_result, sp.sp_op, sp.sp_stmt_body, sp.sp_array_desc,
-             sp.sp_exec_opts, sp.sp_exec_stats]
+             sp.sp_exec_opts, sp.sp_exec_stats, sp.sp_me_gather_links]
     out = (ctypes.c_int64 * len(order))()
     assert sp.lib.sp_abi_struct_sizes(out, len(order)) == len(order)
     for cls, n in zip(order, out):
