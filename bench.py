@@ -371,8 +371,10 @@ def run_ours(args, rank, world, local_rank):
     me_steps = [ev[k][1].elapsed_time(ev[k][2]) for k in range(K)]
     jac_ms, me_ms = sum(jac_steps), sum(me_steps)
     # the median and the best step beside the mean (this rank's events)
-    step_stats = {"jacobi_ms": {"median": round(float(np.median(jac_steps)), 4), "best": round(min(jac_steps), 4)},
-                  "me_ms": {"median": round(float(np.median(me_steps)), 4), "best": round(min(me_steps), 4)}}
+    step_stats = {"jacobi_ms": {"median": round(float(np.median(jac_steps)), 4), "best": round(min(jac_steps), 4),
+                                "steps": [round(x, 4) for x in jac_steps]},
+                  "me_ms": {"median": round(float(np.median(me_steps)), 4), "best": round(min(me_steps), 4),
+                            "steps": [round(x, 4) for x in me_steps]}}
 
     def max_over_ranks(x):
         if world == 1:

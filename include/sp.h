@@ -351,12 +351,16 @@ int sp_get_unique_id(uint8_t out_id[128]);
 int sp_comm_init(sp_comm** out, const uint8_t id[128], int32_t nranks, int32_t rank, int32_t device);
 int sp_comm_destroy(sp_comm* c);
 
-/* Distributed time-tiled Jacobi over contiguous slabs.  Rank r owns global cells
- * [x_begin, x_begin + n_local); a_local/work_local hold [x_begin - H, x_begin + n_local + H)
- * (H = halo of time_tile; cells outside [0, n_global) unused), 16-byte aligned, x_begin a
- * multiple of 4.  Per pass the ranks exchange H halo cells with each neighbour (grouped
- * ncclSend/ncclRecv on `stream`), then run sp_jacobi1d_pass_segment.  On return a_local
- * holds the rank's slab of a^(steps) (and its halos are stale). */
+/* Distributed time-tiled Jacobi over contiguous slabs (NCCL baseline of the fused peer path
+ * below).  Rank r owns global cells [x_begin, x_begin + n_local); a_local/work_local hold
+ * [x_begin - H, x_begin + n_local + H) (H = halo of time_tile; cells outside [0, n_global)
+ * unused), 16-byte aligned, x_begin a multiple of 4.  Per pass: the two edge segments (first /
+ * last H owned cells) run first (sp_jacobi1d_pass_segment), then the next pass's halo exchange
+ * (grouped ncclSend/ncclRecv of H cells with each neighbour) runs on the communicator's side
+ * stream while the interior segment computes on `stream`; the next pass waits for the exchange.
+ * Slabs shorter than 3H run whole, exchange after.  The communicator's asynchronous error is
+ * checked after every exchange (SP_ERR_NCCL).  On return (stream-ordered) a_local holds the
+ * rank's slab of a^(steps) (its halos are stale). */
 int sp_jacobi1d_timetiled_dist(sp_comm* c, float* a_local, float* work_local, int64_t n_global,
                                int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
                                int32_t space_tile, void* stream);
@@ -474,6 +478,11 @@ int sp_ipc_close_handle(void* ptr);
  * (ncclCommGetAsyncError; ncclSuccess = 0, ncclInProgress = 7, anything else = the
  * communicator failed and must be destroyed).  Host call, does not synchronize. */
 int sp_comm_async_error(sp_comm* c, int32_t* nccl_result);
+/* Wait for `stream` with a deadline while polling the communicator's asynchronous error; on
+ * an NCCL error, or when timeout_ms elapses first (a peer died or hangs), the communicator
+ * is aborted (ncclCommAbort) and SP_ERR_NCCL returned (sp_last_nccl_error: the NCCL result,
+ * ncclInProgress = 7 for the timeout); the comm must then only be destroyed.  Host call. */
+int sp_comm_sync(sp_comm* c, void* stream, int64_t timeout_ms);
 
 /* ncclAllGather of `bytes` per rank (device buffers) — used for the ME results. */
 int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t bytes, void* stream);

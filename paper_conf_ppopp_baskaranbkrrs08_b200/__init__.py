@@ -170,6 +170,7 @@ SYMBOLS = {
                                                       ctypes.POINTER(i64), ctypes.POINTER(i64), i32, i32, i32, vp]),
     "sp_allgather": (ctypes.c_int, [vp, vp, vp, i64, vp]),
     "sp_comm_async_error": (ctypes.c_int, [vp, ctypes.POINTER(i32)]),
+    "sp_comm_sync": (ctypes.c_int, [vp, vp, i64]),
     "sp_jacobi1d_untiled": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_tile_search": (ctypes.c_int, [ctypes.POINTER(sp_tile_problem), ctypes.POINTER(sp_tile_result)]),
     "sp_me_sad_search_unrestricted": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i64, i32, i32, vp, vp, vp, vp]),
@@ -885,6 +886,11 @@ class Comm:
                                          int(search_range), fr, _ptr(mv), _ptr(sad), _stream(stream)),
                "sp_me_sad_search_dist")
         return mv, sad
+
+    def sync(self, timeout_ms: int = 60000, stream=None):
+        """Wait for the stream with a deadline (sp_comm_sync): raises SPError(SP_ERR_NCCL) and
+        aborts the communicator on an NCCL failure or when the deadline passes."""
+        _check(lib.sp_comm_sync(self.handle, _stream(stream), int(timeout_ms)), "sp_comm_sync")
 
     def async_error(self) -> int:
         """ncclCommGetAsyncError of this communicator (0 = healthy, 7 = in progress)."""

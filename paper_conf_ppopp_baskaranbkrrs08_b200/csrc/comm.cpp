@@ -15,7 +15,9 @@
 #include <cuda_runtime.h>
 #include <dlfcn.h>
 
+#include <chrono>
 #include <cstdlib>
+#include <thread>
 #include <cstring>
 #include <mutex>
 #include <vector>
@@ -27,6 +29,9 @@
 struct sp_comm {
     ncclComm_t comm = nullptr;
     int32_t rank = 0, nranks = 1, device = 0;
+    cudaStream_t side = nullptr;     // halo exchange of the overlapped pass loop
+    cudaEvent_t ev_edge = nullptr;   // edge tiles of a pass done (main -> side)
+    cudaEvent_t ev_xchg = nullptr;   // halos of the next pass received (side -> main)
 };
 
 namespace {
@@ -43,6 +48,7 @@ struct Nccl {
     ncclResult_t (*AllGather)(const void*, void*, size_t, ncclDataType_t, ncclComm_t, cudaStream_t) = nullptr;
     ncclResult_t (*CommGetAsyncError)(ncclComm_t, ncclResult_t*) = nullptr;
     ncclResult_t (*Broadcast)(const void*, void*, size_t, ncclDataType_t, int, ncclComm_t, cudaStream_t) = nullptr;
+    ncclResult_t (*CommAbort)(ncclComm_t) = nullptr;
 };
 
 Nccl& nccl() {
@@ -65,6 +71,7 @@ Nccl& nccl() {
         SP_SYM(AllGather, "ncclAllGather");
         SP_SYM(CommGetAsyncError, "ncclCommGetAsyncError");
         SP_SYM(Broadcast, "ncclBroadcast");
+        SP_SYM(CommAbort, "ncclCommAbort");
 #undef SP_SYM
         n.ok = n.GetUniqueId && n.CommInitRank && n.CommDestroy && n.Send && n.Recv && n.GroupStart && n.GroupEnd &&
                n.AllGather;
@@ -168,12 +175,23 @@ extern "C" int sp_comm_init(sp_comm** out, const uint8_t id[128], int32_t nranks
         sp::set_nccl_error((int)r);
         return SP_ERR_NCCL;
     }
+    if (cudaStreamCreateWithFlags(&c->side, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaEventCreateWithFlags(&c->ev_edge, cudaEventDisableTiming) != cudaSuccess ||
+        cudaEventCreateWithFlags(&c->ev_xchg, cudaEventDisableTiming) != cudaSuccess) {
+        sp::set_cuda_error((int)cudaGetLastError());
+        n.CommDestroy(c->comm);
+        delete c;
+        return SP_ERR_CUDA;
+    }
     *out = c;
     return SP_OK;
 }
 
 extern "C" int sp_comm_destroy(sp_comm* c) {
     if (!c) return SP_ERR_INVALID_ARG;
+    if (c->side) cudaStreamDestroy(c->side);
+    if (c->ev_edge) cudaEventDestroy(c->ev_edge);
+    if (c->ev_xchg) cudaEventDestroy(c->ev_xchg);
     Nccl& n = nccl();
     if (c->comm && n.ok) {
         ncclResult_t r = n.CommDestroy(c->comm);
@@ -188,6 +206,29 @@ extern "C" int sp_comm_destroy(sp_comm* c) {
     return SP_OK;
 }
 
+namespace {
+// asynchronous NCCL failure of the communicator (anything but success / in progress)
+int check_async(sp_comm* c) {
+    Nccl& n = nccl();
+    if (!n.CommGetAsyncError) return SP_OK;
+    ncclResult_t r = ncclSuccess;
+    SP_NCCL_TRY(n.CommGetAsyncError(c->comm, &r));
+    if (r != ncclSuccess && r != ncclInProgress) {
+        sp::set_nccl_error((int)r);
+        return SP_ERR_NCCL;
+    }
+    return SP_OK;
+}
+}  // namespace
+
+// NCCL baseline of the multi-GPU Jacobi (the fused peer-memory kernel is the product path):
+// per pass the slab's two EDGE segments (the first / last H owned cells — the only cells a
+// neighbour reads) run first, the halo exchange of the next pass (grouped ncclSend/ncclRecv)
+// then runs on a side stream while the INTERIOR segment computes on `stream`, and the next
+// pass waits for the exchange (the per-time-tile synchronisation, here
+// overlapped with the interior work).  Buffer positions: b[j] <-> global x_begin - H + j; the
+// edge / interior kernels write disjoint owned cells, the exchange reads the new edge cells and
+// writes only halo cells, so nothing races.
 extern "C" int sp_jacobi1d_timetiled_dist(sp_comm* c, float* a_local, float* work_local, int64_t n_global,
                                           int64_t x_begin, int64_t n_local, int32_t steps, int32_t time_tile,
                                           int32_t space_tile, void* stream) {
@@ -200,25 +241,96 @@ extern "C" int sp_jacobi1d_timetiled_dist(sp_comm* c, float* a_local, float* wor
     if (steps == 0) return SP_OK;
     Nccl& n = nccl();
     const cudaStream_t s = (cudaStream_t)stream;
-    std::vector<Slab> slabs{{a_local, work_local, x_begin, n_local}};
     const int64_t x_end = x_begin + n_local;
     const int left = (x_begin > 0) ? c->rank - 1 : -1;
     const int right = (x_end < n_global) ? c->rank + 1 : -1;
-    return pass_loop(slabs, n_global, steps, time_tile, space_tile, s, [&](std::vector<float*>& cur) -> int {
+    const int64_t g0 = x_begin - H, len = n_local + 2 * H;
+    auto exchange = [&](float* b, cudaStream_t q) -> int {  // b's halos <- the neighbours' edge cells
         if (left < 0 && right < 0) return SP_OK;
-        float* b = cur[0];  // b[j] <-> global x_begin - H + j
         SP_NCCL_TRY(n.GroupStart());
         if (left >= 0) {
-            SP_NCCL_TRY(n.Send(b + H, H, ncclFloat32, left, c->comm, s));  // my first H owned cells
-            SP_NCCL_TRY(n.Recv(b, H, ncclFloat32, left, c->comm, s));      // left halo
+            SP_NCCL_TRY(n.Send(b + H, H, ncclFloat32, left, c->comm, q));  // my first H owned cells
+            SP_NCCL_TRY(n.Recv(b, H, ncclFloat32, left, c->comm, q));      // left halo
         }
         if (right >= 0) {
-            SP_NCCL_TRY(n.Send(b + n_local, H, ncclFloat32, right, c->comm, s));  // my last H owned
-            SP_NCCL_TRY(n.Recv(b + H + n_local, H, ncclFloat32, right, c->comm, s));
+            SP_NCCL_TRY(n.Send(b + n_local, H, ncclFloat32, right, c->comm, q));  // my last H owned
+            SP_NCCL_TRY(n.Recv(b + H + n_local, H, ncclFloat32, right, c->comm, q));
         }
         SP_NCCL_TRY(n.GroupEnd());
-        return SP_OK;
-    });
+        return check_async(c);
+    };
+    auto segment = [&](float* src, float* dst, int64_t ob, int64_t oe, int32_t h) -> int {
+        if (oe <= ob) return SP_OK;
+        return sp_jacobi1d_pass_segment(src, dst, n_global, g0, len, ob, oe, h, time_tile, space_tile, stream);
+    };
+    // edges split off only when an interior remains (and a neighbour exists)
+    const bool split = (left >= 0 || right >= 0) && n_local >= 3 * (int64_t)H;
+    const int64_t ib = left >= 0 ? x_begin + H : x_begin, ie = right >= 0 ? x_end - H : x_end;
+    float* cur = a_local;
+    float* nxt = work_local;
+    {
+        SP_NVTX("halo exchange");
+        if ((st = exchange(cur, s))) return st;
+    }
+    for (int32_t done = 0; done < steps; done += time_tile) {
+        const int32_t h = steps - done < time_tile ? steps - done : time_tile;
+        const bool more = done + time_tile < steps;
+        if (!split) {
+            if ((st = segment(cur, nxt, x_begin, x_end, h))) return st;
+            if (more && (st = exchange(nxt, s))) return st;
+        } else {
+            if (left >= 0 && (st = segment(cur, nxt, x_begin, x_begin + H, h))) return st;
+            if (right >= 0 && (st = segment(cur, nxt, x_end - H, x_end, h))) return st;
+            if (more) {
+                SP_CUDA_TRY(cudaEventRecord(c->ev_edge, s));
+                SP_CUDA_TRY(cudaStreamWaitEvent(c->side, c->ev_edge, 0));
+                {
+                    SP_NVTX("halo exchange (overlapped)");
+                    if ((st = exchange(nxt, c->side))) return st;
+                }
+                SP_CUDA_TRY(cudaEventRecord(c->ev_xchg, c->side));
+            }
+            if ((st = segment(cur, nxt, ib, ie, h))) return st;
+            if (more) SP_CUDA_TRY(cudaStreamWaitEvent(s, c->ev_xchg, 0));
+        }
+        std::swap(cur, nxt);
+    }
+    if (cur != a_local && n_local > 0)
+        SP_CUDA_TRY(cudaMemcpyAsync(a_local + H, cur + H, n_local * sizeof(float), cudaMemcpyDeviceToDevice, s));
+    return SP_OK;
+}
+
+// Failure detection with a deadline: wait for `stream` while polling the communicator's
+// asynchronous error; on an NCCL error or when timeout_ms passes first (a peer died or hangs),
+// the communicator is aborted (ncclCommAbort: its kernels return) and SP_ERR_NCCL is returned
+// (sp_last_nccl_error: the NCCL error, or ncclInProgress = 7 for a timeout).
+extern "C" int sp_comm_sync(sp_comm* c, void* stream, int64_t timeout_ms) {
+    if (!c || timeout_ms < 0) return SP_ERR_INVALID_ARG;
+    Nccl& n = nccl();
+    const auto t0 = std::chrono::steady_clock::now();
+    for (;;) {
+        const cudaError_t q = cudaStreamQuery((cudaStream_t)stream);
+        if (q == cudaSuccess) return SP_OK;
+        if (q != cudaErrorNotReady) {
+            sp::set_cuda_error((int)q);
+            return SP_ERR_CUDA;
+        }
+        ncclResult_t r = ncclSuccess;
+        if (n.CommGetAsyncError && n.CommGetAsyncError(c->comm, &r) == ncclSuccess && r != ncclSuccess &&
+            r != ncclInProgress) {
+            if (n.CommAbort) n.CommAbort(c->comm);
+            c->comm = nullptr;
+            sp::set_nccl_error((int)r);
+            return SP_ERR_NCCL;
+        }
+        if (std::chrono::steady_clock::now() - t0 > std::chrono::milliseconds(timeout_ms)) {
+            if (n.CommAbort) n.CommAbort(c->comm);
+            c->comm = nullptr;
+            sp::set_nccl_error((int)ncclInProgress);
+            return SP_ERR_NCCL;
+        }
+        std::this_thread::sleep_for(std::chrono::microseconds(100));
+    }
 }
 
 extern "C" int sp_comm_async_error(sp_comm* c, int32_t* nccl_result) {
@@ -243,8 +355,11 @@ extern "C" int sp_allgather(sp_comm* c, const void* send, void* recv, int64_t by
 }
 
 // Single-GPU loopback transport of the same partitioned pass loop (test vehicle for the
-// decomposition; not a performance path).  Slab r owns [x_begins[r], x_begins[r] +
-// n_locals[r]); slabs must tile [0, n_global) in order.
+// decomposition and for the overlapped schedule of sp_jacobi1d_timetiled_dist; not a performance
+// path).  Slab r owns [x_begins[r], x_begins[r] + n_locals[r]); slabs must tile [0, n_global) in
+// order.  Per pass: every slab's edge segments, then the halo copies on a side stream while the
+// interior segments run on `stream` (the exchange of the dist path, with cudaMemcpyAsync in
+// place of ncclSend/ncclRecv).
 extern "C" int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_locals, int32_t nranks, int64_t n_global,
                                               const int64_t* x_begins, const int64_t* n_locals, int32_t steps,
                                               int32_t time_tile, int32_t space_tile, void* stream) {
@@ -263,20 +378,90 @@ extern "C" int sp_jacobi1d_timetiled_loopback(float** a_locals, float** work_loc
     if (expect != n_global || steps < 0) return SP_ERR_INVALID_ARG;
     if (steps == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
-    return pass_loop(slabs, n_global, steps, time_tile, space_tile, s, [&](std::vector<float*>& cur) -> int {
+    cudaStream_t side = nullptr;
+    cudaEvent_t ev_edge = nullptr, ev_xchg = nullptr;
+    SP_CUDA_TRY(cudaStreamCreateWithFlags(&side, cudaStreamNonBlocking));
+    SP_CUDA_TRY(cudaEventCreateWithFlags(&ev_edge, cudaEventDisableTiming));
+    SP_CUDA_TRY(cudaEventCreateWithFlags(&ev_xchg, cudaEventDisableTiming));
+    std::vector<float*> cur(nranks), nxt(nranks);
+    for (int r = 0; r < nranks; ++r) {
+        cur[r] = slabs[r].a;
+        nxt[r] = slabs[r].w;
+    }
+    auto exchange = [&](std::vector<float*>& b, cudaStream_t q) -> int {
         for (int r = 0; r < nranks; ++r) {
             const int64_t nl = slabs[r].n_local;
             if (r > 0)  // left halo <- left neighbour's last H owned cells
-                SP_CUDA_TRY(cudaMemcpyAsync(cur[r], cur[r - 1] + slabs[r - 1].n_local, H * sizeof(float),
-                                            cudaMemcpyDeviceToDevice, s));
+                SP_CUDA_TRY(cudaMemcpyAsync(b[r], b[r - 1] + slabs[r - 1].n_local, H * sizeof(float),
+                                            cudaMemcpyDeviceToDevice, q));
             if (r + 1 < nranks)  // right halo <- right neighbour's first H owned cells
-                SP_CUDA_TRY(cudaMemcpyAsync(cur[r] + H + nl, cur[r + 1] + H, H * sizeof(float),
-                                            cudaMemcpyDeviceToDevice, s));
+                SP_CUDA_TRY(cudaMemcpyAsync(b[r] + H + nl, b[r + 1] + H, H * sizeof(float), cudaMemcpyDeviceToDevice,
+                                            q));
         }
         return SP_OK;
-    });
+    };
+    auto segment = [&](int r, int64_t ob, int64_t oe, int32_t h) -> int {
+        if (oe <= ob) return SP_OK;
+        const Slab& sl = slabs[r];
+        return sp_jacobi1d_pass_segment(cur[r], nxt[r], n_global, sl.x_begin - H, sl.n_local + 2 * H, ob, oe, h,
+                                        time_tile, space_tile, s);
+    };
+    int st = exchange(cur, s);
+    for (int32_t done = 0; st == SP_OK && done < steps; done += time_tile) {
+        const int32_t h = steps - done < time_tile ? steps - done : time_tile;
+        const bool more = done + time_tile < steps;
+        std::vector<char> split(nranks);
+        // 1. edge segments of split slabs, whole unsplit slabs
+        for (int r = 0; r < nranks && st == SP_OK; ++r) {
+            const Slab& sl = slabs[r];
+            const int64_t xe = sl.x_begin + sl.n_local;
+            split[r] = nranks > 1 && sl.n_local >= 3 * (int64_t)H;
+            if (!split[r]) {
+                st = segment(r, sl.x_begin, xe, h);
+                continue;
+            }
+            if (r > 0) st = segment(r, sl.x_begin, sl.x_begin + H, h);
+            if (st == SP_OK && r + 1 < nranks) st = segment(r, xe - H, xe, h);
+        }
+        if (st) break;
+        // 2. the next pass's halos on the side stream, after every edge cell exists
+        if (more) {
+            if (cudaEventRecord(ev_edge, s) != cudaSuccess || cudaStreamWaitEvent(side, ev_edge, 0) != cudaSuccess) {
+                st = SP_ERR_CUDA;
+                break;
+            }
+            if ((st = exchange(nxt, side))) break;
+            if (cudaEventRecord(ev_xchg, side) != cudaSuccess) {
+                st = SP_ERR_CUDA;
+                break;
+            }
+        }
+        // 3. interiors of split slabs, concurrently with the exchange
+        for (int r = 0; r < nranks && st == SP_OK; ++r) {
+            if (!split[r]) continue;
+            const Slab& sl = slabs[r];
+            const int64_t xe = sl.x_begin + sl.n_local;
+            st = segment(r, r > 0 ? sl.x_begin + H : sl.x_begin, r + 1 < nranks ? xe - H : xe, h);
+        }
+        if (st) break;
+        if (more && cudaStreamWaitEvent(s, ev_xchg, 0) != cudaSuccess) st = SP_ERR_CUDA;
+        std::swap(cur, nxt);
+    }
+    for (int r = 0; st == SP_OK && r < nranks; ++r)
+        if (cur[r] != slabs[r].a && slabs[r].n_local > 0 &&
+            cudaMemcpyAsync(slabs[r].a + H, cur[r] + H, slabs[r].n_local * sizeof(float), cudaMemcpyDeviceToDevice,
+                            s) != cudaSuccess)
+            st = SP_ERR_CUDA;
+    if (st == SP_ERR_CUDA) sp::set_cuda_error((int)cudaGetLastError());
+    cudaEventDestroy(ev_edge);
+    cudaEventDestroy(ev_xchg);
+    cudaStreamDestroy(side);  // (destroy after pending work: resources are released on completion)
+    return st;
 }
 
+// NCCL baseline of the ME all-gather (the fused peer-store gather of sp_me_sad_search_gather is
+// the product path): this rank's range, then one ncclBroadcast per rank and output array, each
+// rank the root of its own range, in place in the global arrays (an all-gather-v).
 extern "C" int sp_me_sad_search_dist(sp_comm* c, const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t width,
                                      int32_t frame_height, int32_t n_pairs_buffer, int64_t pair_stride,
                                      int32_t pair_base, int32_t range, const int64_t* flat_ranges, int16_t* mv,
@@ -305,5 +490,5 @@ extern "C" int sp_me_sad_search_dist(sp_comm* c, const uint8_t* ref, const uint8
         SP_NCCL_TRY(n.Broadcast(best_sad + off, best_sad + off, (size_t)(4 * cnt), ncclUint8, q, c->comm, s));
     }
     SP_NCCL_TRY(n.GroupEnd());
-    return SP_OK;
+    return check_async(c);
 }

@@ -189,6 +189,30 @@ def test_loopback_partition_equals_oracle(P):
     _check(got, want)
 
 
+@pytest.mark.parametrize("bounds,steps,tt", [([0, 40, 200, 240, 401], 45, 16), ([0, 36, 72, 108, 150], 40, 16),
+                                             ([0, 12, 400, 1000], 23, 5), ([0, 1000, 1004 + 3000], 70, 32)])
+def test_loopback_split_schedule_mixed_slabs(bounds, steps, tt):
+    """The overlapped schedule (edge segments, halo exchange on a side stream, interior
+    segments) with slabs shorter and longer than 3H side by side (short ones run whole)."""
+    n = bounds[-1]
+    H = sp.halo_of(tt)
+    a = sp_inputs.jacobi_input(n, seed=n + steps)
+    want = oracle.jacobi1d(a, steps)
+    slabs = [(b, e - b) for b, e in zip(bounds[:-1], bounds[1:])]
+    assert all(nl >= H for _, nl in slabs) and all(xb % 4 == 0 for xb, _ in slabs)
+    locs, works = [], []
+    for xb, nl in slabs:
+        buf = torch.zeros(nl + 2 * H, dtype=torch.float32, device="cuda")
+        lo, hi = max(0, xb - H), min(n, xb + nl + H)
+        buf[lo - (xb - H): hi - (xb - H)] = torch.from_numpy(a[lo:hi]).cuda()
+        locs.append(buf)
+        works.append(torch.zeros_like(buf))
+    sp.jacobi1d_timetiled_loopback(locs, works, n, [s[0] for s in slabs], [s[1] for s in slabs], steps, tt, 8)
+    torch.cuda.synchronize()
+    got = np.concatenate([locs[r][H:H + slabs[r][1]].cpu().numpy() for r in range(len(slabs))])
+    _check(got, want)
+
+
 def test_pass_segment_rejects_missing_halo():
     src = torch.zeros(1000, device="cuda")
     dst = torch.zeros(1000, device="cuda")
