@@ -43,7 +43,7 @@ import numpy as np
 __all__ = [
     "SPError", "lib", "plan_buffers", "jacobi1d_plan", "jacobi1d_tile_footprint", "jacobi1d_timetiled",
     "jacobi1d_pass_segment", "jacobi1d_timetiled_loopback", "me_sad_search", "me_ref_window", "me_search_sequence",
-    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "jacobi1d_resident", "get_unique_id", "MEShard", "me_sad_search_range", "PER_ARRAY", "COMPONENTS", "halo_of",
+    "jacobi1d", "me_search", "Comm", "jacobi1d_timetiled_fused", "jacobi1d_timetiled_stream", "Jacobi1DHost", "MESearchHost", "jacobi1d_resident", "get_unique_id", "MEShard", "Prepared", "me_search_prepared", "jacobi1d_resident_prepared", "me_sad_search_range", "PER_ARRAY", "COMPONENTS", "halo_of",
 ]
 
 _HERE = os.path.dirname(os.path.abspath(__file__))
@@ -786,6 +786,51 @@ class MEShard:
         for q in self._own:
             lib.sp_device_free(vp(q))
         self._own = []
+
+
+class Prepared:
+    """A libsp call with its arguments marshalled once (ctypes objects, device pointers, the
+    stream), for latency-bound configurations where Python-side argument conversion would
+    otherwise dominate (J1, M2: a few microseconds of GPU work per call).  Calling it issues
+    exactly the C entry point; the tensors it was prepared with must stay alive and unmoved."""
+
+    def __init__(self, cfn, args, where: str, keep=()):
+        self._f, self._a, self._w, self._keep = cfn, tuple(args), where, tuple(keep)
+
+    def __call__(self):
+        st = self._f(*self._a)
+        if st:
+            raise SPError(st, self._w)
+
+
+def me_search_prepared(frames, width: int, frame_height: int, search_range: int, out=None, stream=None) -> Prepared:
+    """sp_me_sad_search over the consecutive pairs of a CUDA uint8 sequence [F, H, pitch],
+    prepared once (outputs allocated here unless given); call the result to run the search."""
+    import torch
+    ref, cur = frames[:-1], frames[1:]
+    n_pairs, rows_in_buffer, _ = ref.shape
+    pitch = ref.stride(1)
+    pair_stride = ref.stride(0) if n_pairs > 1 else pitch * rows_in_buffer
+    mbx, mby = width // 16, frame_height // 16
+    if out is None:
+        out = (torch.empty((n_pairs, mby, mbx, 2), dtype=torch.int16, device=frames.device),
+               torch.empty((n_pairs, mby, mbx), dtype=torch.int32, device=frames.device))
+    mv, sad = out[0], out[1]
+    args = (vp(ref.data_ptr()), vp(cur.data_ptr()), i64(pitch), i32(width), i32(rows_in_buffer), i32(0),
+            i32(frame_height), i32(n_pairs), i64(pair_stride), i32(16), i32(search_range), i32(0), i32(mby),
+            vp(mv.data_ptr()), vp(sad.data_ptr()), None, _stream(stream))
+    p = Prepared(lib.sp_me_sad_search, args, "sp_me_sad_search", keep=(frames, mv, sad))
+    p.mv, p.sad = mv, sad
+    return p
+
+
+def jacobi1d_resident_prepared(inp, steps: int, out=None, stream=None) -> Prepared:
+    """sp_jacobi1d_resident prepared once (small domains: one thread-block cluster)."""
+    out = inp if out is None else out
+    args = (vp(inp.data_ptr()), vp(out.data_ptr()), i64(inp.numel()), i32(steps), _stream(stream))
+    p = Prepared(lib.sp_jacobi1d_resident, args, "sp_jacobi1d_resident", keep=(inp, out))
+    p.out = out
+    return p
 
 
 class MESearchHost:

@@ -33,7 +33,7 @@ using namespace sp::ptx;
         }                                                                                \
     } while (0)
 
-__device__ long long g_out[1024];
+__device__ long long g_out[4096];
 
 // (a) barrier latency: ITER bar.sync per CTA, cycles per barrier (thread 0's clock)
 __global__ void bar_kernel(int iters) {
@@ -70,12 +70,13 @@ __global__ void pingpong_kernel(int* flags, int iters) {
     if (blockIdx.x == 0) g_out[0] = t1 - t0;
 }
 
-// unit-counter atomic round trip (one warp, dependent chain)
+// unit-counter atomic round trip (one thread, each atomic's address depends on the previous
+// result, so the round trips cannot overlap)
 __global__ void atomic_kernel(int* ctr, int iters) {
     if (threadIdx.x != 0) return;
     int v = 0;
     const long long t0 = clock64();
-    for (int i = 0; i < iters; ++i) v += atomicAdd(ctr, 1) & 1;
+    for (int i = 0; i < iters; ++i) v = atomicAdd(ctr + ((unsigned)v >> 30), 1);
     const long long t1 = clock64();
     g_out[blockIdx.x] = t1 - t0 + (v == -1);
 }
@@ -112,14 +113,14 @@ __global__ void tma_kernel(const uint8_t* src, size_t span, uint32_t bytes, int 
     }
     const long long t1 = clock64();
     g_out[blockIdx.x] = t1 - t0;
-    if (blockIdx.x == 0) g_out[1023] = wait_done;
+    if (blockIdx.x == 0) g_out[4095] = wait_done;
 }
 
 int main() {
     int sms = 0, clk_khz = 0;
     CK(cudaDeviceGetAttribute(&sms, cudaDevAttrMultiProcessorCount, 0));
     CK(cudaDeviceGetAttribute(&clk_khz, cudaDevAttrClockRate, 0));
-    std::vector<long long> h(1024);
+    std::vector<long long> h(4096);
     printf("{\"sms\": %d, \"clock_khz_attr\": %d", sms, clk_khz);
     // (a) barriers
     printf(", \"barrier_cycles\": {");
@@ -166,10 +167,13 @@ int main() {
     CK(cudaFuncSetAttribute(tma_kernel, cudaFuncAttributeMaxDynamicSharedMemorySize, 2 * 32768));
     printf(", \"tma\": [");
     first = true;
+    // ctas per SM: 0 = one CTA on the whole GPU; k >= 1 = k CTAs on every SM (k double-buffered
+    // copies in flight per SM: the kernels keep 16 warps x one prefetch in flight)
     for (uint32_t bytes : {1024u, 4096u, 6400u, 7168u, 16384u, 32768u}) {
-        for (int all : {0, 1}) {
-            const int grid = all ? sms : 1;
-            const int chunks = all ? (int)(span / 4 / bytes / sms) : 2000;
+        for (int k : {0, 1, 4, 8, 14}) {
+            if (k * 2 * bytes > 220 * 1024) continue;
+            const int grid = k ? sms * k : 1;
+            const int chunks = k ? (int)(span / 4 / bytes / grid) : 2000;
             tma_kernel<<<grid, 32, 2 * bytes>>>(src, span, bytes, chunks);
             CK(cudaDeviceSynchronize());
             cudaEvent_t e0, e1;
@@ -181,15 +185,15 @@ int main() {
             CK(cudaDeviceSynchronize());
             float ms = 0;
             CK(cudaEventElapsedTime(&ms, e0, e1));
-            CK(cudaMemcpyFromSymbol(h.data(), g_out, sizeof(long long) * 1024));
+            CK(cudaMemcpyFromSymbol(h.data(), g_out, sizeof(long long) * 4096));
             double cyc = 0;
             for (int i = 0; i < grid; ++i) cyc += (double)h[i];
             cyc /= grid;
             const double bytes_moved = (double)bytes * chunks;  // per CTA
-            printf("%s{\"bytes\": %u, \"ctas\": %d, \"bytes_per_clk_per_sm\": %.2f, \"gb_per_s_total\": %.1f, "
-                   "\"mbar_wait_complete_cycles\": %lld}",
-                   first ? "" : ", ", bytes, grid, bytes_moved / cyc, bytes_moved * grid / (ms * 1e-3) / 1e9,
-                   h[1023]);
+            const double per_sm = k ? bytes_moved * k / cyc : bytes_moved / cyc;
+            printf("%s{\"bytes\": %u, \"ctas\": %d, \"ctas_per_sm\": %d, \"bytes_per_clk_per_sm\": %.2f, "
+                   "\"gb_per_s_total\": %.1f, \"mbar_wait_complete_cycles\": %lld}",
+                   first ? "" : ", ", bytes, grid, k, per_sm, bytes_moved * grid / (ms * 1e-3) / 1e9, h[4095]);
             first = false;
         }
     }

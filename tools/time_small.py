@@ -35,7 +35,13 @@ def main():
                      ("J1 cluster-resident", lambda: sp.jacobi1d_resident(a0, 64, out=a))]:
         b, m = ev_time(fn)
         print(f"{name}: best {b:.1f} us, median {m:.1f} us  ({4094 * 64 / (b * 1e-6) / 1e9:.1f} GUpd/s)")
+    res = sp.jacobi1d_resident_prepared(a0, 64, out=a)
+    b, m = ev_time(res)
+    print(f"J1 cluster-resident, prepared call: best {b:.1f} us, median {m:.1f} us")
     fr = torch.from_numpy(sp_inputs.me_sequence(2, 352, 288, 16)).cuda()
+    pm = sp.me_search_prepared(fr, 352, 288, 16)
+    b, m = ev_time(pm)
+    print(f"M2 CIF +-16, 1 pair, prepared call: best {b:.1f} us, median {m:.1f} us ({390028 / (b * 1e-6) / 1e9:.1f} GSAD/s)")
     for surf in (False, True):
         b, m = ev_time(lambda: sp.me_search_sequence(fr, 352, 288, 16, with_surface=surf))
         print(f"M2 CIF +-16, 1 pair{' + full surface' if surf else ''}: best {b:.1f} us, median {m:.1f} us "
