@@ -143,7 +143,13 @@ struct MeGeom {
     // the first 64 bytes of stage 1's phase-1 copy (row 0), which a warp already building
     // the next macroblock's copies overwrote — a cross-warp race, rare with balanced warps.
     static constexpr int kSlot = kCopy + 128;
-    static constexpr int kSmem = kOffPh + 6 * kSlot + 128;  // + alignment slack
+    // One-warp CTAs (R = 16) keep ONE set of phase copies: the warp's own __syncwarp orders its
+    // compute of macroblock m before its phase build of m + 1, so the second set (which lets
+    // 4-warp CTAs get by with one CTA barrier per macroblock) only cost shared memory — 19.8 KB
+    // per CTA held the SM to 10 one-warp CTAs (ncu: 9.9 warps active, ALU pipe idle 11 %);
+    // 12.5 KB lets the register limit (16 CTAs) bind.
+    static constexpr int kPhaseSets = kWarps == 1 ? 1 : 2;
+    static constexpr int kSmem = kOffPh + 3 * kPhaseSets * kSlot + 128;  // + alignment slack
     static_assert(kCopy % 128 == 0, "copies must keep 128-byte alignment");
     static_assert(kSlot >= kCopy + 3 * 32 && kSlot % 128 == 0, "phase copy slots must not overlap");
     static_assert(kWarps == 1 || kWarps == 4, "tail mapping assumes 1 or 4 warps");
@@ -218,7 +224,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     // byte phase ph of stage st (ph = 0: the TMA'd window).  Copy ph starts 32*ph bytes past
     // a 128-byte boundary, so the four phases a quarter warp reads hit distinct banks.
     auto phase_copy = [&](int st, int ph) -> uint8_t* {
-        return ph == 0 ? smem + st * G::kCopy : smem + G::kOffPh + (3 * st + ph - 1) * G::kSlot + 32 * ph;
+        return ph == 0 ? smem + st * G::kCopy
+                       : smem + G::kOffPh + (3 * (G::kPhaseSets == 1 ? 0 : st) + ph - 1) * G::kSlot + 32 * ph;
     };
     struct Pos {
         int pair, byr, bx;
@@ -329,14 +336,14 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         tieB[tid][1] = make_uint4(b[4], b[5], b[6], b[7]);
     }
     // tail candidates: tie bits and staged-copy offsets (stage 0, stage 1), per thread
-    __shared__ uint32_t tinfo[G::kTailPer][3][G::kThreads];
+    __shared__ uint32_t tinfo[G::kTailPer][1 + G::kPhaseSets][G::kThreads];
 #pragma unroll
     for (int t = 0; t < G::kTailPer; ++t) {
         int dxt, dyt;
         tail_candidate<R>(warp, lane, t, dxt, dyt);
         tinfo[t][0][tid] = tie_bits(dxt, dyt, R);
 #pragma unroll
-        for (int st = 0; st < 2; ++st)
+        for (int st = 0; st < G::kPhaseSets; ++st)
             tinfo[t][1 + st][tid] =
                 (uint32_t)(phase_copy(st, (dxt + R) & 3) - smem) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
     }
@@ -363,6 +370,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // (the atomic's latency hides under the move-in wait and the phase build)
         if (tid == 0) mbS[s ^ 1] = atomicAdd(A.counter, 1u) + Gs;
         mbar_wait(&full[s], (it >> 1) & 1);
+        if (G::kPhaseSets == 1) __syncwarp();  // every lane done reading the single phase set
         PMARK(0);
         if (!(SP_ME_EXP & 128)) {  // (128: timing-only build without the phase build)
             // byte-phase copies (word q of copy p = bytes [4q+p, 4q+p+4) of the row):
@@ -420,7 +428,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const uint8_t* tp[G::kTailPer];
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) {
-            tp[t] = smem + tinfo[t][1 + s][tid];
+            tp[t] = smem + tinfo[t][1 + (G::kPhaseSets == 1 ? 0 : s)][tid];
             ta[t] = 0;
         }
         {

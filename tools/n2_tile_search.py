@@ -1,17 +1,22 @@
-"""the paper's tile-size search (§4.3) with libsp sp_tile_search.
+"""the paper's tile-size search (§4.3) with libsp sp_tile_search,
+its two constants S and L CALIBRATED by B200 microbenchmarks (tools/microbench/n2_calib.cu ->
+profiles/r02_n2_calibration.json), and the model's optimum set beside N1's measured optimum.
 
-Two uses (host only, prints JSON lines):
-1. The paper's own settings (8800 GTX: P_low = 32 threads .. 256, M_up = 16 KB / blocks per
-   multiprocessor) for the ME nest of Fig. 2 and the Jacobi
-   band, sweeping the unstated cost constants S (sync per process) and L (per element):
-   which (S, L) ratios reproduce the paper's optima, ME (32,16,16,16) and Jacobi
-   (space 256, time 32)?  — "parity unpinned" (S, L are not in the paper).
-2. B200 settings (P = 128-256 threads, M_up = the CTA's shared-memory budget), constants from
-   the measured microarchitecture (CTA barrier ~ 40 cycles; moving one 4-byte element by
-   TMA at ~22 B/clk/SM -> L ~ 0.2 cycles per element per SM, i.e. 0.2*P per process).
-    python tools/n2_tile_search.py
+    python tools/n2_tile_search.py [calibration.json]   -> JSON lines (profiles/r02_n2_tile_search.jsonl)
+
+Model: C = sum_k prod_{i<=r_k} (N_i/t_i) (P S + V_k L / P) over staged arrays (moves in and out),
+subject to sum_k M_k(t) <= M_up and prod t_i >= P; V_k, M_k from Alg. 2 on the tile box.
+Constants, in SM clock cycles:
+  S(P) = barrier(P) / P         synchronisation per process per movement (bar.sync with P threads)
+  L(P) = P * 4 B / B_sm          moving one 4-byte (Jacobi) or 1-byte (ME) element, B_sm = bulk-TMA
+                                 bytes per clock per SM with the kernels' copies in flight
+                                 (HBM-bound when every SM streams)
+Measured optima (N1, profiles/r01_jacobi_variant_sweep.txt, r01_n1_ablation.jsonl):
+  Jacobi J3: time tile 64, space tile 1664 owned (+ 2 x 64 halo = 1792 staged per warp strip)
+  ME M4: one macroblock's whole 65 x 65 candidate set x 16 x 16 pixels per CTA iteration.
 """
 import json
+import os
 import sys
 
 sys.path.insert(0, ".")
@@ -33,33 +38,52 @@ JAC_REFS = [  # (t, i') band after skewing i' = i + t (time tiles are parallelog
 POW2 = [1, 2, 4, 8, 16, 32, 64]
 
 
+def constants(cal, P, elem_bytes, chunk):
+    bars = {int(k): v for k, v in cal["barrier_cycles"].items()}
+    S = bars[P] / P
+    # bulk TMA with the most copies in flight per SM at this chunk size (the kernels keep
+    # 16 warps x 1 prefetch in flight: HBM-bound)
+    rows = [r for r in cal["tma"] if r["bytes"] == chunk and r["ctas_per_sm"] > 0]
+    B = max(r["bytes_per_clk_per_sm"] for r in rows)
+    return S, P * elem_bytes / B, B
+
+
 def main():
-    # ---- 1. paper settings ---------------------------------------------------------------
-    # ME: problem 8192 x 8192 search positions (Figs. 4/6 "64M"), WS = 16; 32 blocks share 16
-    # multiprocessors -> 2 blocks per MP -> M_up = 8 KB = 8192 one-byte elements; P = 256.
-    for ratio in [0.01, 0.1, 1, 10, 100, 1000]:
-        r = sp.tile_search([8192, 8192, 16, 16], ME_REFS, [POW2, POW2, [4, 8, 16], [4, 8, 16]], mup_elems=8192,
-                           procs=256, sync_cost=ratio, elem_cost=1.0)
-        print(json.dumps({"exp": "paper_me", "S_over_L": ratio, "tile_ijkl": r["tile"], "cost": r["cost"],
-                          "local_elems": r["local_elems"], "paper_optimum": [32, 16, 16, 16]}))
-    # Jacobi large N: 128 blocks, 64 threads, M_up = 2^11 bytes = 2^9 words
-    for ratio in [0.01, 0.1, 1, 10, 100, 1000]:
-        r = sp.tile_search([4096, 512 * 1024], JAC_REFS, [[8, 16, 32, 64, 128], [32, 64, 128, 256, 512]],
-                           mup_elems=512, procs=64, sync_cost=ratio, elem_cost=1.0)
-        print(json.dumps({"exp": "paper_jacobi", "S_over_L": ratio, "tile_time_space": r["tile"], "cost": r["cost"],
-                          "local_elems": r["local_elems"], "paper_optimum": [32, 256]}))
-    # ---- 2. B200 settings ------------------------------------------------------------------
+    path = sys.argv[1] if len(sys.argv) > 1 else os.path.join("profiles", "r02_n2_calibration.json")
+    cal = json.load(open(path))
+    out = []
+    # ---- Jacobi: the (t, i') band of J3, P = 32 lanes of a warp (the outer process is a warp),
+    # M_up = one warp strip (K = 28: 1792 fp32 cells held in registers / one staged copy)
+    P = 32
+    S, L, B = constants(cal, P, 4, 7168)
+    cand_t = [8, 16, 32, 48, 64, 96, 128]
+    cand_s = [256, 512, 1024, 1664, 2048, 4096]
+    for mup in (1792, 4096):
+        r = sp.tile_search([1024, 1 << 26], JAC_REFS, [cand_t, cand_s], mup_elems=mup, procs=P, sync_cost=S,
+                           elem_cost=L)
+        out.append({"exp": "b200_jacobi", "P": P, "S_cycles": round(S, 4), "L_cycles": round(L, 4),
+                    "tma_bytes_per_clk_sm": B, "mup_words": mup, "model_tile_time_space": r["tile"],
+                    "model_cost_cycles": r["cost"], "local_elems": r["local_elems"],
+                    "measured_optimum_time_space": [64, 1664],
+                    "measured_source": "profiles/r01_jacobi_variant_sweep.txt (K = 28: Tt 32..80)"})
+    # model cost of the measured optimum and of its neighbours (same objective, fixed tiles)
+    for tt, ss in [(64, 1664), (32, 1664), (128, 1664), (64, 1024)]:
+        r = sp.tile_search([1024, 1 << 26], JAC_REFS, [[tt], [ss]], mup_elems=0, procs=P, sync_cost=S, elem_cost=L)
+        out.append({"exp": "b200_jacobi_cost_at", "tile_time_space": [tt, ss], "model_cost_cycles": r["cost"],
+                    "local_elems": r["local_elems"]})
+    # ---- ME: Fig. 2 nest over ONE macroblock's search (N_i = N_j = 2R + 1 = 65, WS = 16),
+    # P = 128 threads (4 warps per CTA), M_up = the CTA's shared-memory budget (52 KB at 4 CTAs/SM)
     P = 128
-    S = 40.0          # cycles per CTA barrier (B300_MICROARCH: BAR ~ 20-50 cycles)
-    L = 0.18 * P      # cycles per element per process: 4 B elements at ~22 B/clk/SM by TMA
-    r = sp.tile_search([8192, 8192, 16, 16], ME_REFS, [POW2 + [128], POW2 + [128], [16], [16]],
-                       mup_elems=48 * 1024, procs=P, sync_cost=S, elem_cost=L)
-    print(json.dumps({"exp": "b200_me", "P": P, "S": S, "L": L, "mup_bytes": 48 * 1024, "tile_ijkl": r["tile"],
-                      "cost": r["cost"], "local_elems": r["local_elems"]}))
-    r = sp.tile_search([1024, 1 << 26], JAC_REFS, [[8, 16, 24, 32, 48, 64], [256, 512, 1024, 2048, 4096]],
-                       mup_elems=10 * 1024, procs=P, sync_cost=S, elem_cost=L)
-    print(json.dumps({"exp": "b200_jacobi", "P": P, "S": S, "L": L, "mup_words": 10 * 1024,
-                      "tile_time_space": r["tile"], "cost": r["cost"], "local_elems": r["local_elems"]}))
+    S, L, B = constants(cal, P, 1, 6400)
+    r = sp.tile_search([65, 65, 16, 16], ME_REFS, [[8, 16, 32, 65], [8, 16, 32, 65], [4, 8, 16], [4, 8, 16]],
+                       mup_elems=52 * 1024, procs=P, sync_cost=S, elem_cost=L)
+    out.append({"exp": "b200_me", "P": P, "S_cycles": round(S, 4), "L_cycles": round(L, 4),
+                "tma_bytes_per_clk_sm": B, "mup_bytes": 52 * 1024, "model_tile_ijkl": r["tile"],
+                "model_cost_cycles": r["cost"], "local_elems": r["local_elems"],
+                "measured_optimum_ijkl": [65, 65, 16, 16],
+                "measured_source": "round-1 ME design: one macroblock's full candidate set per CTA iteration"})
+    for o in out:
+        print(json.dumps(o))
 
 
 if __name__ == "__main__":

@@ -64,6 +64,9 @@ mark("sp.me_search_sequence (CIF +-32: 4-warp CTAs, two stages per CTA)")
 sp.me_search_sequence(fr3, 352, 288, 32)
 mark("sp.me_search_host (CIF +-32, streamed)")
 sp.MESearchHost(2, 352, 288, fr3.shape[2], 32).run(fr3.cpu().pin_memory())
+mark("sp.me_sad_search_range (flat range splitting a pair, R = 16 and 32)")
+sp.me_sad_search_range(fr, 352, 288, 16, 7, 29)
+sp.me_sad_search_range(fr3, 352, 288, 32, 3, 11)
 mark("sp.me_sad_search_direct")
 sp.me_sad_search_direct(fr2[:-1], fr2[1:], 130, 70, 8)
 torch.cuda.synchronize()
