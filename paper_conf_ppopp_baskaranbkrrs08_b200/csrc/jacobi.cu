@@ -123,9 +123,6 @@ struct PassArgs {
     float* pushR[2];
     int* edge_cnt;  // [2][passes]
     int32_t nE_left, nE_right;
-    // persistent mode: warp k (of the four sharing an SM sub-partition) starts its first unit
-    // k * stagger_ns late (experiment: SP_JACOBI_STAGGER; 0 = off)
-    int32_t stagger_ns;
 };
 
 // Spin (acquire, system scope) until *flag >= e.  A peer that never arrives (crashed rank,
@@ -574,10 +571,6 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         mbar_init(&bar[1], 1);
         fence_mbar_init();
     }
-    if (A.stagger_ns > 0 && A.done) {
-        const int k = ((warp >> 2) & 1) | ((int)((blockIdx.x / (gridDim.x >> 1 ? gridDim.x >> 1 : 1)) & 1) << 1);
-        for (int r = 0; r < k; ++r) __nanosleep(A.stagger_ns);
-    }
     __syncwarp();
     // persistent mode: this warp's finished, unpublished tiles (oldest first; at most two).
     // A tile is published (done flag) once its TMA store has completed — at the next tile's
@@ -622,27 +615,11 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             t = u - (int64_t)pass * A.tiles;
         }
     };
-#ifdef SP_JAC_GRAB2
-    int64_t spare = -1;  // (experiment) second unit of the last grab, warp-uniform
-#endif
     auto grab = [&](int64_t u_static) -> int64_t {  // warp-uniform
         if (!pers) return u_static;
-#ifdef SP_JAC_GRAB2
-        if (spare >= 0) {
-            const int64_t r = spare;
-            spare = -1;
-            return r;
-        }
-        int v = 0;
-        if (lane == 0) v = atomicAdd(next_unit, 2);
-        v = __shfl_sync(0xffffffffu, v, 0);
-        spare = (int64_t)v + 1;
-        return (int64_t)v;
-#else
         int v = 0;
         if (lane == 0) v = atomicAdd(next_unit, 1);
         return (int64_t)__shfl_sync(0xffffffffu, v, 0);
-#endif
     };
     int64_t u_cur = grab(first);
     int64_t cur_t;
@@ -993,17 +970,7 @@ int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v, bool p
     int64_t cap = (int64_t)v.sms * (peer ? v.occ_peer : v.occ);
     if (env_cap > 0 && env_cap < cap) cap = env_cap;
     const int grid = (int)(a.tiles < cap ? a.tiles : cap);
-    static const int32_t env_stagger = [] {
-        const char* e = std::getenv("SP_JACOBI_STAGGER");
-        return e ? (int32_t)std::atoi(e) : 0;
-    }();
-    if (env_stagger > 0 && a.done) {
-        PassArgs b = a;
-        b.stagger_ns = env_stagger;
-        (peer ? v.kernel_peer : v.kernel)<<<grid, v.threads, smem_bytes(v), stream>>>(b);
-    } else {
-        (peer ? v.kernel_peer : v.kernel)<<<grid, v.threads, smem_bytes(v), stream>>>(a);
-    }
+    (peer ? v.kernel_peer : v.kernel)<<<grid, v.threads, smem_bytes(v), stream>>>(a);
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }
