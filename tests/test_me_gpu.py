@@ -151,3 +151,29 @@ def test_pad_frames_edge_extension():
     for f in range(2):
         want = np.pad(fr[f, :, :W], pad, mode="edge")
         assert np.array_equal(out[f, :, :W + 2 * pad], want)
+
+
+@pytest.mark.parametrize("W,H", [(96, 80), (352, 288), (64, 64), (48, 32), (100, 70), (160, 96), (16, 48), (80, 16),
+                                 (129, 47), (208, 144)])
+@pytest.mark.parametrize("R", [16, 32])
+@pytest.mark.parametrize("gen", ["seq", "uniform", "flat"])
+def test_border_macroblock_variants_without_surface(W, H, R, gen):
+    """Without a surface, border macroblocks whose valid displacements fit in half the
+    candidate frame are searched with the half-width / half-height thread tiles (me.cu
+    border_search): MVs and SADs must still equal the oracle on every macroblock — frames
+    whose sides are multiples of 16 (first and last MB rows / columns qualify), others (only
+    the first ones do), tiny frames where both sides bind, and flat frames (every candidate
+    ties: the tie-break across the variant's candidate frame and tails)."""
+    pitch = _pitch(W)
+    if gen == "seq":
+        fr = sp_inputs.me_sequence(3, W, H, R, seed=W * 3 + H + R, pitch=pitch)
+    elif gen == "uniform":
+        fr = sp_inputs.me_uniform_frames(3, W, H, seed=W + H, pitch=pitch)
+    else:
+        fr = np.zeros((3, H, pitch), np.uint8)
+        fr[0], fr[1], fr[2] = 7, 7, 200
+    mv, sad, _ = _gpu(fr, W, H, R)
+    for p in range(2):
+        omv, osad, _ = _oracle_pair(fr, p, W, H, R, surface=False)
+        assert np.array_equal(mv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(sad[p].reshape(-1), osad), p
