@@ -200,8 +200,13 @@ __device__ __forceinline__ bool tail_slot(int warp, int lane, int t, int& k) {
 // keeps its registers and code layout.  Candidates dx = dx0 + p + 4 (TX g + j), dy = dy0 +
 // TY d + i; column tails at dx = dx0 + 4 TX kGx, row tails at dy = dy0 + TY kDy; invalid
 // ones never enter the key.  Returns the thread's minimal key.
+#ifdef SP_ME_BORDER_INLINE
+#define SP_ME_BORDER_ATTR __forceinline__
+#else
+#define SP_ME_BORDER_ATTR __noinline__
+#endif
 template <int R, int TX, int TY>
-__device__ __noinline__ uint32_t border_search(uint8_t* smem, int s, int dx0, int dy0, int dxlo, int dxhi, int dylo,
+__device__ SP_ME_BORDER_ATTR uint32_t border_search(uint8_t* smem, int s, int dx0, int dy0, int dxlo, int dxhi, int dylo,
                                                int dyhi, int tid) {
     using G = MeGeom<R>;
     // (the kernel's shared-memory layout: raw window / byte-phase copies / current block)
@@ -537,7 +542,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // (warp-uniform; never with a surface, whose every entry must be written)
         int dx0 = -R, dy0 = -R;
         bool hx = false, hy = false;
-        if (!interior && !A.surface) {
+        if (!interior && !A.surface && !(SP_ME_EXP & 256)) {  // (256: timing-only build without border tiles)
             const int cx = dxlo - ((dxlo + R) & 7);
             hx = dxhi <= cx + R;
             hy = dyhi - dylo <= R;
@@ -681,7 +686,9 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             const uint32_t tot = __reduce_add_sync(0xffffffffu, part);
             if (lane == 0) {
                 lsum[s] = tot;
-                ltie[s] = (CX >= dxlo && CX <= dxhi && CY >= dylo && CY <= dyhi) ? tie_bits(CX, CY, R) : 0xffffffffu;
+                ltie[s] = (A.unrestricted || (CX >= dxlo && CX <= dxhi && CY >= dylo && CY <= dyhi))
+                              ? tie_bits(CX, CY, R)
+                              : 0xffffffffu;
             }
         }
         PMARK(4);
