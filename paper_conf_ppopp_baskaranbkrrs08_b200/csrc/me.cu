@@ -181,121 +181,6 @@ __device__ __forceinline__ bool tail_candidate(int warp, int lane, int t, int& d
     return col;
 }
 
-// Tail candidate t of thread (warp, lane) as (column?, k): a column tail has dy = dy0 + k, a
-// row tail dx = dx0 + k, in the candidate frame whose main block starts at (dx0, dy0).
-template <int R>
-__device__ __forceinline__ bool tail_slot(int warp, int lane, int t, int& k) {
-    int dx, dy;
-    const bool col = tail_candidate<R>(warp, lane, t, dx, dy);
-    k = col ? dy + R : dx + R;
-    return col;
-}
-
-// Border macroblocks.  When the valid displacements of a macroblock fit in R + 1 columns (or
-// rows) — the first / last macroblock column (row) of a frame whose width (height) is a
-// multiple of 16 — at most half of the 2R x 2R main candidates can be valid: the thread tile
-// then shrinks to TX = 2 dx (TY = 4 dy) candidates over a candidate frame starting at dx0
-// (dy0), so the CTA computes the valid half instead of computing and masking all of it
-// (CIF +-16: 76 of 396 macroblocks, 9 % of the SAD work).  Out of line: the interior path
-// keeps its registers and code layout.  Candidates dx = dx0 + p + 4 (TX g + j), dy = dy0 +
-// TY d + i; column tails at dx = dx0 + 4 TX kGx, row tails at dy = dy0 + TY kDy; invalid
-// ones never enter the key.  Returns the thread's minimal key.
-#ifdef SP_ME_BORDER_INLINE
-#define SP_ME_BORDER_ATTR __forceinline__
-#else
-#define SP_ME_BORDER_ATTR __noinline__
-#endif
-template <int R, int TX, int TY>
-__device__ SP_ME_BORDER_ATTR uint32_t border_search(uint8_t* smem, int s, int dx0, int dy0, int dxlo, int dxhi, int dylo,
-                                               int dyhi, int tid) {
-    using G = MeGeom<R>;
-    // (the kernel's shared-memory layout: raw window / byte-phase copies / current block)
-    auto phase_base = [&](int ph) -> const uint8_t* {
-        return ph == 0 ? smem + s * G::kCopy
-                       : smem + G::kOffPh + (3 * (G::kPhaseSets == 1 ? 0 : s) + ph - 1) * G::kSlot + 32 * ph;
-    };
-    const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
-    constexpr int win = G::kWin;
-    constexpr int kDy = G::kThreads / (4 * G::kGx);
-    constexpr int NW = TX + 3;
-    const int lane = tid & 31, warp = tid >> 5;
-    const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
-    const int CX = dx0 + 4 * TX * G::kGx, CY = dy0 + TY * kDy;  // tail column / row
-    // tails: window address (row dy + R, byte dx + R of the matching phase copy) and key bits
-    const uint8_t* tp[G::kTailPer];
-    uint32_t ttie[G::kTailPer];
-    bool tval[G::kTailPer];
-#pragma unroll
-    for (int t = 0; t < G::kTailPer; ++t) {
-        int k;
-        const bool col = tail_slot<R>(warp, lane, t, k);
-        const bool inside = k < (col ? TY * kDy : 4 * TX * G::kGx);  // (beyond: not a candidate)
-        const int dx = col ? CX : dx0 + k, dy = col ? dy0 + k : CY;
-        tval[t] = inside && dx >= dxlo && dx <= dxhi && dy >= dylo && dy <= dyhi;
-        ttie[t] = tie_bits(dx, dy, R);
-        tp[t] = inside ? phase_base((dx + R) & 3) + (dy + R) * win + 4 * ((dx + R) >> 2) : phase_base(0);
-    }
-    uint32_t acc[TX][TY], ta[G::kTailPer];
-#pragma unroll
-    for (int j = 0; j < TX; ++j)
-#pragma unroll
-        for (int i = 0; i < TY; ++i) acc[j][i] = 0;
-#pragma unroll
-    for (int t = 0; t < G::kTailPer; ++t) ta[t] = 0;
-    const uint8_t* rowp = phase_base(p) + (dy0 + R + TY * d) * win + 4 * ((dx0 + R) / 4 + TX * g);
-    uint32_t Rw[TY][NW];
-    auto load_row = [&](uint32_t(&w)[NW], const uint8_t* src) {
-        if constexpr (TX == 4) {
-            const uint4 a = *reinterpret_cast<const uint4*>(src);
-            const uint4 b = *reinterpret_cast<const uint4*>(src + 16);
-            w[0] = a.x; w[1] = a.y; w[2] = a.z; w[3] = a.w; w[4] = b.x; w[5] = b.y; w[6] = b.z;
-        } else {  // 8-byte aligned: (dx0 + R) and 8 g are multiples of 8
-            const uint2 a = *reinterpret_cast<const uint2*>(src);
-            const uint2 b = *reinterpret_cast<const uint2*>(src + 8);
-            w[0] = a.x; w[1] = a.y; w[2] = b.x; w[3] = b.y; w[4] = *reinterpret_cast<const uint32_t*>(src + 16);
-        }
-    };
-#pragma unroll
-    for (int rr = 0; rr < TY - 1; ++rr) load_row(Rw[rr], rowp + rr * win);
-#pragma unroll 1
-    for (int vb = 0; vb < kMB; vb += TY) {
-#pragma unroll
-        for (int vv = 0; vv < TY; ++vv) {
-            const int v = vb + vv;
-            load_row(Rw[(vv + TY - 1) % TY], rowp + (v + TY - 1) * win);
-            const uint4 cv = cq[v];
-            const uint32_t Cv[4] = {cv.x, cv.y, cv.z, cv.w};
-#pragma unroll
-            for (int t = 0; t < G::kTailPer; ++t) {
-                const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
-#pragma unroll
-                for (int k = 0; k < 4; ++k) ta[t] = sad4(tq[k], Cv[k], ta[t]);
-            }
-#pragma unroll
-            for (int k = 0; k < 4; ++k)
-#pragma unroll
-                for (int i = 0; i < TY; ++i)
-#pragma unroll
-                    for (int j = 0; j < TX; ++j) acc[j][i] = sad4(Rw[(vv + i) % TY][j + k], Cv[k], acc[j][i]);
-        }
-    }
-    uint32_t key = 0xffffffffu;
-#pragma unroll
-    for (int j = 0; j < TX; ++j) {
-        const int dx = dx0 + p + 4 * (TX * g + j);
-#pragma unroll
-        for (int i = 0; i < TY; ++i) {
-            const int dy = dy0 + TY * d + i;
-            if (dx >= dxlo && dx <= dxhi && dy >= dylo && dy <= dyhi)
-                key = min(key, acc[j][i] * kKeyMul + tie_bits(dx, dy, R));
-        }
-    }
-#pragma unroll
-    for (int t = 0; t < G::kTailPer; ++t)
-        if (tval[t]) key = min(key, ta[t] * kKeyMul + ttie[t]);
-    return key;
-}
-
 // Frames still streaming in (sp_me_search_host): wait for a pair's ready flag (relaxed poll,
 // then an acquire and a proxy fence order the observed copy before the TMA reads that follow).
 // Out of line: the common device-resident path keeps its register / uniform-datapath layout.
@@ -327,7 +212,6 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     __shared__ __align__(8) uint64_t full[2];
     __shared__ uint32_t red32[2][nwarps];  // per-stage per-warp minimal key
     __shared__ uint32_t lsum[2];           // per-stage SAD of the corner candidate (R, R)
-    __shared__ uint32_t ltie[2];           // per-stage tie bits of the corner candidate, ~0u if invalid
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
 
@@ -368,10 +252,11 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         uint32_t b = red32[sp][0];
 #pragma unroll
         for (int w = 1; w < nwarps; ++w) b = min(b, red32[sp][w]);
-        const uint32_t lsad = lsum[sp], lt = ltie[sp];
+        const uint32_t lsad = lsum[sp];
         const Pos q = locate(mbp);
-        const bool lvalid = lt != 0xffffffffu;  // (the corner of the macroblock's candidate frame)
-        if (lvalid) b = min(b, lsad * kKeyMul + lt);
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
+        const bool lvalid = A.unrestricted || ((x0 + R + 16 <= W) && (y0 + R + 16 <= Hf));
+        if (lvalid) b = min(b, lsad * kKeyMul + tie_bits(R, R, R));
         const size_t idx = ((size_t)q.pair * A.mb_rows + q.byr) * mbx + q.bx;
         const uint32_t sad = b / kKeyMul, tie = b - sad * kKeyMul;
         const int dy = (int)((tie >> 1) & 127) - R;
@@ -532,30 +417,6 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // lower ones build the next macroblock's copies while these still read this one's
         if (warp >= nwarps / 2) __nanosleep(20000);
 #endif
-        // ---- validity (restricted vectors) only matters near the frame border ----------
-        const Pos q = posS[s];  // (written one macroblock ahead; stable until the next barrier)
-        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
-        const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
-        const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
-        const bool interior = A.unrestricted || (dxlo == -R && dxhi == R && dylo == -R && dyhi == R);
-        // border macroblocks whose valid displacements fit in half the candidate frame
-        // (warp-uniform; never with a surface, whose every entry must be written)
-        int dx0 = -R, dy0 = -R;
-        bool hx = false, hy = false;
-        if (!interior && !A.surface && !(SP_ME_EXP & 256)) {  // (256: timing-only build without border tiles)
-            const int cx = dxlo - ((dxlo + R) & 7);
-            hx = dxhi <= cx + R;
-            hy = dyhi - dylo <= R;
-            if (hx) dx0 = cx;
-            if (hy) dy0 = dylo;
-        }
-        const int CX = dx0 + (hx ? R : 2 * R), CY = dy0 + (hy ? R : 2 * R);  // the frame's corner
-        uint32_t key = 0xffffffffu;
-        if (hx || hy) {
-            if (hx && hy) key = border_search<R, 2, 4>(smem, s, dx0, dy0, dxlo, dxhi, dylo, dyhi, tid);
-            else if (hx) key = border_search<R, 2, 8>(smem, s, dx0, dy0, dxlo, dxhi, dylo, dyhi, tid);
-            else key = border_search<R, 4, 4>(smem, s, dx0, dy0, dxlo, dxhi, dylo, dyhi, tid);
-        } else {
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
         //      thread's tail candidates, all in one row loop ----
         uint32_t acc[kTx][kTy];
@@ -623,6 +484,28 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
         }
         PMARK(3);
+        if (warp == 0) {  // the corner candidate (R, R): 64 (row, word) pieces over warp 0
+            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + s * G::kCopy + (2 * R) * win) + R / 2;
+            const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+            uint32_t part = 0;
+#pragma unroll
+            for (int o = lane; o < 64; o += 32) {
+                const int v = o >> 2, k = o & 3;
+                const uint4 cv = cq4[v];
+                const uint32_t cw = k == 0 ? cv.x : k == 1 ? cv.y : k == 2 ? cv.z : cv.w;
+                part = sad4(rw[v * (win / 4) + k], cw, part);
+            }
+            const uint32_t tot = __reduce_add_sync(0xffffffffu, part);
+            if (lane == 0) lsum[s] = tot;
+        }
+        PMARK(4);
+
+        // ---- validity (restricted vectors) only matters near the frame border ----------
+        const Pos q = posS[s];  // (written one macroblock ahead; stable until the next barrier)
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
+        const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
+        const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
+        const bool interior = A.unrestricted || (dxlo == -R && dxhi == R && dylo == -R && dyhi == R);
         if (!interior) {
 #pragma unroll
             for (int j = 0; j < kTx; ++j) {
@@ -656,6 +539,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         }
         // ---- argmin: min over this thread's keys, key(j, i) = acc * kKeyMul + A_j + B_i,
         //      then one CREDUX per warp ----
+        uint32_t key = 0xffffffffu;
         {
             const uint4 a4 = tieA[p + 4 * g];
             const uint32_t Aj[4] = {a4.x, a4.y, a4.z, a4.w};
@@ -671,27 +555,6 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         }
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) key = min(key, ta[t] * kKeyMul + tinfo[t][0][tid]);
-        }  // (interior / full-frame path)
-        if (warp == 0) {  // the frame's corner candidate (CX, CY): 64 (row, word) pieces over warp 0
-            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + s * G::kCopy + (CY + R) * win) + (CX + R) / 4;
-            const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
-            uint32_t part = 0;
-#pragma unroll
-            for (int o = lane; o < 64; o += 32) {
-                const int v = o >> 2, k = o & 3;
-                const uint4 cv = cq4[v];
-                const uint32_t cw = k == 0 ? cv.x : k == 1 ? cv.y : k == 2 ? cv.z : cv.w;
-                part = sad4(rw[v * (win / 4) + k], cw, part);
-            }
-            const uint32_t tot = __reduce_add_sync(0xffffffffu, part);
-            if (lane == 0) {
-                lsum[s] = tot;
-                ltie[s] = (A.unrestricted || (CX >= dxlo && CX <= dxhi && CY >= dylo && CY <= dyhi))
-                              ? tie_bits(CX, CY, R)
-                              : 0xffffffffu;
-            }
-        }
-        PMARK(4);
         key = __reduce_min_sync(0xffffffffu, key);
         if (lane == 0) red32[s][warp] = key;
         PMARK(7);

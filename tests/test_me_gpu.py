@@ -157,13 +157,11 @@ def test_pad_frames_edge_extension():
                                  (129, 47), (208, 144)])
 @pytest.mark.parametrize("R", [16, 32])
 @pytest.mark.parametrize("gen", ["seq", "uniform", "flat"])
-def test_border_macroblock_variants_without_surface(W, H, R, gen):
-    """Without a surface, border macroblocks whose valid displacements fit in half the
-    candidate frame are searched with the half-width / half-height thread tiles (me.cu
-    border_search): MVs and SADs must still equal the oracle on every macroblock — frames
-    whose sides are multiples of 16 (first and last MB rows / columns qualify), others (only
-    the first ones do), tiny frames where both sides bind, and flat frames (every candidate
-    ties: the tie-break across the variant's candidate frame and tails)."""
+def test_border_macroblocks_without_surface(W, H, R, gen):
+    """MVs and SADs without a surface (the bench's launch form) on frames whose border
+    macroblocks have few valid candidates: sides multiples of 16 or not, tiny frames where both
+    sides bind, flat frames (every candidate ties: the tie-break across the main block, the
+    tails and the corner candidate)."""
     pitch = _pitch(W)
     if gen == "seq":
         fr = sp_inputs.me_sequence(3, W, H, R, seed=W * 3 + H + R, pitch=pitch)
