@@ -42,16 +42,24 @@ using namespace sp::ptx;
 // WARPS strips.
 // SE_ selects the step with scalar edge cells (run_steps_se: no packing moves on the FMA
 // pipe, any K); the packed-edge step (run_steps) needs K <= 32 for its boundary bit masks.
-template <int K_, int WARPS_, int MINB_, bool SE_ = false>
+// IP_ (in place): K + 1 registers per lane hold the K pairs and the step alternates ascending
+// and descending sweeps (see sweep_up / sweep_down), so one register array suffices and K can
+// grow; one staged copy per warp (the next tile streams into it once the registers are loaded)
+// and a direct register -> global move-out.  Device-resident persistent launches only.
+template <int K_, int WARPS_, int MINB_, bool SE_ = false, bool IP_ = false>
 struct JCfg {
     static constexpr int K = K_;
     static constexpr int kWarps = WARPS_;
     static constexpr int kMinBlocks = MINB_;
     static constexpr bool kScalarEdges = SE_;
+    static constexpr bool kInPlace = IP_;
     static constexpr int kThreads = 32 * WARPS_;
     static constexpr int kStrip = 64 * K_;
-    static constexpr int kStage = WARPS_ * 2 * 64 * K_;  // floats of shared memory per CTA
-    static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && (SE_ || K_ <= 32), "K/4 must be odd, K <= 32 unless scalar edges");
+    static constexpr int kStages = IP_ ? 1 : 2;
+    static constexpr int kStage = WARPS_ * kStages * 64 * K_;  // floats of shared memory per CTA
+    static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && (SE_ || IP_ || K_ <= 32),
+                  "K/4 must be odd, K <= 32 unless scalar edges or in place");
+    static_assert(!(SE_ && IP_), "in-place sweeps use packed edges");
 };
 constexpr int kMaxTimeTile = 128;
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
@@ -349,6 +357,111 @@ __device__ __forceinline__ void run_steps_fx(uint64_t (&P)[kK], int h, int lane,
     }
 }
 
+// ---- in-place sweeps (JCfg kInPlace) ------------------------------------------------------
+// K pairs live in K + 1 registers R[0..K].  Before an ascending sweep element j is in R[j + 1];
+// the sweep computes new element j from old j - 1 (R[j]), j (R[j + 1]) and j + 1 (R[j + 2]) and
+// writes it into R[j] — old j - 1 is dead by then — so afterwards element j is in R[j].  A
+// descending sweep computes new j from R[j - 1], R[j], R[j + 1] into R[j + 1] (old j + 1 dead),
+// restoring the first mapping: two steps, no register copies.  Each sweep computes first the
+// edge pair the NEXT sweep needs last and issues its shuffles right away (latency hidden by
+// the rest of the sweep).  Same op order as update(): bit-identical to the definition.
+__device__ __forceinline__ uint64_t nb_left(uint64_t last, int lane) {  // lane-1's last pair -> my left
+    const float a = __shfl_sync(0xffffffffu, f2_lo(last), (lane + 31) & 31);
+    const float b = __shfl_sync(0xffffffffu, f2_hi(last), (lane + 31) & 31);
+    return f2_pack(a, lane == 0 ? a : b);
+}
+__device__ __forceinline__ uint64_t nb_right(uint64_t first, int lane) {  // lane+1's first pair -> my right
+    const float c = __shfl_sync(0xffffffffu, f2_lo(first), (lane + 1) & 31);
+    const float d = __shfl_sync(0xffffffffu, f2_hi(first), (lane + 1) & 31);
+    return f2_pack(lane == 31 ? d : c, d);
+}
+template <int kK>
+__device__ __forceinline__ void sweep_up(uint64_t (&R)[kK + 1], uint64_t& left, uint64_t& right, int lane, uint64_t w2,
+                                         uint64_t mz) {
+    R[0] = update(left, R[1], R[2], w2, mz);
+    const uint64_t rn = nb_right(R[0], lane);  // needed first by the descending sweep
+#pragma unroll
+    for (int j = 1; j < kK - 1; ++j) R[j] = update(R[j], R[j + 1], R[j + 2], w2, mz);
+    R[kK - 1] = update(R[kK - 1], R[kK], right, w2, mz);
+    left = nb_left(R[kK - 1], lane);  // needed last by the descending sweep
+    right = rn;
+}
+template <int kK>
+__device__ __forceinline__ void sweep_down(uint64_t (&R)[kK + 1], uint64_t& left, uint64_t& right, int lane,
+                                           uint64_t w2, uint64_t mz) {
+    R[kK] = update(R[kK - 2], R[kK - 1], right, w2, mz);
+    const uint64_t ln = nb_left(R[kK], lane);  // needed first by the ascending sweep
+#pragma unroll
+    for (int j = kK - 2; j >= 1; --j) R[j + 1] = update(R[j - 1], R[j], R[j + 1], w2, mz);
+    R[1] = update(left, R[0], R[1], w2, mz);
+    right = nb_right(R[1], lane);  // needed last by the ascending sweep
+    left = ln;
+}
+// Dirichlet restore of a fixed cell on the element held at R[j + OFF] (jump table, as
+// restore_one; fx as in FixedCells)
+template <int kK, int OFF>
+__device__ __forceinline__ void restore_one_ip(uint64_t (&R)[kK + 1], int lane, int fx, float val) {
+    if (fx < 0) return;  // warp-uniform
+    const bool me = lane == (fx >> 9), hi = (fx >> 8) & 1;
+#define SP_FIXIP_CASE(J)                                                                                  \
+    case J:                                                                                               \
+        if constexpr (J < kK) {                                                                           \
+            if (me) R[J + OFF] = hi ? f2_pack(f2_lo(R[J + OFF]), val) : f2_pack(val, f2_hi(R[J + OFF]));  \
+        }                                                                                                 \
+        break;
+    switch (fx & 255) {
+        SP_FIXIP_CASE(0) SP_FIXIP_CASE(1) SP_FIXIP_CASE(2) SP_FIXIP_CASE(3) SP_FIXIP_CASE(4) SP_FIXIP_CASE(5)
+        SP_FIXIP_CASE(6) SP_FIXIP_CASE(7) SP_FIXIP_CASE(8) SP_FIXIP_CASE(9) SP_FIXIP_CASE(10) SP_FIXIP_CASE(11)
+        SP_FIXIP_CASE(12) SP_FIXIP_CASE(13) SP_FIXIP_CASE(14) SP_FIXIP_CASE(15) SP_FIXIP_CASE(16) SP_FIXIP_CASE(17)
+        SP_FIXIP_CASE(18) SP_FIXIP_CASE(19) SP_FIXIP_CASE(20) SP_FIXIP_CASE(21) SP_FIXIP_CASE(22) SP_FIXIP_CASE(23)
+        SP_FIXIP_CASE(24) SP_FIXIP_CASE(25) SP_FIXIP_CASE(26) SP_FIXIP_CASE(27) SP_FIXIP_CASE(28) SP_FIXIP_CASE(29)
+        SP_FIXIP_CASE(30) SP_FIXIP_CASE(31) SP_FIXIP_CASE(32) SP_FIXIP_CASE(33) SP_FIXIP_CASE(34) SP_FIXIP_CASE(35)
+        SP_FIXIP_CASE(36) SP_FIXIP_CASE(37) SP_FIXIP_CASE(38) SP_FIXIP_CASE(39) SP_FIXIP_CASE(40) SP_FIXIP_CASE(41)
+        SP_FIXIP_CASE(42) SP_FIXIP_CASE(43) SP_FIXIP_CASE(44) SP_FIXIP_CASE(45) SP_FIXIP_CASE(46) SP_FIXIP_CASE(47)
+        SP_FIXIP_CASE(48) SP_FIXIP_CASE(49) SP_FIXIP_CASE(50) SP_FIXIP_CASE(51) SP_FIXIP_CASE(52) SP_FIXIP_CASE(53)
+        SP_FIXIP_CASE(54) SP_FIXIP_CASE(55) SP_FIXIP_CASE(56) SP_FIXIP_CASE(57) SP_FIXIP_CASE(58) SP_FIXIP_CASE(59)
+        SP_FIXIP_CASE(60) SP_FIXIP_CASE(61) SP_FIXIP_CASE(62) SP_FIXIP_CASE(63)
+        default: break;
+    }
+#undef SP_FIXIP_CASE
+}
+// h steps in place; on return element j is in R[j + 1] (an odd h ends with K register moves)
+template <bool kBoundary, int kK>
+__device__ __forceinline__ void run_steps_ip(uint64_t (&R)[kK + 1], int h, int lane, uint64_t w2, uint64_t mz,
+                                             const FixedCells& f) {
+    uint64_t left = nb_left(R[kK], lane), right = nb_right(R[1], lane);
+    int k = 0;
+    for (; k + 2 <= h; k += 2) {
+        sweep_up<kK>(R, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore_one_ip<kK, 0>(R, lane, f.fx0, f.v0);
+            restore_one_ip<kK, 0>(R, lane, f.fx1, f.v1);
+            if (f.edge) {
+                left = nb_left(R[kK - 1], lane);
+                right = nb_right(R[0], lane);
+            }
+        }
+        sweep_down<kK>(R, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore_one_ip<kK, 1>(R, lane, f.fx0, f.v0);
+            restore_one_ip<kK, 1>(R, lane, f.fx1, f.v1);
+            if (f.edge) {
+                left = nb_left(R[kK], lane);
+                right = nb_right(R[1], lane);
+            }
+        }
+    }
+    if (k < h) {
+        sweep_up<kK>(R, left, right, lane, w2, mz);
+        if (kBoundary) {
+            restore_one_ip<kK, 0>(R, lane, f.fx0, f.v0);
+            restore_one_ip<kK, 0>(R, lane, f.fx1, f.v1);
+        }
+#pragma unroll
+        for (int j = kK; j >= 1; --j) R[j] = R[j - 1];
+    }
+}
+
 // ---- scalar-edge variant ----------------------------------------------------------------
 // fl(x * w) rounded once, as fma(x, w, -0) with the -0 addend opaque (see f2_mul_nofuse):
 // FFMA with an immediate w issues at full rate.
@@ -452,7 +565,9 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     __shared__ __align__(8) uint64_t full[Cfg::kWarps][2];
 
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-    float* const stage0 = smem + warp * 2 * kStrip;  // this warp's two stages
+    float* const stage0 = smem + warp * Cfg::kStages * kStrip;  // this warp's stage(s)
+    constexpr bool kIP = Cfg::kInPlace;
+    static_assert(!(kIP && kPeer), "the in-place geometry has no peer instantiation");
     uint64_t* const bar = full[warp];
     const uint64_t w2 = (uint64_t(kW) << 32) | kW;
     const int64_t GW = (int64_t)gridDim.x * Cfg::kWarps;
@@ -632,9 +747,11 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     __syncwarp();
     auto publish = [&](bool all) {  // lane 0: the oldest unpublished tile (all: every one)
         if (pub_t[0] < 0 || (!all && pub_t[1] < 0)) return;
-        if (all) bulk_wait0();
-        else bulk_wait1();            // every store but the newest tile's has completed
-        fence_proxy_async_global();   // async-proxy writes -> generic release below
+        if constexpr (!kIP) {
+            if (all) bulk_wait0();
+            else bulk_wait1();            // every store but the newest tile's has completed
+            fence_proxy_async_global();   // async-proxy writes -> generic release below
+        }  // (in place: the warp's generic stores precede lane 0's release through __syncwarp)
         st_release_gpu(A.done + pub_t[0], pub_pass[0] + 1);
         if (all && pub_t[1] >= 0) st_release_gpu(A.done + pub_t[1], pub_pass[1] + 1);
         pub_t[0] = all ? -1 : pub_t[1];
@@ -644,7 +761,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 
     int it = 0;
     for (int64_t u = u_cur; u < total; ++it) {
-        const int s = it & 1;
+        const int s = kIP ? 0 : (it & 1);
         float* const buf = stage0 + s * kStrip;
         int64_t x0, st, lo, hi;
         const int64_t t = cur_t;
@@ -687,7 +804,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 #ifdef SP_JAC_DEBUG
         const long long tw0 = clock64();
 #endif
-        mbar_wait(&bar[s], (it >> 1) & 1);
+        mbar_wait(&bar[s], kIP ? (it & 1) : ((it >> 1) & 1));
         __syncwarp();
 #ifdef SP_JAC_DEBUG
         if (lane == 0 && pass > 0) atomicAdd(&g_jac_dbg[2], (unsigned long long)(clock64() - tw0));
@@ -695,17 +812,28 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 #endif
 
         // ---- registers <- staged strip (conflict-free: stride 4K bytes, K/4 odd) ---------
-        uint64_t P[kK];
+        constexpr int O = kIP ? 1 : 0;  // in place: pair j in P[j + 1] (P[0] spare)
+        uint64_t P[kK + O];
         {
             const float4* pu = reinterpret_cast<const float4*>(buf + lane * kK);
             const float4* pv = reinterpret_cast<const float4*>(buf + 32 * kK + lane * kK);
 #pragma unroll
             for (int q = 0; q < kK / 4; ++q) {
                 const float4 u = pu[q], v = pv[q];
-                P[4 * q + 0] = f2_pack(u.x, v.x);
-                P[4 * q + 1] = f2_pack(u.y, v.y);
-                P[4 * q + 2] = f2_pack(u.z, v.z);
-                P[4 * q + 3] = f2_pack(u.w, v.w);
+                P[4 * q + 0 + O] = f2_pack(u.x, v.x);
+                P[4 * q + 1 + O] = f2_pack(u.y, v.y);
+                P[4 * q + 2 + O] = f2_pack(u.z, v.z);
+                P[4 * q + 3 + O] = f2_pack(u.w, v.w);
+            }
+        }
+        // in place, the Dirichlet cells' values are read from the staged strip now: the
+        // prefetch below refills the (single) stage
+        const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= A.n - 1 && A.n - 1 < base + kStrip);
+        FixedCells fc{-1, -1, 0.f, 0.f, false};
+        if constexpr (kIP) {
+            if (boundary) {
+                fc = fixed_cells<kK>(base, A.n, 0 >= base ? buf[0 - base] : 0.f,
+                                     A.n - 1 - base < kStrip ? buf[A.n - 1 - base] : 0.f);
             }
         }
         // ---- prefetch the next tile into the other stage once its store has drained ----
@@ -721,7 +849,15 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             pending = (pers && pn > 0 && 2 * reach < 32)
                           ? (!__all_sync(0xffffffffu, next_flag >= pn) || (kPeer && !peer_ready(tn, pn)))
                           : !deps_ready(tn, pn);
-            if (lane == 0) {
+            if constexpr (kIP) {
+                // one stage: the next tile streams into the buffer this tile was just loaded
+                // from, once every lane's reads of it are done (warp barrier, then the proxy fence)
+                __syncwarp();
+                if (lane == 0 && !pending) {
+                    fence_proxy_async_smem();
+                    issue(tn, pn, 0);
+                }
+            } else if (lane == 0) {
                 bulk_wait_read0();
                 if (!pending) issue(tn, pn, s ^ 1);
             }
@@ -734,8 +870,10 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 #endif
         // ---- h steps in registers ---------------------------------------------------
         {
-            const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= A.n - 1 && A.n - 1 < base + kStrip);
-            if constexpr (Cfg::kScalarEdges) {
+            if constexpr (kIP) {
+                if (boundary) run_steps_ip<true, kK>(P, h, lane, w2, A.mz, fc);
+                else run_steps_ip<false, kK>(P, h, lane, w2, A.mz, fc);
+            } else if constexpr (Cfg::kScalarEdges) {
                 // pair index holding global cell 0 / n-1 in this lane's u / v range (-1: none)
                 int ju0 = -1, jv0 = -1, jun = -1, jvn = -1;
                 float v0 = 0.f, vn = 0.f;
@@ -784,6 +922,28 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         // a hash of (tile, pass), finishes 20 us late, so dependent tiles really wait
         if ((((uint32_t)t * 2654435761u) ^ (uint32_t)(pass * 40503u)) % 8u == 0u) __nanosleep(20000);
 #endif
+        if constexpr (kIP) {
+            // ---- owned cells: registers -> global (16-byte stores; the stage is busy with
+            //      the next tile's move-in) ----
+            const int own_hi = A.H + (int)st;  // strip offsets [H, H + st) are owned
+            float* const gd = dst + (base - A.g0);  // gd[j] <-> strip offset j
+#pragma unroll
+            for (int q = 0; q < kK / 4; ++q) {
+#pragma unroll
+                for (int half = 0; half < 2; ++half) {
+                    const int o = (half ? 32 * kK : 0) + lane * kK + 4 * q;  // 4 cells, 16-byte aligned
+                    auto c = [&](int e) { return half ? f2_hi(P[4 * q + e + 1]) : f2_lo(P[4 * q + e + 1]); };
+                    if (o >= A.H && o + 4 <= own_hi) {
+                        *reinterpret_cast<float4*>(gd + o) = make_float4(c(0), c(1), c(2), c(3));
+                    } else if (o >= A.H && o < own_hi) {  // the ragged end of the last tile
+                        gd[o] = c(0);
+                        if (o + 1 < own_hi) gd[o + 1] = c(1);
+                        if (o + 2 < own_hi) gd[o + 2] = c(2);
+                    }
+                }
+            }
+            __syncwarp();  // every lane's stores precede lane 0's release (publish) of this tile
+        } else {
         // ---- owned cells -> staged buffer -> TMA bulk store ------------------------------
         {
             const int own_hi = A.H + (int)st;  // strip offsets [H, H + st) are owned
@@ -812,8 +972,9 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             }
             if (lane < st - n16) dst[x0 - A.g0 + n16 + lane] = buf[A.H + n16 + lane];
         }
+        }  // (staged move-out)
         if (pers) {
-            if (lane < st - (st & ~int64_t(3))) __threadfence();  // the ragged-tail stores above
+            if (!kIP && lane < st - (st & ~int64_t(3))) __threadfence();  // the ragged-tail stores above
             __syncwarp();
             const int k = pub_t[0] < 0 ? 0 : 1;
             pub_t[k] = t;
@@ -880,7 +1041,7 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 11;
+constexpr int kNumVariants = 12;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
@@ -897,6 +1058,7 @@ Variant* variants() {
         make_variant<JCfg<44, 8, 1, true>>(),  // 8: 88 cells/lane, scalar edges, 8 warps/SM
         make_variant<JCfg<36, 12, 1, true>>(),  // 9: 72 cells/lane, scalar edges, 12 warps/SM (216 KB)
         make_variant<JCfg<44, 4, 2, true>>(),  // 10: as 8 as two 4-warp CTAs per SM
+        make_variant<JCfg<44, 8, 2, false, true>>(),  // 11: in place, 88 cells/lane, 16 warps/SM, one stage (176 KB)
     };
     return v;
 }
