@@ -1041,7 +1041,7 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 12;
+constexpr int kNumVariants = 14;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
@@ -1059,6 +1059,8 @@ Variant* variants() {
         make_variant<JCfg<36, 12, 1, true>>(),  // 9: 72 cells/lane, scalar edges, 12 warps/SM (216 KB)
         make_variant<JCfg<44, 4, 2, true>>(),  // 10: as 8 as two 4-warp CTAs per SM
         make_variant<JCfg<44, 8, 2, false, true>>(),  // 11: in place, 88 cells/lane, 16 warps/SM, one stage (176 KB)
+        make_variant<JCfg<36, 8, 2, false, true>>(),  // 12: in place, 72 cells/lane, 16 warps/SM (144 KB)
+        make_variant<JCfg<52, 8, 2, false, true>>(),  // 13: in place, 104 cells/lane, 16 warps/SM (208 KB)
     };
     return v;
 }
