@@ -431,6 +431,12 @@ __device__ __forceinline__ void run_steps_ip(uint64_t (&R)[kK + 1], int h, int l
                                              const FixedCells& f) {
     uint64_t left = nb_left(R[kK], lane), right = nb_right(R[1], lane);
     int k = 0;
+#ifndef SP_JAC_IP_UNROLL
+#define SP_JAC_IP_UNROLL 1
+#endif
+    // (the two-sweep body is 2 x 3K packed instructions; unrolled further, the loop outgrows the
+    //  instruction cache at these K — ncu: no-instruction stalls)
+#pragma unroll SP_JAC_IP_UNROLL
     for (; k + 2 <= h; k += 2) {
         sweep_up<kK>(R, left, right, lane, w2, mz);
         if (kBoundary) {
