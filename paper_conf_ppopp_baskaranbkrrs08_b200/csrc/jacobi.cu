@@ -62,6 +62,10 @@ struct JCfg {
     static_assert(!(SE_ && IP_), "in-place sweeps use packed edges");
 };
 constexpr int kMaxTimeTile = 128;
+#ifndef SP_JAC_IP_UNROLL
+#define SP_JAC_IP_UNROLL 1
+#endif
+constexpr int kIpUnroll = SP_JAC_IP_UNROLL;  // unroll of the in-place two-sweep loop (build knob)
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
 constexpr uint64_t kNegZero2 = 0x8000000080000000ull;
 
@@ -431,12 +435,9 @@ __device__ __forceinline__ void run_steps_ip(uint64_t (&R)[kK + 1], int h, int l
                                              const FixedCells& f) {
     uint64_t left = nb_left(R[kK], lane), right = nb_right(R[1], lane);
     int k = 0;
-#ifndef SP_JAC_IP_UNROLL
-#define SP_JAC_IP_UNROLL 1
-#endif
     // (the two-sweep body is 2 x 3K packed instructions; unrolled further, the loop outgrows the
     //  instruction cache at these K — ncu: no-instruction stalls)
-#pragma unroll SP_JAC_IP_UNROLL
+#pragma unroll (kIpUnroll)
     for (; k + 2 <= h; k += 2) {
         sweep_up<kK>(R, left, right, lane, w2, mz);
         if (kBoundary) {
