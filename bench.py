@@ -545,7 +545,11 @@ def run_ours(args, rank, world, local_rank):
         "vs_baseline": None, "dtype": "f32/u8", "data": "synthetic",
         "config": bench_config(world, tt, args.halo, args.gather),
         "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4),
-                   "n_local": n_local, "passes_per_step": -(-T // tt)},
+                   "n_local": n_local, "passes_per_step": -(-T // tt),
+                   "space_tile": (sp.jacobi1d_plan(n_local, T, tt, 0)["persistent_space_tile"] if world == 1
+                                  else sp.jacobi1d_plan(n_local, T, tt, 0)["space_tile"]),
+                   "geometry": ("in place: 88 cells/lane in 45 packed registers, one stage per warp" if world == 1
+                                else "staged: 56 cells/lane, two stages per warp (peer instantiation)")},
         "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
                "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},
         "roofline": dominant, "roofline_jacobi": roof_jac, "roofline_jacobi_hbm_regime": roof_hbm,

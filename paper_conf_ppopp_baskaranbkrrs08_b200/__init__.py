@@ -86,7 +86,8 @@ class sp_buffer(ctypes.Structure):
 
 class sp_jacobi_plan(ctypes.Structure):
     _fields_ = [("n", i64), ("steps", i32), ("time_tile", i32), ("halo", i32), ("passes", i32), ("space_tile", i64),
-                ("tiles", i64), ("grid", i32), ("threads", i32), ("smem_bytes", i32), ("cells_per_thread", i32)]
+                ("tiles", i64), ("grid", i32), ("threads", i32), ("smem_bytes", i32), ("cells_per_thread", i32),
+                ("persistent_space_tile", i64), ("persistent_tiles", i64)]
 
 
 class sp_peer_links(ctypes.Structure):

@@ -63,7 +63,7 @@ struct JCfg {
 };
 constexpr int kMaxTimeTile = 128;
 #ifndef SP_JAC_IP_UNROLL
-#define SP_JAC_IP_UNROLL 1
+#define SP_JAC_IP_UNROLL 2  // K = 44: 6.73 ms (unroll 1: 7.12, 4: 6.98) on J3 at Tt = 64 (r2l)
 #endif
 constexpr int kIpUnroll = SP_JAC_IP_UNROLL;  // unroll of the in-place two-sweep loop (build knob)
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
@@ -1050,6 +1050,7 @@ Variant make_variant_peer() {
 
 constexpr int kNumVariants = 14;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
+constexpr int kPersistentVariant = 11;  // in place, K = 44 (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
 Variant* variants() {
@@ -1080,16 +1081,31 @@ int variant_index() {
     }();
     return idx;
 }
+// The persistent launch over device memory (the bench's N = 1 path) takes the in-place
+// geometry: K = 44 in K + 1 registers (4.8 % redundant halo updates at Tt = 64 instead of
+// 7.7 %), 6.73 vs 6.88 ms on J3 (A/B, r2l).  Host-mapped move-in / move-out (sp_jacobi1d_host)
+// keeps the staged TMA move-out of the default geometry: the in-place kernel's direct
+// 16-byte register stores would cross PCIe as small writes.  SP_JACOBI_VARIANT_FUSED (or
+// SP_JACOBI_VARIANT) overrides.
+int persistent_variant_index() {
+    static int idx = [] {
+        const char* e = std::getenv("SP_JACOBI_VARIANT_FUSED");
+        if (!e) e = std::getenv("SP_JACOBI_VARIANT");
+        int i = e ? std::atoi(e) : kPersistentVariant;
+        return (i >= 0 && i < kNumVariants) ? i : kPersistentVariant;
+    }();
+    return idx;
+}
 
 int smem_bytes(const Variant& v) { return v.stage_floats * (int)sizeof(float); }
 
 // occupancy of the selected variant on the current device (cached per device)
-int device_info(Variant& out) {
+int device_info(Variant& out, int vi = -1) {
     static std::mutex mu;
     static Variant cache[64][kNumVariants];
     int dev = 0;
     SP_CUDA_TRY(cudaGetDevice(&dev));
-    const int vi = variant_index();
+    if (vi < 0) vi = variant_index();
     std::lock_guard<std::mutex> lk(mu);
     Variant& d = cache[dev & 63][vi];
     if (!d.ok) {
@@ -1112,8 +1128,8 @@ int device_info(Variant& out) {
 
 inline int32_t halo_of(int32_t time_tile) { return (time_tile + 3) & ~3; }
 
-int geometry(int32_t time_tile, int32_t space_tile, int64_t& S, int32_t& wo) {
-    const Variant& v = variants()[variant_index()];
+int geometry(int32_t time_tile, int32_t space_tile, int64_t& S, int32_t& wo, int vi = -1) {
+    const Variant& v = variants()[vi < 0 ? variant_index() : vi];
     if (time_tile < 1 || time_tile > kMaxTimeTile) return SP_ERR_INVALID_ARG;
     const int32_t H = halo_of(time_tile);
     const int32_t S_max = v.strip - 2 * H;  // owned cells of a warp tile (multiple of 4)
@@ -1235,6 +1251,17 @@ extern "C" int sp_jacobi1d_plan(int64_t n, int32_t steps, int32_t time_tile, int
     out->passes = (steps + time_tile - 1) / time_tile;
     out->space_tile = S;
     out->tiles = (n + S - 1) / S;
+    {
+        int64_t Sp;
+        int32_t wp;
+        if (geometry(time_tile, space_tile, Sp, wp, persistent_variant_index()) == SP_OK) {
+            out->persistent_space_tile = Sp;
+            out->persistent_tiles = (n + Sp - 1) / Sp;
+        } else {  // (an explicit space tile above the in-place maximum cannot happen: it is larger)
+            out->persistent_space_tile = S;
+            out->persistent_tiles = out->tiles;
+        }
+    }
     const Variant& v = variants()[variant_index()];
     out->threads = v.threads;
     out->smem_bytes = smem_bytes(v);
@@ -1334,9 +1361,10 @@ extern "C" int sp_jac_dbg_read(unsigned long long* out) {
 namespace {
 // A pointer the kernel can dereference: device memory as is, page-locked host memory through
 // its device mapping (UVA: usually the same address).  Pageable host memory is rejected.
-int device_view(const void* p, const void** out) {
+int device_view(const void* p, const void** out, bool* host = nullptr) {
     cudaPointerAttributes at;
     SP_CUDA_TRY(cudaPointerGetAttributes(&at, p));
+    if (host) *host = at.type == cudaMemoryTypeHost;
     if (at.type == cudaMemoryTypeDevice || at.type == cudaMemoryTypeManaged) {
         *out = p;
         return SP_OK;
@@ -1359,15 +1387,19 @@ extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* 
         return SP_ERR_INVALID_ARG;
     for (const void* q : {(const void*)in, (const void*)out, (const void*)buf0, (const void*)buf1})
         if (reinterpret_cast<uintptr_t>(q) & 15) return SP_ERR_INVALID_ARG;
+    const float *din = nullptr, *dout = nullptr;
+    bool hin = false, hout = false;
+    int st;
+    if ((st = device_view(in, (const void**)&din, &hin)) || (st = device_view(out, (const void**)&dout, &hout)))
+        return st;
+    // device memory on both ends: the in-place geometry; host-mapped: the staged one
+    const int vi = (hin || hout) ? variant_index() : persistent_variant_index();
     int64_t S;
     int32_t wo;
-    int st = geometry(time_tile, space_tile, S, wo);
-    if (st) return st;
+    if ((st = geometry(time_tile, space_tile, S, wo, vi))) return st;
     const int64_t tiles = (n + S - 1) / S;
     if (flags_len < tiles + 1) return SP_ERR_INVALID_ARG;
     const cudaStream_t s = (cudaStream_t)stream;
-    const float *din = nullptr, *dout = nullptr;
-    if ((st = device_view(in, (const void**)&din)) || (st = device_view(out, (const void**)&dout))) return st;
     if (steps == 0) {
         if (out != in) SP_CUDA_TRY(cudaMemcpyAsync(out, in, (size_t)n * sizeof(float), cudaMemcpyDefault, s));
         return SP_OK;
@@ -1388,7 +1420,7 @@ extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* 
     if ((int64_t)passes * tiles + (int64_t(1) << 20) > INT32_MAX || tiles + skew * (passes - 1) > INT32_MAX)
         return SP_ERR_UNSUPPORTED;  // 32-bit unit counter
     Variant di;
-    if ((st = device_info(di))) return st;
+    if ((st = device_info(di, vi))) return st;
     float* bufs[2] = {buf0, buf1};
     // the last pass must not write the array it reads: then it writes bufs[passes & 1] and the
     // result is copied to out afterwards
