@@ -341,16 +341,15 @@ def run_ours(args, rank, world, local_rank):
             dist.barrier()
         torch.cuda.synchronize()
 
-    # ---- warm-up
-    for _ in range(args.warmup):
-        jacobi_step()
-        me_step()
-    barrier()
-
-    # ---- timed region: K steps, device events on the launching stream
+    # ---- timed region: K steps, device events on the launching stream.  The W warm-up steps
+    # run inside the clock sampler's context, right before the timed region (the sampler's
+    # start-up second would otherwise leave the GPU idle and its clocks ramping into step 1)
     K = args.steps
     ev = [[torch.cuda.Event(enable_timing=True) for _ in range(3)] for _ in range(K)]
     with ClockSampler(local_rank) as clk:
+        for _ in range(args.warmup):
+            jacobi_step()
+            me_step()
         barrier()
         clk.mark()
         e_start = torch.cuda.Event(enable_timing=True)
