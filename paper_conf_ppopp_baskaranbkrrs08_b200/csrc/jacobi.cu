@@ -57,8 +57,8 @@ struct JCfg {
     static constexpr int kStrip = 64 * K_;
     static constexpr int kStages = IP_ ? 1 : 2;
     static constexpr int kStage = WARPS_ * kStages * 64 * K_;  // floats of shared memory per CTA
-    static_assert(K_ % 4 == 0 && (K_ / 4) % 2 == 1 && (SE_ || IP_ || K_ <= 32),
-                  "K/4 must be odd, K <= 32 unless scalar edges or in place");
+    static_assert(K_ % 4 == 0 && ((K_ / 4) % 2 == 1 || IP_) && (SE_ || IP_ || K_ <= 32),
+                  "K/4 must be odd (staged), K <= 32 unless scalar edges or in place");
     static_assert(!(SE_ && IP_), "in-place sweeps use packed edges");
 };
 constexpr int kMaxTimeTile = 128;
@@ -379,27 +379,30 @@ __device__ __forceinline__ uint64_t nb_right(uint64_t first, int lane) {  // lan
     const float d = __shfl_sync(0xffffffffu, f2_hi(first), (lane + 1) & 31);
     return f2_pack(lane == 31 ? d : c, d);
 }
+// The four neighbour registers rotate without copies: an ascending sweep reads its left
+// neighbour first (la) and its right one last (ra), and produces the descending sweep's right
+// neighbour first (rb) and its left one last (lb); the descending sweep reads rb first and lb
+// last and produces la first and ra last — every value is written after its previous
+// holder's last read, so two sweeps return to the same registers with no moves.
 template <int kK>
-__device__ __forceinline__ void sweep_up(uint64_t (&R)[kK + 1], uint64_t& left, uint64_t& right, int lane, uint64_t w2,
-                                         uint64_t mz) {
-    R[0] = update(left, R[1], R[2], w2, mz);
-    const uint64_t rn = nb_right(R[0], lane);  // needed first by the descending sweep
+__device__ __forceinline__ void sweep_up(uint64_t (&R)[kK + 1], const uint64_t& la, const uint64_t& ra, uint64_t& rb,
+                                         uint64_t& lb, int lane, uint64_t w2, uint64_t mz) {
+    R[0] = update(la, R[1], R[2], w2, mz);
+    rb = nb_right(R[0], lane);  // needed first by the descending sweep
 #pragma unroll
     for (int j = 1; j < kK - 1; ++j) R[j] = update(R[j], R[j + 1], R[j + 2], w2, mz);
-    R[kK - 1] = update(R[kK - 1], R[kK], right, w2, mz);
-    left = nb_left(R[kK - 1], lane);  // needed last by the descending sweep
-    right = rn;
+    R[kK - 1] = update(R[kK - 1], R[kK], ra, w2, mz);
+    lb = nb_left(R[kK - 1], lane);  // needed last by the descending sweep
 }
 template <int kK>
-__device__ __forceinline__ void sweep_down(uint64_t (&R)[kK + 1], uint64_t& left, uint64_t& right, int lane,
-                                           uint64_t w2, uint64_t mz) {
-    R[kK] = update(R[kK - 2], R[kK - 1], right, w2, mz);
-    const uint64_t ln = nb_left(R[kK], lane);  // needed first by the ascending sweep
+__device__ __forceinline__ void sweep_down(uint64_t (&R)[kK + 1], const uint64_t& lb, const uint64_t& rb,
+                                           uint64_t& la, uint64_t& ra, int lane, uint64_t w2, uint64_t mz) {
+    R[kK] = update(R[kK - 2], R[kK - 1], rb, w2, mz);
+    la = nb_left(R[kK], lane);  // needed first by the ascending sweep
 #pragma unroll
     for (int j = kK - 2; j >= 1; --j) R[j + 1] = update(R[j - 1], R[j], R[j + 1], w2, mz);
-    R[1] = update(left, R[0], R[1], w2, mz);
-    right = nb_right(R[1], lane);  // needed last by the ascending sweep
-    left = ln;
+    R[1] = update(lb, R[0], R[1], w2, mz);
+    ra = nb_right(R[1], lane);  // needed last by the ascending sweep
 }
 // Dirichlet restore of a fixed cell on the element held at R[j + OFF] (jump table, as
 // restore_one; fx as in FixedCells)
@@ -433,33 +436,33 @@ __device__ __forceinline__ void restore_one_ip(uint64_t (&R)[kK + 1], int lane, 
 template <bool kBoundary, int kK>
 __device__ __forceinline__ void run_steps_ip(uint64_t (&R)[kK + 1], int h, int lane, uint64_t w2, uint64_t mz,
                                              const FixedCells& f) {
-    uint64_t left = nb_left(R[kK], lane), right = nb_right(R[1], lane);
+    uint64_t la = nb_left(R[kK], lane), ra = nb_right(R[1], lane), lb, rb;
     int k = 0;
     // (the two-sweep body is 2 x 3K packed instructions; unrolled further, the loop outgrows the
     //  instruction cache at these K — ncu: no-instruction stalls)
 #pragma unroll (kIpUnroll)
     for (; k + 2 <= h; k += 2) {
-        sweep_up<kK>(R, left, right, lane, w2, mz);
+        sweep_up<kK>(R, la, ra, rb, lb, lane, w2, mz);
         if (kBoundary) {
             restore_one_ip<kK, 0>(R, lane, f.fx0, f.v0);
             restore_one_ip<kK, 0>(R, lane, f.fx1, f.v1);
             if (f.edge) {
-                left = nb_left(R[kK - 1], lane);
-                right = nb_right(R[0], lane);
+                lb = nb_left(R[kK - 1], lane);
+                rb = nb_right(R[0], lane);
             }
         }
-        sweep_down<kK>(R, left, right, lane, w2, mz);
+        sweep_down<kK>(R, lb, rb, la, ra, lane, w2, mz);
         if (kBoundary) {
             restore_one_ip<kK, 1>(R, lane, f.fx0, f.v0);
             restore_one_ip<kK, 1>(R, lane, f.fx1, f.v1);
             if (f.edge) {
-                left = nb_left(R[kK], lane);
-                right = nb_right(R[1], lane);
+                la = nb_left(R[kK], lane);
+                ra = nb_right(R[1], lane);
             }
         }
     }
     if (k < h) {
-        sweep_up<kK>(R, left, right, lane, w2, mz);
+        sweep_up<kK>(R, la, ra, rb, lb, lane, w2, mz);
         if (kBoundary) {
             restore_one_ip<kK, 0>(R, lane, f.fx0, f.v0);
             restore_one_ip<kK, 0>(R, lane, f.fx1, f.v1);
@@ -1048,7 +1051,7 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 14;
+constexpr int kNumVariants = 15;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
 constexpr int kPersistentVariant = 11;  // in place, K = 44 (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
@@ -1069,6 +1072,7 @@ Variant* variants() {
         make_variant<JCfg<44, 8, 2, false, true>>(),  // 11: in place, 88 cells/lane, 16 warps/SM, one stage (176 KB)
         make_variant<JCfg<36, 8, 2, false, true>>(),  // 12: in place, 72 cells/lane, 16 warps/SM (144 KB)
         make_variant<JCfg<52, 8, 2, false, true>>(),  // 13: in place, 104 cells/lane, 16 warps/SM (208 KB)
+        make_variant<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
     };
     return v;
 }
