@@ -547,7 +547,7 @@ def run_ours(args, rank, world, local_rank):
                    "n_local": n_local, "passes_per_step": -(-T // tt),
                    "space_tile": (sp.jacobi1d_plan(n_local, T, tt, 0)["persistent_space_tile"] if world == 1
                                   else sp.jacobi1d_plan(n_local, T, tt, 0)["space_tile"]),
-                   "geometry": ("in place: 88 cells/lane in 45 packed registers, one stage per warp" if world == 1
+                   "geometry": ("in place: 80 cells/lane in 41 packed registers, one stage per warp" if world == 1
                                 else "staged: 56 cells/lane, two stages per warp (peer instantiation)")},
         "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
                "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},

@@ -185,7 +185,7 @@ typedef struct {
     int32_t smem_bytes;  /* dynamic shared memory per CTA */
     int32_t cells_per_thread; /* register cells per thread */
     /* the persistent launch over DEVICE memory (sp_jacobi1d_timetiled_fused, _stream with
-     * device in / out) uses the in-place geometry: 88 register cells per thread in 45 packed
+     * device in / out) uses the in-place geometry: 80 register cells per thread in 41 packed
      * registers, alternating sweeps; with space_tile = 0 its tile is larger: */
     int64_t persistent_space_tile; /* S of that launch (space_tile if given) */
     int64_t persistent_tiles;      /* its tiles per pass (<= tiles: flags sized by `tiles` suffice) */
@@ -218,8 +218,8 @@ int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32
  * Every CTA of the launch must be co-resident (the grid is the occupancy limit); a tile whose
  * dependences never complete traps after ~20 s instead of hanging.  footprint_log as in
  * sp_jacobi1d_timetiled, laid out [passes][persistent_tiles][2] (sp_jacobi1d_plan).
- * Geometry: the in-place kernel (sp_jacobi_plan.persistent_space_tile): each lane keeps 44
- * packed cell pairs in 45 registers and alternates ascending / descending sweeps, so no second
+ * Geometry: the in-place kernel (sp_jacobi_plan.persistent_space_tile): each lane keeps 40
+ * packed cell pairs in 41 registers and alternates ascending / descending sweeps, so no second
  * register copy is needed; the tile is staged once per warp and stored from registers. */
 int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n, int32_t steps,
                                 int32_t time_tile, int32_t space_tile, int64_t* footprint_log, void* stream);

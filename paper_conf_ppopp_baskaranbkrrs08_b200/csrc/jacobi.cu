@@ -63,7 +63,7 @@ struct JCfg {
 };
 constexpr int kMaxTimeTile = 128;
 #ifndef SP_JAC_IP_UNROLL
-#define SP_JAC_IP_UNROLL 2  // K = 44: 6.73 ms (unroll 1: 7.12, 4: 6.98) on J3 at Tt = 64 (r2l)
+#define SP_JAC_IP_UNROLL 2  // K = 40: 6.59-6.64 ms (unroll 1: 6.97, 4: 6.75) on J3 at Tt = 64 (r2o)
 #endif
 constexpr int kIpUnroll = SP_JAC_IP_UNROLL;  // unroll of the in-place two-sweep loop (build knob)
 constexpr uint32_t kW = 0x3EAAAAABu;  // fl32(1/3)
@@ -1053,7 +1053,7 @@ Variant make_variant_peer() {
 
 constexpr int kNumVariants = 15;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
-constexpr int kPersistentVariant = 11;  // in place, K = 44 (profiles/r02_jacobi_inplace.txt)
+constexpr int kPersistentVariant = 14;  // in place, K = 40 (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
 Variant* variants() {
@@ -1086,8 +1086,9 @@ int variant_index() {
     return idx;
 }
 // The persistent launch over device memory (the bench's N = 1 path) takes the in-place
-// geometry: K = 44 in K + 1 registers (4.8 % redundant halo updates at Tt = 64 instead of
-// 7.7 %), 6.73 vs 6.88 ms on J3 (A/B, r2l).  Host-mapped move-in / move-out (sp_jacobi1d_host)
+// geometry: K = 40 in K + 1 registers (5.3 % redundant halo updates at Tt = 64 instead of
+// 7.7 %), 6.59-6.64 vs 6.87 ms on J3 (A/B, r2o; K = 44: 6.74 — its loop keeps 16 register
+// moves per 4 steps on the FMA pipe at the 128-register limit, K = 40's keeps 3).  Host-mapped move-in / move-out (sp_jacobi1d_host)
 // keeps the staged TMA move-out of the default geometry: the in-place kernel's direct
 // 16-byte register stores would cross PCIe as small writes.  SP_JACOBI_VARIANT_FUSED (or
 // SP_JACOBI_VARIANT) overrides.
