@@ -415,6 +415,7 @@ int sp_jacobi1d_timetiled_peer(const sp_peer_links* links, float* a_local, float
  * 2 * passes] (tiles = ceil(n_local / space tile)), zeroed by the call; same links, buffer
  * layout and epoch protocol as sp_jacobi1d_timetiled_peer (advance epoch0 by the pass count
  * between calls).  All ranks of a run must use the same entry point. */
+/* (Geometry: the in-place kernel of sp_jacobi1d_timetiled_fused, with the peer push.) */
 int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* links, float* a_local, float* work_local, int32_t* flags,
                                      int64_t flags_len, int64_t n_global, int64_t x_begin, int64_t n_local,
                                      int32_t steps, int32_t time_tile, int32_t space_tile, void* stream);

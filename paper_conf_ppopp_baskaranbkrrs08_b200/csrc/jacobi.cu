@@ -577,7 +577,6 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
     float* const stage0 = smem + warp * Cfg::kStages * kStrip;  // this warp's stage(s)
     constexpr bool kIP = Cfg::kInPlace;
-    static_assert(!(kIP && kPeer), "the in-place geometry has no peer instantiation");
     uint64_t* const bar = full[warp];
     const uint64_t w2 = (uint64_t(kW) << 32) | kW;
     const int64_t GW = (int64_t)gridDim.x * Cfg::kWarps;
@@ -995,7 +994,9 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             const bool eL = A.pushL[0] && x0 < A.own_begin + A.H;
             const bool eR = A.pushR[0] && x0 + st > A.own_end - A.H;
             if (eL || eR) {  // warp-uniform
-                if (lane == 0) {
+                if constexpr (kIP) {
+                    __threadfence();  // every lane's direct stores of this tile are visible (GPU scope)
+                } else if (lane == 0) {
                     bulk_wait0();  // this tile's cells are in global memory ...
                     fence_proxy_async_global();  // ... and ordered before the release below
                 }
@@ -1028,7 +1029,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 struct Variant {
     int K, warps, threads, strip, stage_floats;
     void (*kernel)(PassArgs);
-    void (*kernel_peer)(PassArgs) = nullptr;  // kPeer instantiation (default variant only)
+    void (*kernel_peer)(PassArgs) = nullptr;  // kPeer instantiation (default and persistent variants)
     int sms = 0, occ = 0, occ_peer = 0;
     bool ok = false;
 };
@@ -1072,7 +1073,7 @@ Variant* variants() {
         make_variant<JCfg<44, 8, 2, false, true>>(),  // 11: in place, 88 cells/lane, 16 warps/SM, one stage (176 KB)
         make_variant<JCfg<36, 8, 2, false, true>>(),  // 12: in place, 72 cells/lane, 16 warps/SM (144 KB)
         make_variant<JCfg<52, 8, 2, false, true>>(),  // 13: in place, 104 cells/lane, 16 warps/SM (208 KB)
-        make_variant<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
+        make_variant_peer<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
     };
     return v;
 }
@@ -1542,7 +1543,8 @@ extern "C" int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* L, float* a
         return SP_ERR_INVALID_ARG;
     int64_t S;
     int32_t wo;
-    int st = geometry(time_tile, space_tile, S, wo);
+    const int vi = persistent_variant_index();  // (the in-place geometry, as the single-GPU persistent launch)
+    int st = geometry(time_tile, space_tile, S, wo, vi);
     if (st) return st;
     const int32_t H = halo_of(time_tile);
     if ((has_left || has_right) && n_local < H) return SP_ERR_INVALID_ARG;
@@ -1552,7 +1554,7 @@ extern "C" int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* L, float* a
     if (flags_len < tiles + 1 + 2 * (int64_t)passes) return SP_ERR_INVALID_ARG;
     if ((int64_t)passes * tiles + (int64_t(1) << 20) > INT32_MAX) return SP_ERR_UNSUPPORTED;
     Variant di;
-    if ((st = device_info(di))) return st;
+    if ((st = device_info(di, vi))) return st;
     const cudaStream_t s = (cudaStream_t)stream;
     SP_CUDA_TRY(cudaMemsetAsync(flags, 0, (size_t)(tiles + 1 + 2 * (int64_t)passes) * sizeof(int32_t), s));
     // edge tiles per side: tile t (owned [x0, x0 + st)) produces one of the first / last H
