@@ -46,6 +46,12 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 #ifndef SP_ME_EXP
 #define SP_ME_EXP 0
 #endif
+#ifndef SP_ME_SKIP
+#define SP_ME_SKIP 1
+#endif
+#ifndef SP_ME_SCRAMBLE
+#define SP_ME_SCRAMBLE 1
+#endif
 #if SP_ME_EXP & 32  // development instrumentation: (smid, start, end) global timer per CTA
 __device__ unsigned long long g_me_cta[4096][3];
 __device__ __forceinline__ unsigned long long globaltimer() {
@@ -93,6 +99,7 @@ struct MeArgs {
     uint32_t flat_mb0;
     int32_t pair_base;
     uint32_t total_mb;  // macroblocks of this launch (fast kernel)
+    uint32_t nrows;     // macroblock rows of this launch (total_mb / mbx)
 };
 
 // Fused all-gather of the results over peer memory (sp_me_sad_search_gather): every
@@ -231,10 +238,19 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         int pair, byr, bx;
     };
     auto locate = [&](uint32_t mb) -> Pos {
+#if SP_ME_SCRAMBLE
+        // column-major over the launch's macroblock rows: consecutive grabs come from
+        // different rows, so the border rows (whose dead warps skip their main candidates)
+        // spread over the whole launch instead of coinciding on every SM
+        const uint32_t col = mb / A.nrows, f = mb - col * A.nrows + A.flat_mb0 / mbx;
+        const uint32_t pair = f / (uint32_t)A.mb_rows;
+        return Pos{(int)pair, (int)(f - pair * (uint32_t)A.mb_rows), (int)col};
+#else
         mb += A.flat_mb0;
         const uint32_t pair = mb / per_pair, rem = mb - pair * per_pair;
         const uint32_t byr = rem / mbx;
         return Pos{(int)pair, (int)byr, (int)(rem - byr * mbx)};
+#endif
     };
     auto issue = [&](uint32_t mb, int st) {  // single thread: stage the window + cur of mb
         const Pos q = locate(mb);
@@ -417,6 +433,19 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // lower ones build the next macroblock's copies while these still read this one's
         if (warp >= nwarps / 2) __nanosleep(20000);
 #endif
+        // ---- validity (restricted vectors) only matters near the frame border ----------
+        const Pos q = posS[s];  // (written one macroblock ahead; stable until the next barrier)
+        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
+        const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
+        const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
+        const bool interior = A.unrestricted || (dxlo == -R && dxhi == R && dylo == -R && dyhi == R);
+        // a warp whose whole band of main dy candidates is invalid skips them (warp-uniform;
+        // 4-warp CTAs: warp w holds dy in [-R + 16 w, -R + 16 w + 15]); its tails still run
+        bool main_dead = false;
+        if (SP_ME_SKIP && nwarps > 1 && !interior && !A.surface) {
+            const int blo = -R + 2 * kTy * warp, bhi = blo + 2 * kTy - 1;
+            main_dead = bhi < dylo || blo > dyhi;
+        }
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
         //      thread's tail candidates, all in one row loop ----
         uint32_t acc[kTx][kTy];
@@ -431,7 +460,20 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             tp[t] = smem + tinfo[t][1 + (G::kPhaseSets == 1 ? 0 : s)][tid];
             ta[t] = 0;
         }
-        {
+        if (main_dead) {  // tails only (one LDS.128 of the current row, 4 LDS.32 + 4 SADs per tail)
+            const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+#pragma unroll 4
+            for (int v = 0; v < kMB; ++v) {
+                const uint4 cv = cq[v];
+                const uint32_t Cv[4] = {cv.x, cv.y, cv.z, cv.w};
+#pragma unroll
+                for (int t = 0; t < G::kTailPer; ++t) {
+                    const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
+#pragma unroll
+                    for (int k = 0; k < 4; ++k) ta[t] = sad4(tq[k], Cv[k], ta[t]);
+                }
+            }
+        } else {
             // Candidate (j, i) compares cur row v with window row 8d + i + v.  Loop over v with
             // a ring of the 8 window rows in use (row rho in slot rho & 7, 7 words each: the
             // 4 dx candidates x 4 words of one byte phase); body unrolled 8x so every ring
@@ -499,13 +541,6 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             if (lane == 0) lsum[s] = tot;
         }
         PMARK(4);
-
-        // ---- validity (restricted vectors) only matters near the frame border ----------
-        const Pos q = posS[s];  // (written one macroblock ahead; stable until the next barrier)
-        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
-        const int dxlo = -x0 > -R ? -x0 : -R, dxhi = W - 16 - x0 < R ? W - 16 - x0 : R;
-        const int dylo = -y0 > -R ? -y0 : -R, dyhi = Hf - 16 - y0 < R ? Hf - 16 - y0 : R;
-        const bool interior = A.unrestricted || (dxlo == -R && dxhi == R && dylo == -R && dyhi == R);
         if (!interior) {
 #pragma unroll
             for (int j = 0; j < kTx; ++j) {
@@ -838,7 +873,7 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
     if (n_pairs == 0 || rows == 0 || mbx == 0) return SP_OK;
     const cudaStream_t s = (cudaStream_t)stream;
     MeArgs a{width, frame_height, row0_global, range, n_pairs, mbx, mb_row_begin, rows, 2 * range + 16, pad,
-             pad > 0 ? 1 : 0, mv, best_sad, surface, ready, nullptr, 0u, 0, 0u};
+             pad > 0 ? 1 : 0, mv, best_sad, surface, ready, nullptr, 0u, 0, 0u, 0u};
     const GatherArgs nox{};
     if (fast_range(range)) {
         int st0;
@@ -854,6 +889,7 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
         const int64_t total = (int64_t)mbx * rows * n_pairs;
         if (total >= (int64_t(1) << 31)) return SP_ERR_UNSUPPORTED;  // 32-bit macroblock indices in the kernel
         a.total_mb = (uint32_t)total;
+        a.nrows = (uint32_t)(rows * n_pairs);
         // (the streamed-frames variant is a separate instantiation: the flag wait in its move-in
         // costs the device-resident kernel its uniform-datapath index math, 2 % of M4)
         if (range == 32)
@@ -924,7 +960,7 @@ int me_range_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t
     }
     MeArgs a{width, frame_height, 0, range, n_pairs_buffer, (int32_t)mbx, 0, (int32_t)mby, 2 * range + 16, 0, 0,
              mv, best_sad, nullptr, nullptr, nullptr, (uint32_t)(flat_begin * mbx), pair_base,
-             (uint32_t)((flat_end - flat_begin) * mbx)};
+             (uint32_t)((flat_end - flat_begin) * mbx), (uint32_t)(flat_end - flat_begin)};
     int st;
     if ((st = counter_slot(s, &a.counter))) return st;
     CUtensorMap rm, cm;
