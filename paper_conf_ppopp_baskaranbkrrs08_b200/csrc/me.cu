@@ -46,11 +46,15 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 #ifndef SP_ME_EXP
 #define SP_ME_EXP 0
 #endif
+// SP_ME_SKIP: a warp whose whole dy band of main candidates is invalid (the first two and the
+// last macroblock rows at 1080p, R = 32) runs only its tail candidates: M4 8.368 -> 8.327 ms
+// (A/B, r2t).  SP_ME_SCRAMBLE (off): column-major macroblock order, meant to spread those rows
+// over the launch, measured slower (8.43 ms).
 #ifndef SP_ME_SKIP
 #define SP_ME_SKIP 1
 #endif
 #ifndef SP_ME_SCRAMBLE
-#define SP_ME_SCRAMBLE 1
+#define SP_ME_SCRAMBLE 0
 #endif
 #if SP_ME_EXP & 32  // development instrumentation: (smid, start, end) global timer per CTA
 __device__ unsigned long long g_me_cta[4096][3];
