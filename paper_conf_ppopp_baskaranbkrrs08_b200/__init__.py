@@ -741,28 +741,23 @@ class MEShard:
             self.n_pairs, self.mby, self.mbx)
         dist.barrier()
 
-    def needed_rows(self, f: int) -> tuple[int, int]:
-        """Rows [r0, r1) of global frame f this rank's range reads (empty: (0, 0)): as the
+    def needed_rows(self, f: int) -> list[tuple[int, int]]:
+        """Rows of global frame f this rank's range reads, as disjoint intervals [r0, r1): as the
         reference of pair f (band rows with the R-row halo) and as the current frame of pair f - 1."""
         from . import partition
-        lo, hi = self.height, 0
-        for p, r0, r1 in self.pieces:
-            if p == f:  # ref
-                a, b = partition.me_band_rows(r0, r1, self.height, self.range)
-                lo, hi = min(lo, a), max(hi, b)
-            if p + 1 == f:  # cur
-                lo, hi = min(lo, 16 * r0), max(hi, 16 * r1)
-        return (lo, hi) if lo < hi else (0, 0)
+        return partition.me_needed_rows(self.pieces, f, self.height, self.range)
 
     def load_frames(self, frame_fn):
         """Fill the needed rows of this rank's frames from frame_fn(f) -> host uint8 [H, >= W]."""
         import torch
         for k in range(self.frames.shape[0]):
             f = self.pair_base + k
-            r0, r1 = self.needed_rows(f)
-            if r1 > r0:
-                fr = np.ascontiguousarray(np.asarray(frame_fn(f))[r0:r1, : self.width])
-                self.frames[k, r0:r1, : self.width].copy_(torch.from_numpy(fr))
+            bands = self.needed_rows(f)
+            if bands:
+                full = np.asarray(frame_fn(f))
+                for r0, r1 in bands:
+                    fr = np.ascontiguousarray(full[r0:r1, : self.width])
+                    self.frames[k, r0:r1, : self.width].copy_(torch.from_numpy(fr))
 
     def run(self, stream=None):
         """Search this rank's range; every rank's results land in every rank's mv / sad

@@ -68,3 +68,23 @@ def split_flat_range(begin: int, end: int, mby: int) -> list[tuple[int, int, int
         out.append((p, r, r + (e - k)))
         k = e
     return out
+
+
+def me_needed_rows(pieces, f: int, frame_height: int, search_range: int) -> list[tuple[int, int]]:
+    """Rows of global frame f that the range `pieces` (split_flat_range output) reads, as sorted
+    disjoint intervals [r0, r1): as the reference of pair f (the band rows with the R-row halo,
+    me_band_rows) and as the current frame of pair f - 1 (the current blocks' rows).  A range that
+    ends inside pair f - 1 and starts pair f needs two separate bands of frame f."""
+    iv = []
+    for p, r0, r1 in pieces:
+        if p == f:  # reference frame of pair p
+            iv.append(me_band_rows(r0, r1, frame_height, search_range))
+        if p + 1 == f:  # current frame of pair p
+            iv.append((16 * r0, 16 * r1))
+    out = []
+    for a, b in sorted(x for x in iv if x[1] > x[0]):
+        if out and a <= out[-1][1]:
+            out[-1] = (out[-1][0], max(out[-1][1], b))
+        else:
+            out.append((a, b))
+    return out
