@@ -437,11 +437,12 @@ template <bool kBoundary, int kK>
 __device__ __forceinline__ void run_steps_ip(uint64_t (&R)[kK + 1], int h, int lane, uint64_t w2, uint64_t mz,
                                              const FixedCells& f) {
     uint64_t la = nb_left(R[kK], lane), ra = nb_right(R[1], lane), lb, rb;
-    int k = 0;
+    const bool odd = h & 1;
     // (the two-sweep body is 2 x 3K packed instructions; unrolled further, the loop outgrows the
-    //  instruction cache at these K — ncu: no-instruction stalls)
+    //  instruction cache at these K — ncu: no-instruction stalls.  One down-counter: at the
+    //  128-register limit every loop-carried scalar counts)
 #pragma unroll (kIpUnroll)
-    for (; k + 2 <= h; k += 2) {
+    for (int r = h >> 1; r > 0; --r) {
         sweep_up<kK>(R, la, ra, rb, lb, lane, w2, mz);
         if (kBoundary) {
             restore_one_ip<kK, 0>(R, lane, f.fx0, f.v0);
@@ -461,7 +462,7 @@ __device__ __forceinline__ void run_steps_ip(uint64_t (&R)[kK + 1], int h, int l
             }
         }
     }
-    if (k < h) {
+    if (odd) {
         sweep_up<kK>(R, la, ra, rb, lb, lane, w2, mz);
         if (kBoundary) {
             restore_one_ip<kK, 0>(R, lane, f.fx0, f.v0);
