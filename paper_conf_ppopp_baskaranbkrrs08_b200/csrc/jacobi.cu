@@ -1053,7 +1053,7 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 18;
+constexpr int kNumVariants = 15;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
 constexpr int kPersistentVariant = 14;  // in place, K = 40 (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
@@ -1075,10 +1075,8 @@ Variant* variants() {
         make_variant<JCfg<36, 8, 2, false, true>>(),  // 12: in place, 72 cells/lane, 16 warps/SM (144 KB)
         make_variant<JCfg<52, 8, 2, false, true>>(),  // 13: in place, 104 cells/lane, 16 warps/SM (208 KB)
         make_variant_peer<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
-        make_variant<JCfg<32, 4, 5, false, true>>(),  // 15: in place, 64 cells/lane, 20 warps/SM (<= 102 registers)
-        make_variant<JCfg<36, 4, 5, false, true>>(),  // 16: in place, 72 cells/lane, 20 warps/SM
-        make_variant<JCfg<28, 4, 6, false, true>>(),  // 17: in place, 56 cells/lane, 24 warps/SM (<= 85 registers)
-    };
+    };  // (in place at 20 / 24 warps per SM, <= 102 / 85 registers, spilled into the loop:
+        //  7.45-8.9 ms on J3, profiles/r02_jacobi_inplace.txt r2x)
     return v;
 }
 
