@@ -78,6 +78,24 @@ __device__ unsigned long long g_me_prof[8];
     } while (0)
 #endif
 
+// Division of a 32-bit index by a launch constant d >= 1 with a host-computed magic number
+// (Granlund-Montgomery, exact for every 32-bit n): one IMAD.HI, two shifts and two adds instead
+// of the ~20-instruction reciprocal sequence — the macroblock index -> (pair, row, column)
+// split runs on one thread per macroblock, serially in the one-warp R = 16 CTAs.
+struct FastDiv {
+    uint32_t m, s1, s2;
+};
+inline FastDiv make_fastdiv(uint32_t d) {
+    uint32_t l = 0;
+    while (l < 32 && (uint64_t(1) << l) < d) ++l;  // l = ceil(log2 d)
+    const uint64_t m = ((uint64_t(1) << 32) * ((uint64_t(1) << l) - d)) / d + 1;
+    return FastDiv{(uint32_t)m, l < 1 ? l : 1u, l < 1 ? 0u : l - 1};
+}
+__device__ __forceinline__ uint32_t fdiv(uint32_t n, const FastDiv& f) {
+    const uint32_t t = __umulhi(f.m, n);
+    return (t + ((n - t) >> f.s1)) >> f.s2;
+}
+
 struct MeArgs {
     int32_t width, frame_height, row0, range, n_pairs;
     int32_t mbx, mb_row_begin, mb_rows;
@@ -104,6 +122,7 @@ struct MeArgs {
     int32_t pair_base;
     uint32_t total_mb;  // macroblocks of this launch (fast kernel)
     uint32_t nrows;     // macroblock rows of this launch (total_mb / mbx)
+    FastDiv div_per_pair, div_mbx;  // by mb_rows * mbx and by mbx
 };
 
 // Fused all-gather of the results over peer memory (sp_me_sad_search_gather): every
@@ -251,8 +270,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         return Pos{(int)pair, (int)(f - pair * (uint32_t)A.mb_rows), (int)col};
 #else
         mb += A.flat_mb0;
-        const uint32_t pair = mb / per_pair, rem = mb - pair * per_pair;
-        const uint32_t byr = rem / mbx;
+        const uint32_t pair = fdiv(mb, A.div_per_pair), rem = mb - pair * per_pair;
+        const uint32_t byr = fdiv(rem, A.div_mbx);
         return Pos{(int)pair, (int)byr, (int)(rem - byr * mbx)};
 #endif
     };
@@ -894,6 +913,8 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
         if (total >= (int64_t(1) << 31)) return SP_ERR_UNSUPPORTED;  // 32-bit macroblock indices in the kernel
         a.total_mb = (uint32_t)total;
         a.nrows = (uint32_t)(rows * n_pairs);
+        a.div_per_pair = make_fastdiv((uint32_t)(rows * mbx));
+        a.div_mbx = make_fastdiv((uint32_t)mbx);
         // (the streamed-frames variant is a separate instantiation: the flag wait in its move-in
         // costs the device-resident kernel its uniform-datapath index math, 2 % of M4)
         if (range == 32)
@@ -965,6 +986,8 @@ int me_range_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_t
     MeArgs a{width, frame_height, 0, range, n_pairs_buffer, (int32_t)mbx, 0, (int32_t)mby, 2 * range + 16, 0, 0,
              mv, best_sad, nullptr, nullptr, nullptr, (uint32_t)(flat_begin * mbx), pair_base,
              (uint32_t)((flat_end - flat_begin) * mbx), (uint32_t)(flat_end - flat_begin)};
+    a.div_per_pair = make_fastdiv((uint32_t)(mby * mbx));
+    a.div_mbx = make_fastdiv((uint32_t)mbx);
     int st;
     if ((st = counter_slot(s, &a.counter))) return st;
     CUtensorMap rm, cm;
