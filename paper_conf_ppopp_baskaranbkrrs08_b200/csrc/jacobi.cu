@@ -15,7 +15,12 @@
 //     warp strips overlap by H cells on each side, so h steps need no barrier at all
 //     (overlapped "concurrent start" tiling, reading R-J4);
 //   * move-out (H7): only owned cells, at the final step (reading R-J5), registers ->
-//     shared memory -> coalesced 128-bit global stores.
+//     shared memory -> TMA bulk store.
+// Two geometries (JCfg): the staged one (two register copies of 56 cells per lane, two
+// shared-memory stages per warp) and, for the persistent launches over device memory, the
+// in-place one (80 cells per lane in 41 packed registers updated by alternating ascending /
+// descending sweeps, one stage per warp, direct 16-byte register -> global move-out), which
+// fits longer strips in the same registers: 5.3 % instead of 7.7 % redundant halo updates.
 // Arithmetic is b = ((a[i-1] + a[i]) + a[i+1]) * w, each op rounded to nearest fp32, never
 // contracted (PTX add.rn/mul.rn), w = fl32(1/3) — bit-identical to the definition.
 #include <cooperative_groups.h>
