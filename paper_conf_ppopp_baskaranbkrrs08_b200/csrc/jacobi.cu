@@ -67,6 +67,9 @@ struct JCfg {
     static_assert(!(SE_ && IP_), "in-place sweeps use packed edges");
 };
 constexpr int kMaxTimeTile = 128;
+#ifndef SP_JAC_TIMING
+#define SP_JAC_TIMING 0  // timing-only builds (wrong results): 1 no dependence waits, 2 no publication, 4 static units
+#endif
 #ifndef SP_JAC_IP_UNROLL
 #define SP_JAC_IP_UNROLL 2  // K = 40: 6.59-6.64 ms (unroll 1: 6.97, 4: 6.75) on J3 at Tt = 64 (r2o)
 #endif
@@ -631,7 +634,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         if constexpr (kPeer) {
             if (pers && !peer_ready(t, pass)) return false;
         }
-        if (!pers || pass == 0) return true;
+        if (!pers || pass == 0 || (SP_JAC_TIMING & 1)) return true;
         bool ok = true;
         for (int64_t q0 = t - reach; q0 <= t + reach; q0 += 32) {
             const int64_t q = q0 + lane;
@@ -746,7 +749,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         }
     };
     auto grab = [&](int64_t u_static) -> int64_t {  // warp-uniform
-        if (!pers) return u_static;
+        if (!pers || (SP_JAC_TIMING & 4)) return u_static;
         int v = 0;
         if (lane == 0) v = atomicAdd(next_unit, 1);
         return (int64_t)__shfl_sync(0xffffffffu, v, 0);
@@ -761,7 +764,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
     }
     __syncwarp();
     auto publish = [&](bool all) {  // lane 0: the oldest unpublished tile (all: every one)
-        if (pub_t[0] < 0 || (!all && pub_t[1] < 0)) return;
+        if (pub_t[0] < 0 || (!all && pub_t[1] < 0) || (SP_JAC_TIMING & 2)) return;
         if constexpr (!kIP) {
             if (all) bulk_wait0();
             else bulk_wait1();            // every store but the newest tile's has completed
@@ -862,7 +865,8 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         if (lane == 0 && pers) publish(A.skew != 0);
         if (u_next < total) {
             pending = (pers && pn > 0 && 2 * reach < 32)
-                          ? (!__all_sync(0xffffffffu, next_flag >= pn) || (kPeer && !peer_ready(tn, pn)))
+                          ? (!(SP_JAC_TIMING & 1) && !__all_sync(0xffffffffu, next_flag >= pn)) ||
+                                (kPeer && !peer_ready(tn, pn))
                           : !deps_ready(tn, pn);
             if constexpr (kIP) {
                 // one stage: the next tile streams into the buffer this tile was just loaded
