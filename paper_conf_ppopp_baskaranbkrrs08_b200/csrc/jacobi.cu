@@ -68,7 +68,7 @@ struct JCfg {
 };
 constexpr int kMaxTimeTile = 128;
 #ifndef SP_JAC_TIMING
-#define SP_JAC_TIMING 0  // timing-only builds (wrong results): 1 no dependence waits, 2 no publication, 4 static units
+#define SP_JAC_TIMING 0  // timing-only builds (wrong results): 1 no dependence waits, 2 no publication, 4 static units, 8 twice the steps per tile
 #endif
 #ifndef SP_JAC_IP_UNROLL
 #define SP_JAC_IP_UNROLL 2  // K = 40: 6.59-6.64 ms (unroll 1: 6.97, 4: 6.75) on J3 at Tt = 64 (r2o)
@@ -890,8 +890,9 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         // ---- h steps in registers ---------------------------------------------------
         {
             if constexpr (kIP) {
-                if (boundary) run_steps_ip<true, kK>(P, h, lane, w2, A.mz, fc);
-                else run_steps_ip<false, kK>(P, h, lane, w2, A.mz, fc);
+                const int hh = (SP_JAC_TIMING & 8) ? 2 * h : h;  // (timing: loop time vs tile-boundary time)
+                if (boundary) run_steps_ip<true, kK>(P, hh, lane, w2, A.mz, fc);
+                else run_steps_ip<false, kK>(P, hh, lane, w2, A.mz, fc);
             } else if constexpr (Cfg::kScalarEdges) {
                 // pair index holding global cell 0 / n-1 in this lane's u / v range (-1: none)
                 int ju0 = -1, jv0 = -1, jun = -1, jvn = -1;
