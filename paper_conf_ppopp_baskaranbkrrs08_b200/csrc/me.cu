@@ -40,7 +40,7 @@ namespace {
 using namespace sp::ptx;
 
 constexpr int kMB = 16;      // macroblock edge (WS = 16)
-constexpr int kTy = 8;       // dy candidates per thread
+constexpr int kTy = 8;       // dy candidates per thread (R = 32; MeGeom<R>::kTy)
 constexpr int kTx = 4;       // dx candidates per thread (same byte phase, stride 4)
 
 #ifndef SP_ME_EXP
@@ -53,6 +53,10 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 #ifndef SP_ME_SKIP
 #define SP_ME_SKIP 1
 #endif
+#ifndef SP_ME_R16_TY
+#define SP_ME_R16_TY 4
+#endif
+constexpr int sp_me_kTy = 8;
 #ifndef SP_ME_SCRAMBLE
 #define SP_ME_SCRAMBLE 0
 #endif
@@ -161,6 +165,8 @@ template <int R>
 struct MeGeom {
     static constexpr int kWin = 2 * R + 16;              // window edge (bytes per row, rows)
     static constexpr int kCopy = kWin * kWin;            // bytes per staged copy (multiple of 128)
+    // R = 16: 4 x 4 tiles over two warps (SP_ME_R16_TY 4; 8 = one warp of 4 x 8 tiles)
+    static constexpr int kTy = R == 16 ? SP_ME_R16_TY : ::sp_me_kTy;
     static constexpr int kThreads = R * R / kTy;         // one 4 x kTy candidate tile per thread
     static constexpr int kWarps = kThreads / 32;         // 4 (R = 32) or 1 (R = 16)
     static constexpr int kGx = R / 8;                    // dx groups per byte phase
@@ -182,7 +188,8 @@ struct MeGeom {
     static constexpr int kSmem = kOffPh + 3 * kPhaseSets * kSlot + 128;  // + alignment slack
     static_assert(kCopy % 128 == 0, "copies must keep 128-byte alignment");
     static_assert(kSlot >= kCopy + 3 * 32 && kSlot % 128 == 0, "phase copy slots must not overlap");
-    static_assert(kWarps == 1 || kWarps == 4, "tail mapping assumes 1 or 4 warps");
+    static_assert(kWarps == 1 || kWarps == 2 || kWarps == 4, "tail mapping assumes 1, 2 or 4 warps");
+    static constexpr int kMinBlocks = kWarps == 4 ? 4 : kWarps == 2 ? 11 : 16;  // CTAs per SM (registers)
     static_assert(kTailPer * kThreads == 4 * R, "tail candidates must spread evenly");
 };
 
@@ -204,8 +211,9 @@ __device__ __forceinline__ uint32_t tie_bits(int dx, int dy, int R) {
 // over warp 0.  Row tails of one warp read consecutive dx (conflict-free words).
 template <int R>
 __device__ __forceinline__ bool tail_candidate(int warp, int lane, int t, int& dx, int& dy) {
-    const bool col = MeGeom<R>::kWarps == 4 ? warp < 2 : t == 0;
-    const int k = MeGeom<R>::kWarps == 4 ? 32 * (warp & 1) + lane : lane;
+    constexpr int nw = MeGeom<R>::kWarps;
+    const bool col = nw == 4 ? warp < 2 : nw == 2 ? warp == 0 : t == 0;
+    const int k = nw == 4 ? 32 * (warp & 1) + lane : lane;
     dx = col ? R : -R + k;
     dy = col ? -R + k : R;
     return col;
@@ -230,10 +238,11 @@ __device__ __noinline__ void wait_ready(const int32_t* flag) {
 enum { kPlain = 0, kStreamed = 1, kGather = 2 };
 
 template <int R, int kMode>
-__global__ void __launch_bounds__(MeGeom<R>::kThreads, (R == 32 ? 4 : 16))
+__global__ void __launch_bounds__(MeGeom<R>::kThreads, MeGeom<R>::kMinBlocks)
 me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant__ CUtensorMap cur_map, MeArgs A,
               const __grid_constant__ GatherArgs X) {
     using G = MeGeom<R>;
+    constexpr int kTy = G::kTy;  // (shadows the R = 32 default)
     constexpr bool kStream = kMode == kStreamed;
     constexpr int win = G::kWin;
     constexpr int side = 2 * R + 1;
@@ -356,7 +365,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     // per d (tie(j, i) = A_j + B_i, no carries between the fields)
     constexpr int kDy = G::kThreads / (4 * G::kGx);
     __shared__ uint4 tieA[4 * G::kGx];
-    __shared__ uint4 tieB[kDy][2];
+    __shared__ uint4 tieB[kDy][kTy / 4];
     if (tid < 4 * G::kGx) {
         uint32_t a[4];
         for (int j = 0; j < 4; ++j) {
@@ -366,13 +375,12 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         tieA[tid] = make_uint4(a[0], a[1], a[2], a[3]);
     }
     if (tid < kDy) {
-        uint32_t b[8];
-        for (int i = 0; i < 8; ++i) {
+        uint32_t b[kTy];
+        for (int i = 0; i < kTy; ++i) {
             const int dy = -R + kTy * tid + i;
             b[i] = ((uint32_t)abs(dy) << 8) | ((uint32_t)(dy + R) << 1);
         }
-        tieB[tid][0] = make_uint4(b[0], b[1], b[2], b[3]);
-        tieB[tid][1] = make_uint4(b[4], b[5], b[6], b[7]);
+        for (int q = 0; q < kTy / 4; ++q) tieB[tid][q] = make_uint4(b[4 * q], b[4 * q + 1], b[4 * q + 2], b[4 * q + 3]);
     }
     // tail candidates: tie bits and staged-copy offsets (stage 0, stage 1), per thread
     __shared__ uint32_t tinfo[G::kTailPer][1 + G::kPhaseSets][G::kThreads];
@@ -466,7 +474,8 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         // 4-warp CTAs: warp w holds dy in [-R + 16 w, -R + 16 w + 15]); its tails still run
         bool main_dead = false;
         if (SP_ME_SKIP && nwarps > 1 && !interior && !A.surface) {
-            const int blo = -R + 2 * kTy * warp, bhi = blo + 2 * kTy - 1;
+            constexpr int kDyWarp = (32 / (4 * G::kGx)) * kTy;  // dy values of a warp's main candidates
+            const int blo = -R + kDyWarp * warp, bhi = blo + kDyWarp - 1;
             main_dead = bhi < dylo || blo > dyhi;
         }
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
@@ -601,8 +610,15 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         {
             const uint4 a4 = tieA[p + 4 * g];
             const uint32_t Aj[4] = {a4.x, a4.y, a4.z, a4.w};
-            const uint4 b0 = tieB[d][0], b1 = tieB[d][1];
-            const uint32_t Bi[8] = {b0.x, b0.y, b0.z, b0.w, b1.x, b1.y, b1.z, b1.w};
+            uint32_t Bi[kTy];
+#pragma unroll
+            for (int q = 0; q < kTy / 4; ++q) {
+                const uint4 bq = tieB[d][q];
+                Bi[4 * q] = bq.x;
+                Bi[4 * q + 1] = bq.y;
+                Bi[4 * q + 2] = bq.z;
+                Bi[4 * q + 3] = bq.w;
+            }
 #pragma unroll
             for (int i = 0; i < kTy; ++i) {
                 uint32_t ki = 0xffffffffu;
