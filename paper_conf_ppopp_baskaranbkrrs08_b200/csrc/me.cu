@@ -53,8 +53,11 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 #ifndef SP_ME_SKIP
 #define SP_ME_SKIP 1
 #endif
+// SP_ME_R16_TY: dy candidates per thread at R = 16.  8 (one warp of 4 x 8 tiles) is the
+// default; 4 (two warps of 4 x 4 tiles, 64 registers, 20 warps per SM) measured slower on CIF
+// +-16 at throughput: 70.2 vs 72.6 % of the VABSDIFF4 roof (r3d).
 #ifndef SP_ME_R16_TY
-#define SP_ME_R16_TY 4
+#define SP_ME_R16_TY 8
 #endif
 constexpr int sp_me_kTy = 8;
 #ifndef SP_ME_SCRAMBLE
@@ -165,7 +168,7 @@ template <int R>
 struct MeGeom {
     static constexpr int kWin = 2 * R + 16;              // window edge (bytes per row, rows)
     static constexpr int kCopy = kWin * kWin;            // bytes per staged copy (multiple of 128)
-    // R = 16: 4 x 4 tiles over two warps (SP_ME_R16_TY 4; 8 = one warp of 4 x 8 tiles)
+    // R = 16: SP_ME_R16_TY dy per thread (8: one warp of 4 x 8 tiles; 4: two warps of 4 x 4)
     static constexpr int kTy = R == 16 ? SP_ME_R16_TY : ::sp_me_kTy;
     static constexpr int kThreads = R * R / kTy;         // one 4 x kTy candidate tile per thread
     static constexpr int kWarps = kThreads / 32;         // 4 (R = 32) or 1 (R = 16)
