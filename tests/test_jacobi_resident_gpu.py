@@ -61,3 +61,17 @@ def test_J1_and_long_run_at_capacity():
     _check(got[idx], oracle.jacobi1d_points(a, 4096, idx))
     with pytest.raises(sp.SPError):
         sp.jacobi1d_resident(torch.zeros(n + 1, device="cuda"), 4)
+
+
+def test_prepared_call_J1():
+    """jacobi1d_resident_prepared (the latency-config call form, arguments marshalled once):
+    J1 out of place, called twice on the same buffers, equals the oracle."""
+    a0 = sp_inputs.jacobi_input(4096, seed=2008)
+    want = oracle.jacobi1d(a0, 64)
+    src = torch.from_numpy(a0).cuda()
+    dst = torch.empty_like(src)
+    call = sp.jacobi1d_resident_prepared(src, 64, out=dst)
+    call()
+    call()
+    torch.cuda.synchronize()
+    _check(dst, want)

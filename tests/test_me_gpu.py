@@ -175,3 +175,18 @@ def test_border_macroblocks_without_surface(W, H, R, gen):
         omv, osad, _ = _oracle_pair(fr, p, W, H, R, surface=False)
         assert np.array_equal(mv[p].reshape(-1, 2), omv), p
         assert np.array_equal(sad[p].reshape(-1), osad), p
+
+
+def test_prepared_call_equals_oracle():
+    """me_search_prepared (arguments marshalled once, the latency-config call form) runs the
+    same entry point: repeated calls give the oracle's MVs / SADs."""
+    W, H, R = 352, 288, 16
+    fr = sp_inputs.me_sequence(3, W, H, R, seed=41)
+    call = sp.me_search_prepared(torch.from_numpy(fr).cuda(), W, H, R)
+    for _ in range(3):
+        call()
+    torch.cuda.synchronize()
+    for p in range(2):
+        omv, osad, _ = _oracle_pair(fr, p, W, H, R, surface=False)
+        assert np.array_equal(call.mv[p].cpu().numpy().reshape(-1, 2), omv)
+        assert np.array_equal(call.sad[p].cpu().numpy().view(np.uint32).reshape(-1), osad)
