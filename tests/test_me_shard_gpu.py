@@ -88,7 +88,9 @@ def _shard_worker(rank, world, port, W, H, R, pairs, out_dir, calls):
     import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
     import sp_inputs
 
-    torch.cuda.set_device(0)
+    # one GPU per rank when the box has several (NVLink peer memory between devices), else
+    # every rank shares GPU 0 (CUDA IPC between processes on one device: the same code path)
+    torch.cuda.set_device(rank % torch.cuda.device_count())
     dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank, world_size=world)
     pitch = (W + 15) // 16 * 16
     shard = sp.MEShard(pairs, W, H, R, pitch=pitch)

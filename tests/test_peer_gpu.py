@@ -35,7 +35,9 @@ def _worker(rank, world, port, n, steps_list, tt, out_dir, fused=False, space_ti
     import sp_inputs
     from paper_conf_ppopp_baskaranbkrrs08_b200.partition import jacobi_slabs
 
-    torch.cuda.set_device(0)
+    # one GPU per rank when the box has several (NVLink peer memory between devices), else
+    # every rank shares GPU 0 (CUDA IPC between processes on one device: the same code path)
+    torch.cuda.set_device(rank % torch.cuda.device_count())
     dist.init_process_group("gloo", init_method=f"tcp://127.0.0.1:{port}", rank=rank, world_size=world)
     H = sp.halo_of(tt)
     xb, nl = jacobi_slabs(n, world, H)[rank]
