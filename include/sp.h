@@ -185,8 +185,9 @@ typedef struct {
     int32_t smem_bytes;  /* dynamic shared memory per CTA */
     int32_t cells_per_thread; /* register cells per thread */
     /* the persistent launch over DEVICE memory (sp_jacobi1d_timetiled_fused, _stream with
-     * device in / out) uses the in-place geometry: 80 register cells per thread in 41 packed
-     * registers, alternating sweeps; with space_tile = 0 its tile is larger: */
+     * device in / out) uses the in-place geometry when time_tile >= 16 (80 register cells per
+     * thread in 41 packed registers, alternating sweeps; below 16 the pass is HBM-bound and the
+     * staged geometry is kept); with space_tile = 0 its tile is larger: */
     int64_t persistent_space_tile; /* S of that launch (space_tile if given) */
     int64_t persistent_tiles;      /* its tiles per pass (<= tiles: flags sized by `tiles` suffice) */
 } sp_jacobi_plan;

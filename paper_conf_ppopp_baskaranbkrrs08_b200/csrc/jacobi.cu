@@ -1105,14 +1105,18 @@ int variant_index() {
 // keeps the staged TMA move-out of the default geometry: the in-place kernel's direct
 // 16-byte register stores would cross PCIe as small writes.  SP_JACOBI_VARIANT_FUSED (or
 // SP_JACOBI_VARIANT) overrides.
-int persistent_variant_index() {
+// Below a time tile of 16 the pass is HBM-bound and the in-place kernel's scattered 16-byte
+// stores cost more than its shorter halo saves (J3 persistent: Tt = 4 / 8: 34.6 / 17.3 ms in
+// place vs 27.4 / 15.8 staged; Tt = 16: 9.98 vs 10.2), so short time tiles stay staged.
+int persistent_variant_index(int32_t time_tile) {
     static int idx = [] {
         const char* e = std::getenv("SP_JACOBI_VARIANT_FUSED");
         if (!e) e = std::getenv("SP_JACOBI_VARIANT");
         int i = e ? std::atoi(e) : kPersistentVariant;
         return (i >= 0 && i < kNumVariants) ? i : kPersistentVariant;
     }();
-    return idx;
+    static const bool forced = std::getenv("SP_JACOBI_VARIANT_FUSED") || std::getenv("SP_JACOBI_VARIANT");
+    return (time_tile < 16 && !forced) ? variant_index() : idx;
 }
 
 int smem_bytes(const Variant& v) { return v.stage_floats * (int)sizeof(float); }
@@ -1272,7 +1276,7 @@ extern "C" int sp_jacobi1d_plan(int64_t n, int32_t steps, int32_t time_tile, int
     {
         int64_t Sp;
         int32_t wp;
-        if (geometry(time_tile, space_tile, Sp, wp, persistent_variant_index()) == SP_OK) {
+        if (geometry(time_tile, space_tile, Sp, wp, persistent_variant_index(time_tile)) == SP_OK) {
             out->persistent_space_tile = Sp;
             out->persistent_tiles = (n + Sp - 1) / Sp;
         } else {  // (an explicit space tile above the in-place maximum cannot happen: it is larger)
@@ -1411,7 +1415,7 @@ extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* 
     if ((st = device_view(in, (const void**)&din, &hin)) || (st = device_view(out, (const void**)&dout, &hout)))
         return st;
     // device memory on both ends: the in-place geometry; host-mapped: the staged one
-    const int vi = (hin || hout) ? variant_index() : persistent_variant_index();
+    const int vi = (hin || hout) ? variant_index() : persistent_variant_index(time_tile);
     int64_t S;
     int32_t wo;
     if ((st = geometry(time_tile, space_tile, S, wo, vi))) return st;
@@ -1555,7 +1559,7 @@ extern "C" int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* L, float* a
         return SP_ERR_INVALID_ARG;
     int64_t S;
     int32_t wo;
-    const int vi = persistent_variant_index();  // (the in-place geometry, as the single-GPU persistent launch)
+    const int vi = persistent_variant_index(time_tile);  // (as the single-GPU persistent launch)
     int st = geometry(time_tile, space_tile, S, wo, vi);
     if (st) return st;
     const int32_t H = halo_of(time_tile);
