@@ -1063,9 +1063,9 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 15;
+constexpr int kNumVariants = 17;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
-constexpr int kPersistentVariant = 14;  // in place, K = 40 (profiles/r02_jacobi_inplace.txt)
+constexpr int kPersistentVariant = 16;  // in place, K = 40, one 16-warp CTA per SM (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
 Variant* variants() {
@@ -1084,7 +1084,9 @@ Variant* variants() {
         make_variant<JCfg<44, 8, 2, false, true>>(),  // 11: in place, 88 cells/lane, 16 warps/SM, one stage (176 KB)
         make_variant<JCfg<36, 8, 2, false, true>>(),  // 12: in place, 72 cells/lane, 16 warps/SM (144 KB)
         make_variant<JCfg<52, 8, 2, false, true>>(),  // 13: in place, 104 cells/lane, 16 warps/SM (208 KB)
-        make_variant_peer<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
+        make_variant<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
+        make_variant<JCfg<40, 4, 4, false, true>>(),  // 15: as 14 in 4-warp CTAs
+        make_variant_peer<JCfg<40, 16, 1, false, true>>(),  // 16: as 14 in one 16-warp CTA per SM (persistent default)
     };  // (in place at 20 / 24 warps per SM, <= 102 / 85 registers, spilled into the loop:
         //  7.45-8.9 ms on J3, profiles/r02_jacobi_inplace.txt r2x)
     return v;
@@ -1101,7 +1103,8 @@ int variant_index() {
 // The persistent launch over device memory (the bench's N = 1 path) takes the in-place
 // geometry: K = 40 in K + 1 registers (5.3 % redundant halo updates at Tt = 64 instead of
 // 7.7 %), 6.59-6.64 vs 6.87 ms on J3 (A/B, r2o; K = 44: 6.74 — its loop keeps 16 register
-// moves per 4 steps on the FMA pipe at the 128-register limit, K = 40's keeps 3).  Host-mapped move-in / move-out (sp_jacobi1d_host)
+// moves per 4 steps on the FMA pipe at the 128-register limit, K = 40's keeps 3).  One 16-warp
+// CTA per SM rather than two 8-warp CTAs: 6.549 vs 6.579 ms (r3h; 4-warp CTAs: 6.72).  Host-mapped move-in / move-out (sp_jacobi1d_host)
 // keeps the staged TMA move-out of the default geometry: the in-place kernel's direct
 // 16-byte register stores would cross PCIe as small writes.  SP_JACOBI_VARIANT_FUSED (or
 // SP_JACOBI_VARIANT) overrides.

@@ -1,0 +1,5 @@
+set -x
+O=gpurun_out/r3h.txt
+for rep in 1 2; do
+for v in 14 15 16; do echo "== variant $v" >> $O; SP_JACOBI_VARIANT_FUSED=$v timeout 300 python tools/quick_time.py 64 --fused --no-me >> $O 2>&1; done
+done
