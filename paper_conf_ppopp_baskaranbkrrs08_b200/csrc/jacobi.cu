@@ -1063,7 +1063,7 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 19;
+constexpr int kNumVariants = 20;
 constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
 constexpr int kPersistentVariant = 16;  // in place, K = 40, one 16-warp CTA per SM (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
@@ -1089,6 +1089,7 @@ Variant* variants() {
         make_variant_peer<JCfg<40, 16, 1, false, true>>(),  // 16: as 14 in one 16-warp CTA per SM (persistent default)
         make_variant<JCfg<44, 16, 1, false, true>>(),  // 17: in place K = 44, one 16-warp CTA per SM
         make_variant<JCfg<36, 16, 1, false, true>>(),  // 18: in place K = 36, one 16-warp CTA per SM
+        make_variant_peer<JCfg<28, 16, 1>>(),  // 19: as 5 (staged) in one 16-warp CTA per SM (224 KB)
     };  // (in place at 20 / 24 warps per SM, <= 102 / 85 registers, spilled into the loop:
         //  7.45-8.9 ms on J3, profiles/r02_jacobi_inplace.txt r2x)
     return v;
