@@ -1064,7 +1064,10 @@ Variant make_variant_peer() {
 }
 
 constexpr int kNumVariants = 20;
-constexpr int kDefaultVariant = 5;  // K = 28, 8 warps, 2 CTAs/SM (sweep: profiles/r01_jacobi_variant_sweep.txt)
+// K = 28 staged, one 16-warp CTA per SM: the host-buffer path 8.23 vs 8.79 ms and the per-pass
+// HBM-bound regime (Tt = 8) 12.82 vs 13.45 ms against the same geometry as two 8-warp CTAs
+// (variant 5, the round-1 default; profiles/r02_jacobi_inplace.txt r3k)
+constexpr int kDefaultVariant = 19;
 constexpr int kPersistentVariant = 16;  // in place, K = 40, one 16-warp CTA per SM (profiles/r02_jacobi_inplace.txt)
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
