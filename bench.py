@@ -67,6 +67,17 @@ def workload(world, tt):
     return {"name": "J5+M4", "jac_n": JAC5_N, "jac_t": JAC5_T}
 
 
+def _geometry(n_local, T, tt, persistent):
+    """The Jacobi pass kernel's geometry as the library plans it (include/sp.h sp_jacobi_plan):
+    the persistent launches take the in-place one at Tt >= 16, the staged one otherwise."""
+    import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
+    pl = sp.jacobi1d_plan(n_local, T, tt, 0)
+    if persistent and tt >= 16:
+        k = (pl["persistent_space_tile"] + 2 * pl["halo"]) // 64  # strip = 64 K cells per warp
+        return f"in place: {2 * k} cells/lane in {k + 1} packed registers, one stage per warp"
+    return f"staged: {pl['cells_per_thread']} cells/lane, two stages per warp"
+
+
 def bench_config(world, tt, halo="peer", gather="peer"):
     h = (tt + 3) & ~3
     if world == 1:
@@ -545,10 +556,11 @@ def run_ours(args, rank, world, local_rank):
         "config": bench_config(world, tt, args.halo, args.gather),
         "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4),
                    "n_local": n_local, "passes_per_step": -(-T // tt),
-                   "space_tile": (sp.jacobi1d_plan(n_local, T, tt, 0)["persistent_space_tile"] if world == 1
-                                  else sp.jacobi1d_plan(n_local, T, tt, 0)["space_tile"]),
-                   "geometry": ("in place: 80 cells/lane in 41 packed registers, one stage per warp" if world == 1
-                                else "staged: 56 cells/lane, two stages per warp (peer instantiation)")},
+                   # the persistent launches (single GPU and peer-fused) take the in-place
+                   # geometry at Tt >= 16, the staged one below (include/sp.h sp_jacobi_plan)
+                   "space_tile": sp.jacobi1d_plan(n_local, T, tt, 0)["persistent_space_tile" if persistent
+                                                                      else "space_tile"],
+                   "geometry": _geometry(n_local, T, tt, persistent)},
         "me": {"value": round(me_val, 2), "unit": "GSAD/s", "abs_diff_per_s": me_val * 256e9,
                "ms_per_step": round(me_ms / K, 4), "roofline": roof_me, "e2e": me_e2e},
         "roofline": dominant, "roofline_jacobi": roof_jac, "roofline_jacobi_hbm_regime": roof_hbm,
@@ -588,7 +600,10 @@ def main(argv=None):
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--warmup", type=int, default=3)
     ap.add_argument("--impl", choices=["ours", "reference"], default="ours")
-    ap.add_argument("--time-tile", type=int, default=64)
+    # Tt = 128: fastest on J3 with the persistent in-place geometry (K = 56: 6.41 ms vs 6.50 at
+    # Tt = 64; profiles/r02_jacobi_inplace.txt r3p) — the time tile is the paper's own tuning
+    # parameter (§4.3 tile-size search), not part of the J3 / J5 problem definitions
+    ap.add_argument("--time-tile", type=int, default=128)
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--halo", choices=["peer", "nccl"], default="peer",
                     help="multi-GPU Jacobi halo exchange: fused peer stores in the pass kernel, or NCCL send/recv")

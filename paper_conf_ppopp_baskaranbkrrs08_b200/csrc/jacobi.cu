@@ -1063,12 +1063,17 @@ Variant make_variant_peer() {
     return v;
 }
 
-constexpr int kNumVariants = 20;
+constexpr int kNumVariants = 27;
 // K = 28 staged, one 16-warp CTA per SM: the host-buffer path 8.23 vs 8.79 ms and the per-pass
 // HBM-bound regime (Tt = 8) 12.82 vs 13.45 ms against the same geometry as two 8-warp CTAs
 // (variant 5, the round-1 default; profiles/r02_jacobi_inplace.txt r3k)
 constexpr int kDefaultVariant = 19;
-constexpr int kPersistentVariant = 16;  // in place, K = 40, one 16-warp CTA per SM (profiles/r02_jacobi_inplace.txt)
+// in place, K = 56 (112 cells per lane), one 12-warp CTA per SM: J3 6.50 ms at Tt = 64 and
+// 6.41 ms at Tt = 128, against 6.55 / 6.67 ms for K = 40 in one 16-warp CTA (variant 16) — the
+// longer strip cuts the redundant halo (2H / S: 3.7 % vs 5.3 % at H = 64) and the per-tile
+// overhead per update, and 3 warps per SM sub-partition still keep the FMA pipe fed
+// (profiles/r02_jacobi_inplace.txt r3o / r3p: K = 48 / 52 / 60 / 64 at 12 warps, 60 / 68 at 10)
+constexpr int kPersistentVariant = 20;
 constexpr int64_t kDefaultSkew = 512;  // wavefront order: tiles between consecutive passes (host path sweeps on J3: 256 -> 9.6 ms, 512 -> 8.65, 1024 -> 8.89, 2048 -> 10.3)
 
 Variant* variants() {
@@ -1089,10 +1094,17 @@ Variant* variants() {
         make_variant<JCfg<52, 8, 2, false, true>>(),  // 13: in place, 104 cells/lane, 16 warps/SM (208 KB)
         make_variant<JCfg<40, 8, 2, false, true>>(),  // 14: in place, 80 cells/lane (2-way conflicts on the tile load only)
         make_variant<JCfg<40, 4, 4, false, true>>(),  // 15: as 14 in 4-warp CTAs
-        make_variant_peer<JCfg<40, 16, 1, false, true>>(),  // 16: as 14 in one 16-warp CTA per SM (persistent default)
+        make_variant_peer<JCfg<40, 16, 1, false, true>>(),  // 16: as 14 in one 16-warp CTA per SM (round-2 persistent default until r3o)
         make_variant<JCfg<44, 16, 1, false, true>>(),  // 17: in place K = 44, one 16-warp CTA per SM
         make_variant<JCfg<36, 16, 1, false, true>>(),  // 18: in place K = 36, one 16-warp CTA per SM
         make_variant_peer<JCfg<28, 16, 1>>(),  // 19: as 5 (staged) in one 16-warp CTA per SM (224 KB)
+        make_variant_peer<JCfg<56, 12, 1, false, true>>(),  // 20: in place K = 56, one 12-warp CTA per SM (<= 168 regs; persistent default)
+        make_variant<JCfg<48, 12, 1, false, true>>(),  // 21: in place K = 48, one 12-warp CTA per SM
+        make_variant<JCfg<64, 12, 1, false, true>>(),  // 22: in place K = 64, one 12-warp CTA per SM
+        make_variant<JCfg<52, 12, 1, false, true>>(),  // 23: in place K = 52, one 12-warp CTA per SM
+        make_variant<JCfg<60, 12, 1, false, true>>(),  // 24: in place K = 60, one 12-warp CTA per SM
+        make_variant<JCfg<68, 10, 1, false, true>>(),  // 25: in place K = 68, one 10-warp CTA per SM (<= 204 regs)
+        make_variant<JCfg<60, 10, 1, false, true>>(),  // 26: in place K = 60, one 10-warp CTA per SM
     };  // (in place at 20 / 24 warps per SM, <= 102 / 85 registers, spilled into the loop:
         //  7.45-8.9 ms on J3, profiles/r02_jacobi_inplace.txt r2x)
     return v;

@@ -1,0 +1,6 @@
+O=gpurun_out/r3o.txt
+for rep in 1 2; do
+for v in 16 20 21 22; do
+echo "== variant $v" >> $O; SP_JACOBI_VARIANT_FUSED=$v timeout 300 python tools/quick_time.py 64,128 --fused --no-me >> $O 2>&1
+done
+done
