@@ -11,7 +11,8 @@ import sp_inputs  # noqa: E402
 
 
 def main():
-    n, T, tt = 1 << 30, 4096, 64
+    n, T = 1 << 30, 4096
+    tt = int(sys.argv[1]) if len(sys.argv) > 1 else 128
     a = torch.from_numpy(sp_inputs.jacobi_input(n, seed=2008)).cuda()
     w = torch.empty_like(a)
     flags = torch.empty(sp.jacobi1d_plan(n, T, tt, 0)["tiles"] + 1, dtype=torch.int32, device="cuda")
