@@ -492,9 +492,7 @@ def run_ours(args, rank, world, local_rank):
         f_pin = torch.from_numpy(frames_host).pin_memory()
         # host-buffer Jacobi: the kernel reads a_pin and writes the result back over PCIe itself
         # (sp_jacobi1d_host, wavefront order), in place: every call advances the state T steps
-        # (its own time tile: the host-buffer path runs the staged geometry — 16-byte register
-        # stores to mapped host memory cost the in-place one 3x — whose 1,792-cell strips favour
-        # Tt = 64: 8.29e12 vs 8.06e12 point-updates/s at Tt = 128, profiles/r02_bench_repeat.jsonl)
+        # (same time tile as the device-resident run unless --e2e-time-tile says otherwise)
         tt_e2e = args.e2e_time_tile or tt
         jac_host = sp.Jacobi1DHost(n_local, T, tt_e2e)
         # host-buffer ME: frames streamed frame by frame while the search runs, MV / SAD stored
@@ -608,7 +606,7 @@ def main(argv=None):
     # Tt = 64; profiles/r02_jacobi_inplace.txt r3p) — the time tile is the paper's own tuning
     # parameter (§4.3 tile-size search), not part of the J3 / J5 problem definitions
     ap.add_argument("--time-tile", type=int, default=128)
-    ap.add_argument("--e2e-time-tile", type=int, default=64, help="time tile of the N = 1 host-buffer e2e call")
+    ap.add_argument("--e2e-time-tile", type=int, default=0, help="time tile of the N = 1 host-buffer e2e call (0: --time-tile)")
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--halo", choices=["peer", "nccl"], default="peer",
                     help="multi-GPU Jacobi halo exchange: fused peer stores in the pass kernel, or NCCL send/recv")

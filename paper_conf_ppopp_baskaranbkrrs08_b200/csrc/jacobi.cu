@@ -577,8 +577,17 @@ __device__ __forceinline__ void run_steps_se(uint64_t (&P)[kK], int h, int lane,
 // kPeer: the instantiation with the persistent multi-GPU halo exchange (PassArgs::pushL);
 // the single-GPU launches use the one without it (its code would cost the common path
 // registers: 6.89 -> 6.96 ms on J3 when compiled in).
-template <class Cfg, bool kPeer = false>
+// kMode: kPlainPass; kPeerPass (multi-GPU halo pushes, PassArgs above); kHostOutPass (in-place
+// geometry, persistent mode, outL is page-locked HOST memory: the last pass's owned cells leave
+// through the warp's stage and one TMA bulk store per tile — large PCIe writes — instead of
+// 16-byte register stores — scattered 16-byte PCIe writes, 3x the J3 host-path time — and that
+// tile's successor is prefetched only after the store has read the stage).  Separate
+// instantiations keep the device-resident kernel's code unchanged (the host-out branch inside
+// it cost J3 1-2 %, measured).
+enum { kPlainPass = 0, kPeerPass = 1, kHostOutPass = 2 };
+template <class Cfg, int kMode = kPlainPass>
 __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_kernel(PassArgs A) {
+    constexpr bool kPeer = kMode == kPeerPass;
     constexpr int kK = Cfg::K, kStrip = Cfg::kStrip;
     extern __shared__ __align__(128) float smem[];
     __shared__ __align__(8) uint64_t full[Cfg::kWarps][2];
@@ -802,6 +811,8 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         const int h = h_of(pass);
         tile_range(t, x0, st, lo, hi);
         const int64_t base = x0 - A.H;  // buf[j] <-> global base + j
+        // (in place) this tile's owned cells go to host memory: staged move-out (PassArgs::out_host)
+        const bool stage_out = kIP && kMode == kHostOutPass && pass == A.passes - 1;
         if (pers && pending) {  // publish first: never wait while holding a finished tile
             if (lane == 0) publish(true);
             __syncwarp();
@@ -870,9 +881,10 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
                           : !deps_ready(tn, pn);
             if constexpr (kIP) {
                 // one stage: the next tile streams into the buffer this tile was just loaded
-                // from, once every lane's reads of it are done (warp barrier, then the proxy fence)
+                // from, once every lane's reads of it are done (warp barrier, then the proxy
+                // fence) — unless this tile's move-out needs the stage (host output, below)
                 __syncwarp();
-                if (lane == 0 && !pending) {
+                if (lane == 0 && !pending && !stage_out) {
                     fence_proxy_async_smem();
                     issue(tn, pn, 0);
                 }
@@ -942,7 +954,43 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         // a hash of (tile, pass), finishes 20 us late, so dependent tiles really wait
         if ((((uint32_t)t * 2654435761u) ^ (uint32_t)(pass * 40503u)) % 8u == 0u) __nanosleep(20000);
 #endif
-        if constexpr (kIP) {
+        if (kIP && kMode == kHostOutPass && stage_out) {
+            // ---- host output: owned cells -> the (idle) stage -> one TMA bulk store ----
+            const int own_hi = A.H + (int)st;
+            float4* qu = reinterpret_cast<float4*>(buf + lane * kK);
+            float4* qv = reinterpret_cast<float4*>(buf + 32 * kK + lane * kK);
+            constexpr int O2 = kIP ? 1 : 0;
+#pragma unroll
+            for (int q = 0; q < kK / 4; ++q) {
+                const int ou = lane * kK + 4 * q, ov = 32 * kK + lane * kK + 4 * q;
+                if (ou >= A.H && ou < own_hi)
+                    qu[q] = make_float4(f2_lo(P[4 * q + O2]), f2_lo(P[4 * q + 1 + O2]), f2_lo(P[4 * q + 2 + O2]),
+                                        f2_lo(P[4 * q + 3 + O2]));
+                if (ov >= A.H && ov < own_hi)
+                    qv[q] = make_float4(f2_hi(P[4 * q + O2]), f2_hi(P[4 * q + 1 + O2]), f2_hi(P[4 * q + 2 + O2]),
+                                        f2_hi(P[4 * q + 3 + O2]));
+            }
+            fence_proxy_async_smem();
+            __syncwarp();
+            const int64_t n16 = st & ~int64_t(3);
+            if (lane == 0 && n16 > 0) {
+                tma_store_1d(dst + (x0 - A.g0), buf + A.H, (uint32_t)(n16 * 4));
+                bulk_commit();
+            }
+            if (lane < st - n16) dst[x0 - A.g0 + n16 + lane] = buf[A.H + n16 + lane];
+            __syncwarp();  // (the ragged cells are read from the stage before it is refilled)
+            // the successor's move-in, deferred above, once the store has read the stage.  (A
+            // last-pass tile has no dependents: its flag is published without waiting for the
+            // store to complete; the kernel's final bulk wait covers the data.)
+            if (lane == 0) {
+                bulk_wait_read0();  // (also before a pending successor's move-in, next iteration)
+                if (u_next < total && !pending) {
+                    fence_proxy_async_smem();
+                    issue(tn, pn, 0);
+                }
+            }
+            __syncwarp();
+        } else if constexpr (kIP) {
             // ---- owned cells: registers -> global (16-byte stores; the stage is busy with
             //      the next tile's move-in) ----
             const int own_hi = A.H + (int)st;  // strip offsets [H, H + st) are owned
@@ -1040,8 +1088,9 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
 struct Variant {
     int K, warps, threads, strip, stage_floats;
     void (*kernel)(PassArgs);
-    void (*kernel_peer)(PassArgs) = nullptr;  // kPeer instantiation (default and persistent variants)
-    int sms = 0, occ = 0, occ_peer = 0;
+    void (*kernel_peer)(PassArgs) = nullptr;  // kPeerPass instantiation (default and persistent variants)
+    void (*kernel_host)(PassArgs) = nullptr;  // kHostOutPass instantiation (in-place persistent variants)
+    int sms = 0, occ = 0, occ_peer = 0, occ_host = 0;
     bool ok = false;
 };
 
@@ -1059,7 +1108,8 @@ Variant make_variant() {
 template <class Cfg>
 Variant make_variant_peer() {
     Variant v = make_variant<Cfg>();
-    v.kernel_peer = jacobi1d_pass_kernel<Cfg, true>;
+    v.kernel_peer = jacobi1d_pass_kernel<Cfg, kPeerPass>;
+    if constexpr (Cfg::kInPlace) v.kernel_host = jacobi1d_pass_kernel<Cfg, kHostOutPass>;
     return v;
 }
 
@@ -1163,6 +1213,12 @@ int device_info(Variant& out, int vi = -1) {
                                                                       smem_bytes(d)));
             if (d.occ_peer < 1) d.occ_peer = 1;
         }
+        if (d.kernel_host) {
+            SP_CUDA_TRY(cudaFuncSetAttribute(d.kernel_host, cudaFuncAttributeMaxDynamicSharedMemorySize, smem_bytes(d)));
+            SP_CUDA_TRY(cudaOccupancyMaxActiveBlocksPerMultiprocessor(&d.occ_host, d.kernel_host, d.threads,
+                                                                      smem_bytes(d)));
+            if (d.occ_host < 1) d.occ_host = 1;
+        }
         d.ok = true;
     }
     out = d;
@@ -1188,8 +1244,10 @@ int geometry(int32_t time_tile, int32_t space_tile, int64_t& S, int32_t& wo, int
     return SP_OK;
 }
 
-int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v, bool peer = false) {
-    if (peer && !v.kernel_peer) return SP_ERR_UNSUPPORTED;  // (SP_JACOBI_VARIANT other than the default)
+int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v, int mode = kPlainPass) {
+    const bool peer = mode == kPeerPass, host = mode == kHostOutPass;
+    if ((peer && !v.kernel_peer) || (host && !v.kernel_host))
+        return SP_ERR_UNSUPPORTED;  // (SP_JACOBI_VARIANT other than the defaults)
     if (a.tiles <= 0) return SP_OK;
     // SP_JACOBI_GRID_CAP (sanitizer runs): a few CTAs then take many tiles per warp, so
     // racecheck sees both stages of every warp's double buffer in use
@@ -1197,10 +1255,10 @@ int launch_pass(const PassArgs& a, cudaStream_t stream, const Variant& v, bool p
         const char* e = std::getenv("SP_JACOBI_GRID_CAP");
         return e ? (int64_t)std::atoll(e) : (int64_t)0;
     }();
-    int64_t cap = (int64_t)v.sms * (peer ? v.occ_peer : v.occ);
+    int64_t cap = (int64_t)v.sms * (peer ? v.occ_peer : host ? v.occ_host : v.occ);
     if (env_cap > 0 && env_cap < cap) cap = env_cap;
     const int grid = (int)(a.tiles < cap ? a.tiles : cap);
-    (peer ? v.kernel_peer : v.kernel)<<<grid, v.threads, smem_bytes(v), stream>>>(a);
+    (peer ? v.kernel_peer : host ? v.kernel_host : v.kernel)<<<grid, v.threads, smem_bytes(v), stream>>>(a);
     SP_CUDA_TRY(cudaGetLastError());
     return SP_OK;
 }
@@ -1436,7 +1494,8 @@ extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* 
     if ((st = device_view(in, (const void**)&din, &hin)) || (st = device_view(out, (const void**)&dout, &hout)))
         return st;
     // device memory on both ends: the in-place geometry; host-mapped: the staged one
-    const int vi = (hin || hout) ? variant_index() : persistent_variant_index(time_tile);
+    // (host buffers: the in-place kernel stages its last pass's move-out, PassArgs::out_host)
+    const int vi = persistent_variant_index(time_tile);
     int64_t S;
     int32_t wo;
     if ((st = geometry(time_tile, space_tile, S, wo, vi))) return st;
@@ -1473,7 +1532,8 @@ extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* 
     PassArgs p{nullptr, nullptr, n, 0, n, 0, n, S, tiles, time_tile, H, wo, footprint_log, kNegZero2,
                nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, 0ull, nullptr, nullptr,
                flags, {buf0, buf1}, passes, steps, time_tile, din, redirect ? nullptr : const_cast<float*>(dout), skew};
-    if ((st = launch_pass(p, s, di))) return st;
+    // host output written by the in-place kernel: its staged-move-out instantiation
+    if ((st = launch_pass(p, s, di, hout && !redirect && di.kernel_host ? kHostOutPass : kPlainPass))) return st;
     if (redirect)
         SP_CUDA_TRY(cudaMemcpyAsync(out, bufs[passes & 1], (size_t)n * sizeof(float), cudaMemcpyDefault, s));
     return SP_OK;
@@ -1621,7 +1681,7 @@ extern "C" int sp_jacobi1d_timetiled_peer_fused(const sp_peer_links* L, float* a
                 has_left ? L->left_bufs[1] + L->left_n_local + H : nullptr},
                {has_right ? L->right_bufs[0] : nullptr, has_right ? L->right_bufs[1] : nullptr},
                flags + tiles + 1, has_left ? nL : 0, has_right ? nR : 0};
-    if ((st = launch_pass(p, s, di, true))) return st;
+    if ((st = launch_pass(p, s, di, kPeerPass))) return st;
     if (passes & 1)
         SP_CUDA_TRY(cudaMemcpyAsync(a_local + H, work_local + H, (size_t)n_local * sizeof(float),
                                     cudaMemcpyDeviceToDevice, s));

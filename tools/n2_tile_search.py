@@ -12,7 +12,9 @@ Constants, in SM clock cycles:
                                  bytes per clock per SM with the kernels' copies in flight
                                  (HBM-bound when every SM streams)
 Measured optima (N1, profiles/r01_jacobi_variant_sweep.txt, r01_n1_ablation.jsonl):
-  Jacobi J3: time tile 64, space tile 1664 owned (+ 2 x 64 halo = 1792 staged per warp strip)
+  Jacobi J3: time tile 128, space tile 3328 owned (+ 2 x 128 halo = 3584 cells per warp strip,
+             the in-place K = 56 geometry, profiles/r02_jacobi_inplace.txt r3p); the staged
+             K = 28 geometry's optimum was time tile 64, space tile 1664 (1792-cell strips)
   ME M4: one macroblock's whole 65 x 65 candidate set x 16 x 16 pixels per CTA iteration.
 """
 import json
@@ -53,21 +55,23 @@ def main():
     cal = json.load(open(path))
     out = []
     # ---- Jacobi: the (t, i') band of J3, P = 32 lanes of a warp (the outer process is a warp),
-    # M_up = one warp strip (K = 28: 1792 fp32 cells held in registers / one staged copy)
+    # M_up = one warp strip (K = 28: 1792 fp32 cells; in place K = 56: 3584)
     P = 32
     S, L, B = constants(cal, P, 4, 7168)
     cand_t = [8, 16, 32, 48, 64, 96, 128]
     cand_s = [256, 512, 1024, 1664, 2048, 4096]
-    for mup in (1792, 4096):
+    for mup in (1792, 3584, 4096):
         r = sp.tile_search([1024, 1 << 26], JAC_REFS, [cand_t, cand_s], mup_elems=mup, procs=P, sync_cost=S,
                            elem_cost=L)
         out.append({"exp": "b200_jacobi", "P": P, "S_cycles": round(S, 4), "L_cycles": round(L, 4),
                     "tma_bytes_per_clk_sm": B, "mup_words": mup, "model_tile_time_space": r["tile"],
                     "model_cost_cycles": r["cost"], "local_elems": r["local_elems"],
-                    "measured_optimum_time_space": [64, 1664],
-                    "measured_source": "profiles/r01_jacobi_variant_sweep.txt (K = 28: Tt 32..80)"})
+                    "measured_optimum_time_space": [128, 3328] if mup >= 3584 else [64, 1664],
+                    "measured_source": ("profiles/r02_jacobi_inplace.txt r3p (in place K = 56: Tt 64 / 96 / 128)"
+                                        if mup >= 3584 else
+                                        "profiles/r01_jacobi_variant_sweep.txt (staged K = 28: Tt 32..80)")})
     # model cost of the measured optimum and of its neighbours (same objective, fixed tiles)
-    for tt, ss in [(64, 1664), (32, 1664), (128, 1664), (64, 1024)]:
+    for tt, ss in [(64, 1664), (32, 1664), (128, 1664), (64, 1024), (128, 3328), (64, 3456)]:
         r = sp.tile_search([1024, 1 << 26], JAC_REFS, [[tt], [ss]], mup_elems=0, procs=P, sync_cost=S, elem_cost=L)
         out.append({"exp": "b200_jacobi_cost_at", "tile_time_space": [tt, ss], "model_cost_cycles": r["cost"],
                     "local_elems": r["local_elems"]})
