@@ -60,6 +60,14 @@ constexpr int kTx = 4;       // dx candidates per thread (same byte phase, strid
 #define SP_ME_R16_TY 8
 #endif
 constexpr int sp_me_kTy = 8;
+// SP_ME_PHASE_FMA (off): build the byte-phase copies on the FMA pipe (IMAD.HI + IMAD per word)
+// instead of the ALU's funnel shift, to unload the binding ALU pipe (the FMA pipe idles at
+// ~3 %).  Measured slower (r3y, A/B x 3): M4 8.41-8.48 vs 8.30 ms, CIF +-16 72.0 vs 72.7 % —
+// the phase build sits on the path to the CTA barrier, and two dependent multiplies per word
+// lengthen it more than the ALU slots they free.
+#ifndef SP_ME_PHASE_FMA
+#define SP_ME_PHASE_FMA 0
+#endif
 #ifndef SP_ME_SCRAMBLE
 #define SP_ME_SCRAMBLE 0
 #endif
@@ -207,6 +215,17 @@ constexpr uint32_t kKeyMul = 32769u;
 constexpr uint32_t kInvalidSad = 0x1FFF0u;
 __device__ __forceinline__ uint32_t tie_bits(int dx, int dy, int R) {
     return ((uint32_t)(abs(dx) + abs(dy)) << 8) | ((uint32_t)(dy + R) << 1) | (dx > 0 ? 1u : 0u);
+}
+
+// (hi:lo) >> 8 ph for m = 2^(32 - 8 ph), ph in 1..3, on the FMA pipe: lo >> 8 ph = the high word
+// of lo * m, hi << (32 - 8 ph) = the low word of hi * m, and the two do not overlap, so one
+// multiply-add joins them.  (Inline PTX: the compiler would turn a multiply by a power of two
+// back into an ALU shift.)
+__device__ __forceinline__ uint32_t shr_bytes_fma(uint32_t lo, uint32_t hi, uint32_t m) {
+    uint32_t l, r;
+    asm("mul.hi.u32 %0, %1, %2;" : "=r"(l) : "r"(lo), "r"(m));
+    asm("mad.lo.u32 %0, %1, %2, %3;" : "=r"(r) : "r"(hi), "r"(m), "r"(l));
+    return r;
 }
 
 // Tail candidate t of thread (warp, lane): the candidates outside the 2R x 2R register
@@ -437,14 +456,24 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
 #pragma unroll
                     for (int c = 0; c < v4_per_row; ++c) wv[c] = rowv[c];
                     uint4* out = reinterpret_cast<uint4*>(phase_copy(s, ph) + r * win);
+#if SP_ME_PHASE_FMA
+                    const uint32_t m = 1u << (32 - 8 * ph);
+#endif
 #pragma unroll
                     for (int c = 0; c < v4_per_row; ++c) {
                         const uint32_t nx = c + 1 < v4_per_row ? wv[c + 1].x : 0u;
                         uint4 o;
+#if SP_ME_PHASE_FMA
+                        o.x = shr_bytes_fma(wv[c].x, wv[c].y, m);
+                        o.y = shr_bytes_fma(wv[c].y, wv[c].z, m);
+                        o.z = shr_bytes_fma(wv[c].z, wv[c].w, m);
+                        o.w = shr_bytes_fma(wv[c].w, nx, m);
+#else
                         o.x = __funnelshift_r(wv[c].x, wv[c].y, 8 * ph);
                         o.y = __funnelshift_r(wv[c].y, wv[c].z, 8 * ph);
                         o.z = __funnelshift_r(wv[c].z, wv[c].w, 8 * ph);
                         o.w = __funnelshift_r(wv[c].w, nx, 8 * ph);
+#endif
                         out[c] = o;
                     }
                 }
