@@ -66,14 +66,16 @@ def test_peer_fused_halo_equals_oracle(world, tmp_path):
 
 
 @pytest.mark.timeout(600)
-@pytest.mark.parametrize("world,space_tile", [(2, 256), (3, 256), (2, 8)])
-def test_peer_persistent_halo_equals_oracle(world, space_tile, tmp_path):
+@pytest.mark.parametrize("world,space_tile,n,tt,steps_list", [
+    (2, 256, 12011, 16, [37, 16, 5]), (3, 256, 12011, 16, [37, 16, 5]), (2, 8, 12011, 16, [37, 16, 5]),
+    # the bench's N > 1 time tile with the persistent in-place geometry (space tile 0)
+    (2, 0, 50021, 128, [300, 128, 7]), (3, 0, 50021, 128, [300, 128, 7])])
+def test_peer_persistent_halo_equals_oracle(world, space_tile, n, tt, steps_list, tmp_path):
     """sp_jacobi1d_timetiled_peer_fused: every pass of a call in one persistent launch per
     rank, halos pushed by the last edge tile of each side (space tile 8 < halo 16: two edge
-    tiles per side).  Three calls (37, 16, 5 steps) exercise the call-boundary handshake."""
+    tiles per side).  Three calls exercise the call-boundary handshake."""
     import oracle
     import sp_inputs
-    n, tt, steps_list = 12011, 16, [37, 16, 5]
     mp.spawn(_worker, args=(world, _free_port(), n, steps_list, tt, str(tmp_path), True, space_tile), nprocs=world,
              join=True)
     got = np.concatenate([np.load(tmp_path / f"r{r}.npy") for r in range(world)])
