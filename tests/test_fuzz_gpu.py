@@ -23,7 +23,7 @@ def _jacobi_cases(seed, count):
     for _ in range(count):
         n = int(rng.integers(3, 60000))
         steps = int(rng.integers(0, 160))
-        tt = int(rng.choice([1, 3, 8, 16, 17, 32, 64, 100]))
+        tt = int(rng.choice([1, 3, 8, 16, 17, 32, 64, 100, 128]))
         H = sp.halo_of(tt)
         s_max = sp.jacobi1d_plan(1 << 20, 64, tt, 0)["space_tile"]
         S = 0 if rng.random() < 0.4 else int(rng.integers(1, max(2, s_max // 4 + 1))) * 4
