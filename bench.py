@@ -69,10 +69,10 @@ def workload(world, tt):
 
 def _geometry(n_local, T, tt, persistent):
     """The Jacobi pass kernel's geometry as the library plans it (include/sp.h sp_jacobi_plan):
-    the persistent launches take the in-place one at Tt >= 16, the staged one otherwise."""
+    the persistent launches take the in-place one at Tt >= 48, the staged one otherwise."""
     import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
     pl = sp.jacobi1d_plan(n_local, T, tt, 0)
-    if persistent and tt >= 16:
+    if persistent and tt >= 48:
         k = (pl["persistent_space_tile"] + 2 * pl["halo"]) // 64  # strip = 64 K cells per warp
         return f"in place: {2 * k} cells/lane in {k + 1} packed registers, one stage per warp"
     return f"staged: {pl['cells_per_thread']} cells/lane, two stages per warp"
@@ -559,7 +559,7 @@ def run_ours(args, rank, world, local_rank):
         "jacobi": {"value": round(jac_val, 2), "unit": "GPoint-updates/s", "ms_per_step": round(jac_ms / K, 4),
                    "n_local": n_local, "passes_per_step": -(-T // tt),
                    # the persistent launches (single GPU and peer-fused) take the in-place
-                   # geometry at Tt >= 16, the staged one below (include/sp.h sp_jacobi_plan)
+                   # geometry at Tt >= 48, the staged one below (include/sp.h sp_jacobi_plan)
                    "space_tile": sp.jacobi1d_plan(n_local, T, tt, 0)["persistent_space_tile" if persistent
                                                                       else "space_tile"],
                    "geometry": _geometry(n_local, T, tt, persistent)},

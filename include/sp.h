@@ -185,9 +185,10 @@ typedef struct {
     int32_t smem_bytes;  /* dynamic shared memory per CTA */
     int32_t cells_per_thread; /* register cells per thread */
     /* the persistent launch over DEVICE memory (sp_jacobi1d_timetiled_fused, _stream with
-     * device in / out) uses the in-place geometry when time_tile >= 16 (80 register cells per
-     * thread in 41 packed registers, alternating sweeps; below 16 the pass is HBM-bound and the
-     * staged geometry is kept); with space_tile = 0 its tile is larger: */
+     * device in / out, sp_jacobi1d_host, the peer-fused launch) uses the in-place geometry
+     * when time_tile >= 48 (112 register cells per thread in 57 packed registers, alternating
+     * sweeps; with shorter passes the staged geometry is faster); with space_tile = 0 its tile
+     * is larger: */
     int64_t persistent_space_tile; /* S of that launch (space_tile if given) */
     int64_t persistent_tiles;      /* its tiles per pass (<= tiles: flags sized by `tiles` suffice) */
 } sp_jacobi_plan;
@@ -208,7 +209,9 @@ int sp_jacobi1d_tile_footprint(int64_t n, int32_t h, int64_t x0, int64_t space_t
  * staged footprint as the kernel computed it (for checking against the planner). */
 int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32_t time_tile,
                           int32_t space_tile, int64_t* footprint_log, void* stream);
-/* Same result as sp_jacobi1d_timetiled, with every pass in ONE persistent launch: a tile of
+/* Same result as sp_jacobi1d_timetiled, with every pass in ONE persistent launch (time_tile
+ * >= 32; with shorter passes the call runs one launch per pass, which is faster there —
+ * SP_JACOBI_FUSED_PERSISTENT=1 keeps the persistent launch): a tile of
  * pass p+1 starts as soon as the tiles of pass p within reach of its halo are done, so pass
  * boundaries cost neither a launch nor a partly-filled last round of tiles (H8's inter-tile
  * synchronisation, done per tile instead of per pass).
@@ -219,9 +222,10 @@ int sp_jacobi1d_timetiled(float* a, float* work, int64_t n, int32_t steps, int32
  * Every CTA of the launch must be co-resident (the grid is the occupancy limit); a tile whose
  * dependences never complete traps after ~20 s instead of hanging.  footprint_log as in
  * sp_jacobi1d_timetiled, laid out [passes][persistent_tiles][2] (sp_jacobi1d_plan).
- * Geometry: the in-place kernel (sp_jacobi_plan.persistent_space_tile): each lane keeps 40
- * packed cell pairs in 41 registers and alternates ascending / descending sweeps, so no second
- * register copy is needed; the tile is staged once per warp and stored from registers. */
+ * Geometry: the in-place kernel (sp_jacobi_plan.persistent_space_tile): each lane keeps 56
+ * packed cell pairs in 57 registers (one 12-warp CTA per SM) and alternates ascending /
+ * descending sweeps, so no second register copy is needed; the tile is staged once per warp
+ * and stored from registers. */
 int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n, int32_t steps,
                                 int32_t time_tile, int32_t space_tile, int64_t* footprint_log, void* stream);
 

@@ -1176,9 +1176,11 @@ int variant_index() {
 // keeps the staged TMA move-out of the default geometry: the in-place kernel's direct
 // 16-byte register stores would cross PCIe as small writes.  SP_JACOBI_VARIANT_FUSED (or
 // SP_JACOBI_VARIANT) overrides.
-// Below a time tile of 16 the pass is HBM-bound and the in-place kernel's scattered 16-byte
-// stores cost more than its shorter halo saves (J3 persistent: Tt = 4 / 8: 34.6 / 17.3 ms in
-// place vs 27.4 / 15.8 staged; Tt = 16: 9.98 vs 10.2), so short time tiles stay staged.
+// Below a time tile of kInPlaceMinTt the passes are short and the in-place kernel's
+// lane-strided 16-byte stores cost more than its shorter halo saves, so the persistent launch
+// stays staged: J3 persistent, K = 56 in place vs K = 28 staged (r4c): Tt = 16: 11.18 vs 10.83
+// ms, 20: 10.91 vs 11.01, 24: 9.36 vs 8.83, 32: 8.20 vs 7.70, 48: 6.88-6.91 vs 6.97.
+constexpr int kInPlaceMinTt = 48;
 int persistent_variant_index(int32_t time_tile) {
     static int idx = [] {
         const char* e = std::getenv("SP_JACOBI_VARIANT_FUSED");
@@ -1187,7 +1189,7 @@ int persistent_variant_index(int32_t time_tile) {
         return (i >= 0 && i < kNumVariants) ? i : kPersistentVariant;
     }();
     static const bool forced = std::getenv("SP_JACOBI_VARIANT_FUSED") || std::getenv("SP_JACOBI_VARIANT");
-    return (time_tile < 16 && !forced) ? variant_index() : idx;
+    return (time_tile < kInPlaceMinTt && !forced) ? variant_index() : idx;
 }
 
 int smem_bytes(const Variant& v) { return v.stage_floats * (int)sizeof(float); }
@@ -1543,6 +1545,18 @@ extern "C" int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags
                                            int32_t steps, int32_t time_tile, int32_t space_tile,
                                            int64_t* footprint_log, void* stream) {
     if (!a || !work || a == work) return SP_ERR_INVALID_ARG;
+    // Tt < 32 (short tiles, HBM-bound below 16): one launch per pass streams faster than the
+    // persistent launch, whose per-tile unit counter, dependence polls and publications no
+    // longer hide under the tile's few steps — J3 per pass vs persistent (r3v, r4c): Tt = 4:
+    // 26.6 vs 29.6 ms, 8: 12.8 vs 17.0, 16: 9.37 vs 10.83, 24: 8.57 vs 8.83; 32: 7.94 vs 7.70.
+    // Same result, same footprint-log layout (the staged geometry either way);
+    // SP_JACOBI_FUSED_PERSISTENT=1 keeps the persistent launch (tests, sweeps).
+    const char* fp = std::getenv("SP_JACOBI_FUSED_PERSISTENT");  // (read per call: tests toggle it)
+    const bool force_persistent = (fp && std::atoi(fp) != 0) || std::getenv("SP_JACOBI_VARIANT_FUSED");
+    if (time_tile >= 1 && time_tile < 32 && !force_persistent) {
+        if (!flags || flags_len < 1) return SP_ERR_INVALID_ARG;  // (the same contract at every time tile)
+        return sp_jacobi1d_timetiled(a, work, n, steps, time_tile, space_tile, footprint_log, stream);
+    }
     return sp_jacobi1d_timetiled_stream(a, a, a, work, flags, flags_len, n, steps, time_tile, space_tile, 0,
                                         footprint_log, stream);
 }

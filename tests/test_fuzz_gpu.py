@@ -32,7 +32,7 @@ def _jacobi_cases(seed, count):
 
 
 @pytest.mark.parametrize("seed", range(8))
-def test_jacobi_random_shapes_all_entry_points(seed):
+def test_jacobi_random_shapes_all_entry_points(seed, monkeypatch):
     checked = 0
     for n, steps, tt, S, H in _jacobi_cases(100 + seed, 6):
         checked += 1
@@ -42,9 +42,11 @@ def test_jacobi_random_shapes_all_entry_points(seed):
         d = torch.from_numpy(a0.copy()).cuda()
         sp.jacobi1d_timetiled(d, steps, tt, S)
         assert np.array_equal(_bits(d.cpu().numpy()), want), ("per-pass", case)
-        d = torch.from_numpy(a0.copy()).cuda()
-        sp.jacobi1d_timetiled_fused(d, steps, tt, S)
-        assert np.array_equal(_bits(d.cpu().numpy()), want), ("persistent", case)
+        for route in ("1", "0"):  # the persistent launch at every Tt; the default route (per pass below 16)
+            monkeypatch.setenv("SP_JACOBI_FUSED_PERSISTENT", route)
+            d = torch.from_numpy(a0.copy()).cuda()
+            sp.jacobi1d_timetiled_fused(d, steps, tt, S)
+            assert np.array_equal(_bits(d.cpu().numpy()), want), ("persistent" if route == "1" else "fused", case)
         if steps > 0:
             tiles = sp.jacobi1d_plan(n, steps, tt, S)["tiles"]
             reach = -(-H // (S if S else sp.jacobi1d_plan(n, steps, tt, 0)["space_tile"]))

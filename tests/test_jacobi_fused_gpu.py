@@ -12,6 +12,13 @@ import sp_inputs
 pytestmark = pytest.mark.gpu
 
 
+@pytest.fixture(autouse=True)
+def _persistent_at_every_time_tile(monkeypatch):
+    """Below Tt = 16 sp_jacobi1d_timetiled_fused runs one launch per pass by default (faster
+    when HBM binds); this module tests the persistent kernel itself at every time tile."""
+    monkeypatch.setenv("SP_JACOBI_FUSED_PERSISTENT", "1")
+
+
 def _run(a0, steps, tt, S=0, log=None):
     d = torch.from_numpy(a0.copy()).cuda()
     sp.jacobi1d_timetiled_fused(d, steps, tt, S, footprint_log=log)
@@ -31,11 +38,12 @@ def test_J1_config():
 
 
 @pytest.mark.parametrize("n", [3, 5, 33, 64, 65, 1000, 4097])
-@pytest.mark.parametrize("steps", [0, 1, 16, 17, 53])
+@pytest.mark.parametrize("steps", [0, 1, 16, 17, 53, 130])
 def test_edge_shapes(n, steps):
     a = sp_inputs.jacobi_input(n, seed=n * 3 + steps)
     want = oracle.jacobi1d(a, steps)
-    for tt, S in [(16, 32), (16, 4), (5, 8), (1, 4), (16, 0)]:
+    # (16, ...) and below: the staged persistent geometry; 48 / 64: the in-place one
+    for tt, S in [(16, 32), (16, 4), (5, 8), (1, 4), (16, 0), (48, 0), (64, 32), (64, 4)]:
         _check(_run(a, steps, tt, S), want)
 
 
@@ -109,3 +117,22 @@ def test_repeated_calls_reuse_flags():
         sp.jacobi1d_timetiled_fused(d, 40, 16, 0, work=w, flags=flags)
     torch.cuda.synchronize()
     _check(d.cpu().numpy(), oracle.jacobi1d(a, 120))
+
+
+@pytest.mark.parametrize("tt", [1, 5, 8, 15])
+def test_small_time_tiles_default_route(tt, monkeypatch):
+    """Default route below Tt = 16 (per-pass launches): same bits and the same footprint log
+    layout as the persistent launch."""
+    monkeypatch.delenv("SP_JACOBI_FUSED_PERSISTENT", raising=False)
+    n, steps = 20011, 53
+    a = sp_inputs.jacobi_input(n, seed=tt)
+    want = oracle.jacobi1d(a, steps)
+    plan = sp.jacobi1d_plan(n, steps, tt, 0)
+    logs = []
+    for env in (None, "1"):
+        if env:
+            monkeypatch.setenv("SP_JACOBI_FUSED_PERSISTENT", env)
+        log = torch.zeros(plan["passes"] * plan["persistent_tiles"] * 2, dtype=torch.int64, device="cuda")
+        _check(_run(a, steps, tt, 0, log=log), want)
+        logs.append(log.cpu().numpy())
+    assert np.array_equal(logs[0], logs[1])

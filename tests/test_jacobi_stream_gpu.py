@@ -51,7 +51,9 @@ def test_host_in_out_shapes(n, steps):
     """pinned host in and out (the last pass's move-out writes host memory), all pass counts"""
     a = sp_inputs.jacobi_input(n, seed=n + 7 * steps)
     want = oracle.jacobi1d(a, steps)
-    for tt, S in [(16, 0), (16, 8), (5, 4)]:
+    # 16 / 5: the staged persistent geometry; 48 / 64: the in-place one (host output: its
+    # staged-move-out instantiation)
+    for tt, S in [(16, 0), (16, 8), (5, 4), (64, 0), (48, 8)]:
         _check(_stream(a, steps, tt, S, -1, "host", "host"), want)
         _check(_stream(a, steps, tt, S, 0, "host", "cuda"), want)
         _check(_stream(a, steps, tt, S, 16, "cuda", "host"), want)

@@ -50,7 +50,7 @@ def _stress_lib():
 
 def test_stragglers_keep_the_persistent_orders_exact(tmp_path):
     out = str(tmp_path / "jstress.npz")
-    env = dict(os.environ, SP_LIB=_stress_lib())
+    env = dict(os.environ, SP_LIB=_stress_lib(), SP_JACOBI_FUSED_PERSISTENT="1")  # (persistent at every Tt)
     subprocess.check_call([sys.executable, "-c", CHILD, ROOT, out, repr(CASES)], env=env, cwd=ROOT, timeout=600)
     got = np.load(out)
     for k, (n, steps, tt, S) in enumerate(CASES):

@@ -22,15 +22,26 @@ mark("sp.jacobi1d_timetiled")
 sp.jacobi1d_timetiled(a, 37, 16, 256)
 mark("sp.jacobi1d_timetiled")
 sp.jacobi1d_timetiled(a, 20, 5, 0)
-mark("sp.jacobi1d_timetiled_fused")
+mark("sp.jacobi1d_timetiled_fused (persistent launch at every time tile)")
+os.environ["SP_JACOBI_FUSED_PERSISTENT"] = "1"
 sp.jacobi1d_timetiled_fused(a, 37, 16, 256)
 sp.jacobi1d_timetiled_fused(a, 20, 5, 8)
+mark("sp.jacobi1d_timetiled_fused (in-place geometry: Tt >= 48)")
+sp.jacobi1d_timetiled_fused(a, 150, 64, 0)
+sp.jacobi1d_timetiled_fused(a, 130, 48, 8)
+del os.environ["SP_JACOBI_FUSED_PERSISTENT"]
+mark("sp.jacobi1d_timetiled_fused (default route below Tt = 32: one launch per pass)")
+sp.jacobi1d_timetiled_fused(a, 37, 16, 256)
 mark("sp.jacobi1d_timetiled_stream (wavefront, device)")
 o = torch.empty_like(a)
 sp.jacobi1d_timetiled_stream(a, o, 37, 16, 256, 4)
+sp.jacobi1d_timetiled_stream(a, o, 150, 64, 8, 64)
 mark("sp.jacobi1d_host (pinned in/out, 3 passes)")
 h = a.cpu().pin_memory()
 sp.Jacobi1DHost(4099, 37, 16, 256).run(h)
+mark("sp.jacobi1d_host (in place geometry, host-output instantiation)")
+sp.Jacobi1DHost(4099, 150, 64, 8).run(h)
+sp.Jacobi1DHost(4099, 150, 64, 0).run(h)
 mark("sp.jacobi1d_host (1 pass: redirect + copy)")
 sp.Jacobi1DHost(4099, 9, 16, 0).run(h)
 mark("sp.jacobi1d_resident (one cluster, small and large shapes)")
