@@ -1,6 +1,7 @@
 """The latency-bound BASELINE configs 1 and 2 on one B200 (development aid):
 J1 = Jacobi N = 4096, T = 64, Tt = 16 through the persistent pass kernel and the
 cluster-resident kernel; M2 = one CIF pair, +-16 (full surface off / on)."""
+import os
 import sys
 
 import numpy as np
@@ -30,7 +31,12 @@ def main():
     a0 = torch.from_numpy(sp_inputs.jacobi_input(4096, seed=2008)).cuda()
     a, w = a0.clone(), torch.empty_like(a0)
     fl = torch.empty(64, dtype=torch.int32, device="cuda")
-    for name, fn in [("J1 persistent pass kernel (Tt 16, S 512)", lambda: sp.jacobi1d_timetiled_fused(a, 64, 16, 512, work=w, flags=fl)),
+    def persistent():  # (the fused call's default route below Tt = 32 is per-pass launches)
+        os.environ["SP_JACOBI_FUSED_PERSISTENT"] = "1"
+        sp.jacobi1d_timetiled_fused(a, 64, 16, 512, work=w, flags=fl)
+        del os.environ["SP_JACOBI_FUSED_PERSISTENT"]
+
+    for name, fn in [("J1 persistent pass kernel (Tt 16, S 512)", persistent),
                      ("J1 per-pass launches (Tt 16, S 512)", lambda: sp.jacobi1d_timetiled(a, 64, 16, 512, work=w)),
                      ("J1 cluster-resident", lambda: sp.jacobi1d_resident(a0, 64, out=a))]:
         b, m = ev_time(fn)
