@@ -138,6 +138,14 @@ struct MeArgs {
     uint32_t total_mb;  // macroblocks of this launch (fast kernel)
     uint32_t nrows;     // macroblock rows of this launch (total_mb / mbx)
     FastDiv div_per_pair, div_mbx;  // by mb_rows * mbx and by mbx
+    // Class order (R = 16, whole frames, many macroblocks; 0 otherwise): the launch's index
+    // space runs over the interior macroblocks of every pair first, then the top / bottom rows,
+    // then the left / right columns, then the four corners, so the one code path each class
+    // needs (the full search, or a half-frame border search) is the only one the SM's warps run
+    // at a time — mixed, the four search loops do not fit the instruction cache together.
+    int32_t border_order;
+    uint32_t cls_end[3];                 // first index of the rows / columns / corners class
+    FastDiv div_int, div_icols, div_rows2, div_cols2;  // by (rows-2)(mbx-2), mbx-2, 2(mbx-2), 2(rows-2)
 };
 
 // Fused all-gather of the results over peer memory (sp_me_sad_search_gather): every
@@ -241,6 +249,117 @@ __device__ __forceinline__ bool tail_candidate(int warp, int lane, int t, int& d
     return col;
 }
 
+// Tail candidate t of thread (warp, lane) as (column?, k): a column tail has dy = dy0 + k, a
+// row tail dx = dx0 + k, in the candidate frame whose main block starts at (dx0, dy0).
+template <int R>
+__device__ __forceinline__ bool tail_slot(int warp, int lane, int t, int& k) {
+    int dx, dy;
+    const bool col = tail_candidate<R>(warp, lane, t, dx, dy);
+    k = col ? dy + R : dx + R;
+    return col;
+}
+
+// Border macroblocks (one-warp CTAs, class order only).  When the valid displacements of a
+// macroblock fit in R + 1 columns (or rows) — the first / last macroblock column (row) of a
+// frame whose width (height) is a multiple of 16 — at most half of the 2R x 2R main candidates
+// can be valid: the thread tile then shrinks to TX = 2 dx (TY = 4 dy) candidates over a
+// candidate frame starting at dx0 (dy0), so the warp computes the valid half instead of
+// computing and masking all of it (CIF +-16: 76 of 396 macroblocks, 9 % of the SAD work).
+// Candidates dx = dx0 + p + 4 (TX g + j), dy = dy0 + TY d + i; column tails at dx = dx0 +
+// 4 TX kGx, row tails at dy = dy0 + TY kDy; invalid ones never enter the key.  Returns the
+// thread's minimal key.  (Out of line: the interior path keeps its registers and code layout.)
+template <int R, int TX, int TY>
+__device__ __noinline__ uint32_t border_search(const uint8_t* smem, int s, int dx0, int dy0, int dxlo, int dxhi,
+                                               int dylo, int dyhi, int tid) {
+    using G = MeGeom<R>;
+    static_assert(G::kWarps == 1, "border search: one-warp CTAs");
+    // (the kernel's shared-memory layout: raw window / byte-phase copies / current block)
+    auto phase_base = [&](int ph) -> const uint8_t* {
+        return ph == 0 ? smem + s * G::kCopy
+                       : smem + G::kOffPh + (3 * (G::kPhaseSets == 1 ? 0 : s) + ph - 1) * G::kSlot + 32 * ph;
+    };
+    const uint4* cq = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+    constexpr int win = G::kWin;
+    constexpr int kDy = G::kThreads / (4 * G::kGx);
+    constexpr int NW = TX + 3;
+    const int lane = tid & 31, warp = tid >> 5;
+    const int p = tid & 3, g = (tid >> 2) % G::kGx, d = tid / (4 * G::kGx);
+    const int CX = dx0 + 4 * TX * G::kGx, CY = dy0 + TY * kDy;  // tail column / row
+    // tails: window address (row dy + R, byte dx + R of the matching phase copy) and key bits
+    const uint8_t* tp[G::kTailPer];
+    uint32_t ttie[G::kTailPer];
+    bool tval[G::kTailPer];
+#pragma unroll
+    for (int t = 0; t < G::kTailPer; ++t) {
+        int k;
+        const bool col = tail_slot<R>(warp, lane, t, k);
+        const bool inside = k < (col ? TY * kDy : 4 * TX * G::kGx);  // (beyond: not a candidate)
+        const int dx = col ? CX : dx0 + k, dy = col ? dy0 + k : CY;
+        tval[t] = inside && dx >= dxlo && dx <= dxhi && dy >= dylo && dy <= dyhi;
+        ttie[t] = tie_bits(dx, dy, R);
+        tp[t] = inside ? phase_base((dx + R) & 3) + (dy + R) * win + 4 * ((dx + R) >> 2) : phase_base(0);
+    }
+    uint32_t acc[TX][TY], ta[G::kTailPer];
+#pragma unroll
+    for (int j = 0; j < TX; ++j)
+#pragma unroll
+        for (int i = 0; i < TY; ++i) acc[j][i] = 0;
+#pragma unroll
+    for (int t = 0; t < G::kTailPer; ++t) ta[t] = 0;
+    const uint8_t* rowp = phase_base(p) + (dy0 + R + TY * d) * win + 4 * ((dx0 + R) / 4 + TX * g);
+    uint32_t Rw[TY][NW];
+    auto load_row = [&](uint32_t(&w)[NW], const uint8_t* src) {
+        if constexpr (TX == 4) {
+            const uint4 a = *reinterpret_cast<const uint4*>(src);
+            const uint4 b = *reinterpret_cast<const uint4*>(src + 16);
+            w[0] = a.x; w[1] = a.y; w[2] = a.z; w[3] = a.w; w[4] = b.x; w[5] = b.y; w[6] = b.z;
+        } else {  // 8-byte aligned: (dx0 + R) and 8 g are multiples of 8
+            const uint2 a = *reinterpret_cast<const uint2*>(src);
+            const uint2 b = *reinterpret_cast<const uint2*>(src + 8);
+            w[0] = a.x; w[1] = a.y; w[2] = b.x; w[3] = b.y; w[4] = *reinterpret_cast<const uint32_t*>(src + 16);
+        }
+    };
+#pragma unroll
+    for (int rr = 0; rr < TY - 1; ++rr) load_row(Rw[rr], rowp + rr * win);
+#pragma unroll 1
+    for (int vb = 0; vb < kMB; vb += TY) {
+#pragma unroll
+        for (int vv = 0; vv < TY; ++vv) {
+            const int v = vb + vv;
+            load_row(Rw[(vv + TY - 1) % TY], rowp + (v + TY - 1) * win);
+            const uint4 cv = cq[v];
+            const uint32_t Cv[4] = {cv.x, cv.y, cv.z, cv.w};
+#pragma unroll
+            for (int t = 0; t < G::kTailPer; ++t) {
+                const uint32_t* tq = reinterpret_cast<const uint32_t*>(tp[t] + v * win);
+#pragma unroll
+                for (int k = 0; k < 4; ++k) ta[t] = sad4(tq[k], Cv[k], ta[t]);
+            }
+#pragma unroll
+            for (int k = 0; k < 4; ++k)
+#pragma unroll
+                for (int i = 0; i < TY; ++i)
+#pragma unroll
+                    for (int j = 0; j < TX; ++j) acc[j][i] = sad4(Rw[(vv + i) % TY][j + k], Cv[k], acc[j][i]);
+        }
+    }
+    uint32_t key = 0xffffffffu;
+#pragma unroll
+    for (int j = 0; j < TX; ++j) {
+        const int dx = dx0 + p + 4 * (TX * g + j);
+#pragma unroll
+        for (int i = 0; i < TY; ++i) {
+            const int dy = dy0 + TY * d + i;
+            if (dx >= dxlo && dx <= dxhi && dy >= dylo && dy <= dyhi)
+                key = min(key, acc[j][i] * kKeyMul + tie_bits(dx, dy, R));
+        }
+    }
+#pragma unroll
+    for (int t = 0; t < G::kTailPer; ++t)
+        if (tval[t]) key = min(key, ta[t] * kKeyMul + ttie[t]);
+    return key;
+}
+
 // Frames still streaming in (sp_me_search_host): wait for a pair's ready flag (relaxed poll,
 // then an acquire and a proxy fence order the observed copy before the TMA reads that follow).
 // Out of line: the common device-resident path keeps its register / uniform-datapath layout.
@@ -273,6 +392,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     __shared__ __align__(8) uint64_t full[2];
     __shared__ uint32_t red32[2][nwarps];  // per-stage per-warp minimal key
     __shared__ uint32_t lsum[2];           // per-stage SAD of the corner candidate (R, R)
+    __shared__ uint32_t ltie[2];           // (one-warp CTAs) its tie bits, ~0u if invalid
     // align to 128 bytes by offsetting the shared pointer itself (keeps LDS/STS addressing)
     uint8_t* smem = smem_raw + ((128u - (smem_addr(smem_raw) & 127u)) & 127u);
 
@@ -300,6 +420,28 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const uint32_t pair = f / (uint32_t)A.mb_rows;
         return Pos{(int)pair, (int)(f - pair * (uint32_t)A.mb_rows), (int)col};
 #else
+        if constexpr (nwarps == 1) {
+            if (A.border_order) {  // class order (MeArgs::border_order; whole frames, flat_mb0 = 0)
+                const uint32_t mbx2 = mbx - 2, rows2 = (uint32_t)A.mb_rows - 2;
+                if (mb < A.cls_end[0]) {  // interior
+                    const uint32_t pair = fdiv(mb, A.div_int), k = mb - pair * (rows2 * mbx2);
+                    const uint32_t r = fdiv(k, A.div_icols);
+                    return Pos{(int)pair, (int)(1 + r), (int)(1 + k - r * mbx2)};
+                }
+                if (mb < A.cls_end[1]) {  // top / bottom rows without the corners
+                    const uint32_t m = mb - A.cls_end[0], pair = fdiv(m, A.div_rows2), k = m - pair * 2 * mbx2;
+                    const bool top = k < mbx2;
+                    return Pos{(int)pair, top ? 0 : (int)rows2 + 1, (int)(1 + (top ? k : k - mbx2))};
+                }
+                if (mb < A.cls_end[2]) {  // left / right columns without the corners
+                    const uint32_t m = mb - A.cls_end[1], pair = fdiv(m, A.div_cols2), k = m - pair * 2 * rows2;
+                    const bool left = k < rows2;
+                    return Pos{(int)pair, (int)(1 + (left ? k : k - rows2)), left ? 0 : (int)mbx - 1};
+                }
+                const uint32_t m = mb - A.cls_end[2];  // corners
+                return Pos{(int)(m >> 2), (m & 2) ? (int)rows2 + 1 : 0, (m & 1) ? (int)mbx - 1 : 0};
+            }
+        }
         mb += A.flat_mb0;
         const uint32_t pair = fdiv(mb, A.div_per_pair), rem = mb - pair * per_pair;
         const uint32_t byr = fdiv(rem, A.div_mbx);
@@ -324,9 +466,16 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         for (int w = 1; w < nwarps; ++w) b = min(b, red32[sp][w]);
         const uint32_t lsad = lsum[sp];
         const Pos q = locate(mbp);
-        const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
-        const bool lvalid = A.unrestricted || ((x0 + R + 16 <= W) && (y0 + R + 16 <= Hf));
-        if (lvalid) b = min(b, lsad * kKeyMul + tie_bits(R, R, R));
+        bool lvalid;
+        if constexpr (nwarps == 1) {  // the corner candidate of the searched frame (border search: moved)
+            const uint32_t lt = ltie[sp];
+            lvalid = lt != 0xffffffffu;
+            if (lvalid) b = min(b, lsad * kKeyMul + lt);
+        } else {
+            const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
+            lvalid = A.unrestricted || ((x0 + R + 16 <= W) && (y0 + R + 16 <= Hf));
+            if (lvalid) b = min(b, lsad * kKeyMul + tie_bits(R, R, R));
+        }
         const size_t idx = ((size_t)q.pair * A.mb_rows + q.byr) * mbx + q.bx;
         const uint32_t sad = b / kKeyMul, tie = b - sad * kKeyMul;
         const int dy = (int)((tie >> 1) & 127) - R;
@@ -404,15 +553,18 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         }
         for (int q = 0; q < kTy / 4; ++q) tieB[tid][q] = make_uint4(b[4 * q], b[4 * q + 1], b[4 * q + 2], b[4 * q + 3]);
     }
-    // tail candidates: tie bits and staged-copy offsets (stage 0, stage 1), per thread
-    __shared__ uint32_t tinfo[G::kTailPer][1 + G::kPhaseSets][G::kThreads];
+    // tail candidates: tie bits and staged-copy offsets (stage 0, stage 1), per thread.  Two
+    // offsets even with one phase-copy set: a tail of byte phase 0 reads the TMA'd window
+    // itself, which alternates between the two stages (one-warp CTAs read stage 0's window on
+    // every macroblock until round-2 session 3 — wrong tails from a CTA's second macroblock on)
+    __shared__ uint32_t tinfo[G::kTailPer][3][G::kThreads];
 #pragma unroll
     for (int t = 0; t < G::kTailPer; ++t) {
         int dxt, dyt;
         tail_candidate<R>(warp, lane, t, dxt, dyt);
         tinfo[t][0][tid] = tie_bits(dxt, dyt, R);
 #pragma unroll
-        for (int st = 0; st < G::kPhaseSets; ++st)
+        for (int st = 0; st < 2; ++st)
             tinfo[t][1 + st][tid] =
                 (uint32_t)(phase_copy(st, (dxt + R) & 3) - smem) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
     }
@@ -510,6 +662,44 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             const int blo = -R + kDyWarp * warp, bhi = blo + kDyWarp - 1;
             main_dead = bhi < dylo || blo > dyhi;
         }
+        // the corner candidate of the searched frame — (R, R), or the moved corner of a border
+        // search: 64 (row, word) pieces over warp 0 (one-warp CTAs also post its tie bits)
+        auto corner = [&](int cx, int cy, bool cvalid) {
+            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + s * G::kCopy + (cy + R) * win) + (cx + R) / 4;
+            const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
+            uint32_t part = 0;
+#pragma unroll
+            for (int o = lane; o < 64; o += 32) {
+                const int v = o >> 2, k = o & 3;
+                const uint4 cv = cq4[v];
+                const uint32_t cw = k == 0 ? cv.x : k == 1 ? cv.y : k == 2 ? cv.z : cv.w;
+                part = sad4(rw[v * (win / 4) + k], cw, part);
+            }
+            const uint32_t tot = __reduce_add_sync(0xffffffffu, part);
+            if (lane == 0) {
+                lsum[s] = tot;
+                if constexpr (nwarps == 1) ltie[s] = cvalid ? tie_bits(cx, cy, R) : 0xffffffffu;
+            }
+        };
+        uint32_t key = 0xffffffffu;
+        bool bsearch = false;  // (class order, one-warp CTAs) this macroblock took a half-frame border search
+        if constexpr (nwarps == 1) {
+            if (A.border_order && !interior) {
+                // valid dx within R + 1 columns from an 8-byte-aligned origin, or dy within R + 1 rows
+                const int cx = dxlo - ((dxlo + R) & 7);
+                const bool hx = dxhi <= cx + R, hy = dyhi - dylo <= R;
+                if (hx || hy) {
+                    const int dx0 = hx ? cx : -R, dy0 = hy ? dylo : -R;
+                    const int CX = dx0 + (hx ? R : 2 * R), CY = dy0 + (hy ? R : 2 * R);
+                    if (hx && hy) key = border_search<R, 2, 4>(smem, s, dx0, dy0, dxlo, dxhi, dylo, dyhi, tid);
+                    else if (hx) key = border_search<R, 2, 8>(smem, s, dx0, dy0, dxlo, dxhi, dylo, dyhi, tid);
+                    else key = border_search<R, 4, 4>(smem, s, dx0, dy0, dxlo, dxhi, dylo, dyhi, tid);
+                    corner(CX, CY, CX >= dxlo && CX <= dxhi && CY >= dylo && CY <= dyhi);
+                    bsearch = true;
+                }
+            }
+        }
+        if (!bsearch) {
         // ---- 2R x 2R main candidates (4 dx of one byte phase x 8 dy per thread) plus this
         //      thread's tail candidates, all in one row loop ----
         uint32_t acc[kTx][kTy];
@@ -521,7 +711,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const uint8_t* tp[G::kTailPer];
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) {
-            tp[t] = smem + tinfo[t][1 + (G::kPhaseSets == 1 ? 0 : s)][tid];
+            tp[t] = smem + tinfo[t][1 + s][tid];
             ta[t] = 0;
         }
         if (main_dead) {  // tails only (one LDS.128 of the current row, 4 LDS.32 + 4 SADs per tail)
@@ -590,20 +780,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
             }
         }
         PMARK(3);
-        if (warp == 0) {  // the corner candidate (R, R): 64 (row, word) pieces over warp 0
-            const uint32_t* rw = reinterpret_cast<const uint32_t*>(smem + s * G::kCopy + (2 * R) * win) + R / 2;
-            const uint4* cq4 = reinterpret_cast<const uint4*>(smem + G::kOffCur + s * 256);
-            uint32_t part = 0;
-#pragma unroll
-            for (int o = lane; o < 64; o += 32) {
-                const int v = o >> 2, k = o & 3;
-                const uint4 cv = cq4[v];
-                const uint32_t cw = k == 0 ? cv.x : k == 1 ? cv.y : k == 2 ? cv.z : cv.w;
-                part = sad4(rw[v * (win / 4) + k], cw, part);
-            }
-            const uint32_t tot = __reduce_add_sync(0xffffffffu, part);
-            if (lane == 0) lsum[s] = tot;
-        }
+        if (warp == 0) corner(R, R, A.unrestricted || (dxhi >= R && dyhi >= R));
         PMARK(4);
         if (!interior) {
 #pragma unroll
@@ -638,7 +815,6 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         }
         // ---- argmin: min over this thread's keys, key(j, i) = acc * kKeyMul + A_j + B_i,
         //      then one CREDUX per warp ----
-        uint32_t key = 0xffffffffu;
         {
             const uint4 a4 = tieA[p + 4 * g];
             const uint32_t Aj[4] = {a4.x, a4.y, a4.z, a4.w};
@@ -661,6 +837,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         }
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) key = min(key, ta[t] * kKeyMul + tinfo[t][0][tid]);
+        }  // (full-frame search)
         key = __reduce_min_sync(0xffffffffu, key);
         if (lane == 0) red32[s][warp] = key;
         PMARK(7);
@@ -963,6 +1140,27 @@ int me_search_impl(const uint8_t* ref, const uint8_t* cur, int64_t pitch, int32_
         a.nrows = (uint32_t)(rows * n_pairs);
         a.div_per_pair = make_fastdiv((uint32_t)(rows * mbx));
         a.div_mbx = make_fastdiv((uint32_t)mbx);
+        // class order with half-frame border searches (MeArgs::border_order): R = 16, whole
+        // restricted frames on the device, no surface, and enough macroblocks that the class
+        // phases are long against one macroblock per CTA (a single CIF pair, M2, keeps the
+        // plain order: one wave, where the border macroblocks are not on the critical path).
+        // $SP_ME_BORDER = 0 / 1 forces it off / on (whenever eligible) for tests and A/B runs.
+        if (range == 16 && !ready && !surface && pad == 0 && mb_row_begin == 0 && rows == mby && mbx >= 3 &&
+            mby >= 3) {
+            const char* e = std::getenv("SP_ME_BORDER");
+            const bool on = e && *e ? std::atoi(e) != 0 : total >= 8192;
+            if (on) {
+                const uint32_t P = (uint32_t)n_pairs, nI = (uint32_t)((mby - 2) * (mbx - 2));
+                a.border_order = 1;
+                a.cls_end[0] = P * nI;
+                a.cls_end[1] = a.cls_end[0] + P * 2u * (uint32_t)(mbx - 2);
+                a.cls_end[2] = a.cls_end[1] + P * 2u * (uint32_t)(mby - 2);
+                a.div_int = make_fastdiv(nI);
+                a.div_icols = make_fastdiv((uint32_t)(mbx - 2));
+                a.div_rows2 = make_fastdiv(2u * (uint32_t)(mbx - 2));
+                a.div_cols2 = make_fastdiv(2u * (uint32_t)(mby - 2));
+            }
+        }
         // (the streamed-frames variant is a separate instantiation: the flag wait in its move-in
         // costs the device-resident kernel its uniform-datapath index math, 2 % of M4)
         if (range == 32)

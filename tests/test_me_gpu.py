@@ -177,6 +177,61 @@ def test_border_macroblocks_without_surface(W, H, R, gen):
         assert np.array_equal(sad[p].reshape(-1), osad), p
 
 
+@pytest.mark.parametrize("W,H", [(352, 288), (96, 80), (48, 48), (100, 70), (129, 47), (64, 40), (360, 280)])
+@pytest.mark.parametrize("gen", ["seq", "flat"])
+@pytest.mark.parametrize("border", ["1", "0"])
+def test_class_order_border_search(W, H, gen, border, monkeypatch):
+    """R = 16 class order (interior macroblocks of every pair first, then rows, columns,
+    corners) with half-frame border searches, forced on ($SP_ME_BORDER=1) and off, against the
+    oracle on every macroblock of several pairs: sides multiples of 16 or not (then the last
+    row / column keeps the full search inside the border phase), 3 x 3 macroblock frames
+    (one interior macroblock), flat frames (ties across the moved tails and corner)."""
+    R = 16
+    monkeypatch.setenv("SP_ME_BORDER", border)
+    pitch = _pitch(W)
+    if gen == "seq":
+        fr = sp_inputs.me_sequence(6, W, H, R, seed=W * 7 + H, pitch=pitch)
+    else:
+        fr = np.zeros((6, H, pitch), np.uint8)
+        fr[0::2], fr[1::2] = 7, 200
+        fr[2] = 9
+    mv, sad, _ = _gpu(fr, W, H, R)
+    for p in range(5):
+        omv, osad, _ = _oracle_pair(fr, p, W, H, R, surface=False)
+        assert np.array_equal(mv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(sad[p].reshape(-1), osad), p
+
+
+@pytest.mark.parametrize("R", [16, 32])
+def test_many_macroblocks_per_cta_full_surface(R):
+    """More macroblocks than resident CTAs (8 CIF pairs at R = 16: 3,168 macroblocks on
+    2,368 one-warp CTAs; 40 pairs at R = 32), so CTAs run a second macroblock from the other
+    pipeline stage: every SAD of every candidate, tails included, equals the oracle.  (Until
+    round-2 session 3 the one-warp R = 16 kernel read byte-phase-0 tails from stage 0's window
+    on every macroblock; single-wave tests could not see it.)"""
+    W, H = 352, 288
+    P = 8 if R == 16 else 40
+    fr = sp_inputs.me_sequence(P + 1, W, H, R, seed=5 + R)
+    mv, sad, surf = _gpu(fr, W, H, R, with_surface=True)
+    for p in range(P):
+        omv, osad, osurf = _oracle_pair(fr, p, W, H, R)
+        assert np.array_equal(surf[p].reshape(osurf.shape), osurf), p
+        assert np.array_equal(mv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(sad[p].reshape(-1), osad), p
+
+
+def test_class_order_auto_many_pairs():
+    """The automatic class order (>= 8192 macroblocks: 24 CIF pairs) on the R = 16 throughput
+    form: every macroblock of every pair equals the oracle."""
+    W, H, R, P = 352, 288, 16, 24
+    fr = sp_inputs.me_sequence(P + 1, W, H, R, seed=77)
+    mv, sad, _ = _gpu(fr, W, H, R)
+    for p in range(P):
+        omv, osad, _ = _oracle_pair(fr, p, W, H, R, surface=False)
+        assert np.array_equal(mv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(sad[p].reshape(-1), osad), p
+
+
 def test_prepared_call_equals_oracle():
     """me_search_prepared (arguments marshalled once, the latency-config call form) runs the
     same entry point: repeated calls give the oracle's MVs / SADs."""

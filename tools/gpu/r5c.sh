@@ -1,0 +1,8 @@
+O=gpurun_out/r5c.txt
+for v in "" 0 1; do echo "== SP_ME_BORDER=$v" >> $O; SP_ME_BORDER=$v timeout 300 python tools/dbg_me16.py 64 >> $O 2>&1; done
+timeout 1200 python -m pytest tests/test_me_gpu.py tests/test_me_shard_gpu.py tests/test_me_host_gpu.py tests/test_me_stress_gpu.py tests/test_fuzz_gpu.py -x -q > gpurun_out/r5c_pytest_me.txt 2>&1; echo rc=$? >> gpurun_out/r5c_pytest_me.txt
+for rep in 1 2; do
+echo "== new, auto" >> $O; timeout 300 python tools/time_me_r16.py >> $O 2>&1
+echo "== new, SP_ME_BORDER=0" >> $O; SP_ME_BORDER=0 timeout 300 python tools/time_me_r16.py >> $O 2>&1
+echo "== M4 new" >> $O; timeout 300 python tools/quick_time.py --me-only >> $O 2>&1
+done
