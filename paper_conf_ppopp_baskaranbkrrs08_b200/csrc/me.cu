@@ -205,6 +205,7 @@ struct MeGeom {
     // 12.5 KB lets the register limit (16 CTAs) bind.
     static constexpr int kPhaseSets = kWarps == 1 ? 1 : 2;
     static constexpr int kSmem = kOffPh + 3 * kPhaseSets * kSlot + 128;  // + alignment slack
+    static_assert(kSlot * 3 < 65536 && kOffPh < 65536, "16-bit tail offsets (one-warp CTAs)");
     static_assert(kCopy % 128 == 0, "copies must keep 128-byte alignment");
     static_assert(kSlot >= kCopy + 3 * 32 && kSlot % 128 == 0, "phase copy slots must not overlap");
     static_assert(kWarps == 1 || kWarps == 2 || kWarps == 4, "tail mapping assumes 1, 2 or 4 warps");
@@ -268,8 +269,16 @@ __device__ __forceinline__ bool tail_slot(int warp, int lane, int t, int& k) {
 // Candidates dx = dx0 + p + 4 (TX g + j), dy = dy0 + TY d + i; column tails at dx = dx0 +
 // 4 TX kGx, row tails at dy = dy0 + TY kDy; invalid ones never enter the key.  Returns the
 // thread's minimal key.  (Out of line: the interior path keeps its registers and code layout.)
+#ifndef SP_ME_BINLINE
+#define SP_ME_BINLINE 0
+#endif
 template <int R, int TX, int TY>
-__device__ __noinline__ uint32_t border_search(const uint8_t* smem, int s, int dx0, int dy0, int dxlo, int dxhi,
+#if SP_ME_BINLINE
+__device__ __forceinline__
+#else
+__device__ __noinline__
+#endif
+uint32_t border_search(const uint8_t* smem, int s, int dx0, int dy0, int dxlo, int dxhi,
                                                int dylo, int dyhi, int tid) {
     using G = MeGeom<R>;
     static_assert(G::kWarps == 1, "border search: one-warp CTAs");
@@ -556,17 +565,24 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
     // tail candidates: tie bits and staged-copy offsets (stage 0, stage 1), per thread.  Two
     // offsets even with one phase-copy set: a tail of byte phase 0 reads the TMA'd window
     // itself, which alternates between the two stages (one-warp CTAs read stage 0's window on
-    // every macroblock until round-2 session 3 — wrong tails from a CTA's second macroblock on)
-    __shared__ uint32_t tinfo[G::kTailPer][3][G::kThreads];
+    // every macroblock until round-2 session 3 — wrong tails from a CTA's second macroblock on).
+    // One-warp CTAs pack the two 16-bit offsets into one word (shared memory holds them at 16
+    // CTAs per SM: 14,464 of the 14,592 bytes each may take)
+    constexpr bool kPackT = G::kPhaseSets == 1;
+    __shared__ uint32_t tinfo[G::kTailPer][kPackT ? 2 : 3][G::kThreads];
 #pragma unroll
     for (int t = 0; t < G::kTailPer; ++t) {
         int dxt, dyt;
         tail_candidate<R>(warp, lane, t, dxt, dyt);
         tinfo[t][0][tid] = tie_bits(dxt, dyt, R);
 #pragma unroll
-        for (int st = 0; st < 2; ++st)
-            tinfo[t][1 + st][tid] =
+        for (int st = 0; st < 2; ++st) {
+            const uint32_t off =
                 (uint32_t)(phase_copy(st, (dxt + R) & 3) - smem) + (dyt + R) * win + 4 * ((dxt + R) >> 2);
+            if (!kPackT) tinfo[t][1 + st][tid] = off;
+            else if (st == 0) tinfo[t][1][tid] = off;
+            else tinfo[t][1][tid] |= off << 16;
+        }
     }
     // macroblock index and position (pair, MB row, MB column) per stage, written by thread 0
     // one macroblock ahead (before the barrier that precedes their reading)
@@ -711,7 +727,7 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         const uint8_t* tp[G::kTailPer];
 #pragma unroll
         for (int t = 0; t < G::kTailPer; ++t) {
-            tp[t] = smem + tinfo[t][1 + s][tid];
+            tp[t] = smem + (kPackT ? (tinfo[t][1][tid] >> (16 * s)) & 0xffffu : tinfo[t][1 + s][tid]);
             ta[t] = 0;
         }
         if (main_dead) {  // tails only (one LDS.128 of the current row, 4 LDS.32 + 4 SADs per tail)
