@@ -31,6 +31,20 @@ def test_cif_sequence_vs_oracle(gen):
         assert np.array_equal(sad[p].reshape(-1), osad)
 
 
+def test_cif_many_pairs_multi_macroblock_ctas():
+    """R = 16 streamed-frames kernel with more macroblocks than resident CTAs (24 CIF pairs:
+    9,504 macroblocks on 2,368 one-warp CTAs), so CTAs alternate pipeline stages: every
+    macroblock equals the oracle."""
+    W, H, R, P = 352, 288, 16, 24
+    fr = sp_inputs.me_sequence(P + 1, W, H, R, seed=91)
+    mv, sad = sp.me_search(fr, W, H, R)
+    mv, sad = mv.numpy(), sad.numpy().view(np.uint32)
+    for p in range(P):
+        omv, osad, _ = oracle.me_search(fr[p], fr[p + 1], W, H, R)
+        assert np.array_equal(mv[p].reshape(-1, 2), omv), p
+        assert np.array_equal(sad[p].reshape(-1), osad), p
+
+
 def test_1080p_batch_equals_device_path_and_oracle_samples():
     W, H, R = 1920, 1080, 32
     fr = sp_inputs.me_sequence(9, W, H, R)
