@@ -490,8 +490,9 @@ def run_ours(args, rank, world, local_rank):
     if world == 1:
         a_pin = torch.from_numpy(sp_inputs.jacobi_input(n_local, seed=sp_inputs.JACOBI_BENCH_SEED)).pin_memory()
         f_pin = torch.from_numpy(frames_host).pin_memory()
-        # host-buffer Jacobi: the kernel reads a_pin and writes the result back over PCIe itself
-        # (sp_jacobi1d_host, wavefront order), in place: every call advances the state T steps
+        # host-buffer Jacobi (sp_jacobi1d_host, wavefront order): a_pin moves in by copy-engine
+        # chunks that release their pass-0 tiles, the last pass writes the result back over
+        # PCIe itself; in place: every call advances the state T steps
         # (same time tile as the device-resident run unless --e2e-time-tile says otherwise)
         tt_e2e = args.e2e_time_tile or tt
         jac_host = sp.Jacobi1DHost(n_local, T, tt_e2e)
@@ -516,7 +517,7 @@ def run_ours(args, rank, world, local_rank):
         # Jacobi's own bytes: the state read from and written back to pinned host memory
         e2e = {"value": (n_local - 2) * T * ke / tj / 1e9, "unit": "GPoint-updates/s",
                "h2d_bytes_per_step": 4 * n_local, "d2h_bytes_per_step": 4 * n_local,
-               "api": "sp_jacobi1d_host (kernel move-in/out over PCIe, wavefront order)", "time_tile": tt_e2e}
+               "api": "sp_jacobi1d_host (input: copy-engine chunks into device memory, each releasing its pass-0 tiles; output: the last pass TMA-stores into the pinned array; wavefront order)", "time_tile": tt_e2e}
         me_e2e = {"value": me_valid_sads(ME_W, ME_H, ME_R, ME_PAIRS) * ke / tm / 1e9, "unit": "GSAD/s",
                   "h2d_bytes_per_step": frames_host.nbytes, "d2h_bytes_per_step": ME_PAIRS * mby * mbx * 8,
                   "api": "sp_me_search_host (per-frame H2D overlapped with the search, outputs stored to pinned host)"}

@@ -254,13 +254,24 @@ int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float
                                  int32_t space_tile, int64_t skew, int64_t* footprint_log, void* stream);
 
 /* End-to-end host-buffer call (the public API behind `e2e`): a_host[n] is PAGE-LOCKED host
- * memory holding a^(0); on completion (stream-ordered) it holds a^(steps).  The input is
- * read and the result written by the kernel's own move-in / move-out over PCIe, in the
- * wavefront order of sp_jacobi1d_timetiled_stream (no separate H2D / D2H copies, no
- * device copy of the whole array beyond buf0/buf1).  buf0, buf1, flags as above.
+ * memory holding a^(0); on completion (stream-ordered) it holds a^(steps).  The result is
+ * written by the kernel's own last-pass move-out over PCIe (TMA bulk stores into a_host), in
+ * the wavefront order of sp_jacobi1d_timetiled_stream.  The input:
+ *   flags_len >= sp_jacobi1d_host_flags_len(): moved in by the copy engine — chunks of
+ *     SP_JACOBI_HOST_CHUNK cells copied into buf0 on a library-owned side stream while the
+ *     kernel already runs, each followed by a ready flag (flags[tiles + 1 + chunk]) that
+ *     releases the pass-0 tiles it feeds (the caller's stream waits for the copies before
+ *     it completes);
+ *   flags_len >= sp_jacobi1d_plan().persistent_tiles + 1 only: read by pass 0's own TMA
+ *     move-in straight from a_host.
+ * buf0, buf1 as above (distinct device buffers of n cells, contents clobbered).
  * Errors: SP_ERR_INVALID_ARG for pageable or misaligned a_host. */
+#define SP_JACOBI_HOST_CHUNK (1 << 21) /* cells per copy-engine input chunk (8 MiB) */
 int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t* flags, int64_t flags_len, int64_t n,
                      int32_t steps, int32_t time_tile, int32_t space_tile, void* stream);
+/* flags_len that selects the copy-engine input of sp_jacobi1d_host (host-only): persistent
+ * tiles + 1 + ceil(n / SP_JACOBI_HOST_CHUNK).  Errors: SP_ERR_INVALID_ARG. */
+int sp_jacobi1d_host_flags_len(int64_t n, int32_t steps, int32_t time_tile, int32_t space_tile, int64_t* flags_len);
 
 /* Cluster-resident form for small domains (the paper's "fits in the scratchpad" regime,
  * P:L964-1052, Figs. 5 and 7): the whole array is moved in once into the registers of ONE

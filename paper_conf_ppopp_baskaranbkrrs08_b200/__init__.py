@@ -153,6 +153,7 @@ SYMBOLS = {
     "sp_jacobi1d_timetiled_fused": (ctypes.c_int, [vp, vp, vp, i64, i64, i32, i32, i32, vp, vp]),
     "sp_jacobi1d_timetiled_stream": (ctypes.c_int, [vp, vp, vp, vp, vp, i64, i64, i32, i32, i32, i64, vp, vp]),
     "sp_jacobi1d_host": (ctypes.c_int, [vp, vp, vp, vp, i64, i64, i32, i32, i32, vp]),
+    "sp_jacobi1d_host_flags_len": (ctypes.c_int, [i64, i32, i32, i32, ctypes.POINTER(i64)]),
     "sp_jacobi1d_resident_capacity": (ctypes.c_int, [ctypes.POINTER(i64)]),
     "sp_jacobi1d_resident": (ctypes.c_int, [vp, vp, i64, i32, vp]),
     "sp_me_sad_search": (ctypes.c_int, [vp, vp, i64, i32, i32, i32, i32, i32, i64, i32, i32, i32, i32, vp, vp, vp, vp]),
@@ -487,17 +488,29 @@ def jacobi1d_resident(inp, steps: int, out=None, stream=None):
     return out
 
 
+def jacobi1d_host_flags_len(n: int, steps: int, time_tile: int = 64, space_tile: int = 0) -> int:
+    """flags length that selects sp_jacobi1d_host's copy-engine input (host-only)."""
+    c = i64()
+    _check(lib.sp_jacobi1d_host_flags_len(int(n), int(steps), int(time_tile), int(space_tile), ctypes.byref(c)),
+           "sp_jacobi1d_host_flags_len")
+    return c.value
+
+
 class Jacobi1DHost:
     """Reusable device scratch for the end-to-end host-buffer call (sp_jacobi1d_host): two
-    n-cell device buffers and the completion flags, allocated once."""
+    n-cell device buffers and the completion / input-ready flags, allocated once.
+    direct_input=True sizes the flags for pass 0's own PCIe reads of the host array instead
+    of the copy-engine input (the round-2 form; A/B and tests)."""
 
-    def __init__(self, n: int, steps: int, time_tile: int = 64, space_tile: int = 0, device="cuda"):
+    def __init__(self, n: int, steps: int, time_tile: int = 64, space_tile: int = 0, device="cuda",
+                 direct_input: bool = False):
         import torch
         self.n, self.steps, self.time_tile, self.space_tile = n, steps, time_tile, space_tile
         self.buf0 = torch.empty(n, dtype=torch.float32, device=device)
         self.buf1 = torch.empty(n, dtype=torch.float32, device=device)
-        self.flags = torch.empty(jacobi1d_plan(n, steps, time_tile, space_tile)["tiles"] + 1, dtype=torch.int32,
-                                 device=device)
+        nf = (jacobi1d_plan(n, steps, time_tile, space_tile)["persistent_tiles"] + 1 if direct_input
+              else jacobi1d_host_flags_len(n, steps, time_tile, space_tile))
+        self.flags = torch.empty(nf, dtype=torch.int32, device=device)
 
     def run(self, a_pinned, stream=None):
         """In place on a PINNED CPU float32 tensor: a_pinned <- J^steps(a_pinned) (stream-ordered;

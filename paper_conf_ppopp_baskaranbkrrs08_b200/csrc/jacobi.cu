@@ -143,6 +143,12 @@ struct PassArgs {
     float* pushR[2];
     int* edge_cnt;  // [2][passes]
     int32_t nE_left, nE_right;
+    // Host-buffer input by the copy engine (sp_jacobi1d_host; kHostOutPass only, null
+    // otherwise): in0 is a device buffer that copies on a side stream fill in chunks of
+    // in_chunk cells, each followed by in_ready[chunk] = 1; a pass-0 tile's move-in waits for
+    // the chunks its footprint touches (relaxed poll, then acquire + proxy fence).
+    const int* in_ready;
+    int64_t in_chunk;
 };
 
 // Spin (acquire, system scope) until *flag >= e.  A peer that never arrives (crashed rank,
@@ -643,6 +649,15 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
         if constexpr (kPeer) {
             if (pers && !peer_ready(t, pass)) return false;
         }
+        if constexpr (kMode == kHostOutPass) {
+            if (pers && pass == 0 && A.in_ready) {  // its input chunks have arrived
+                int64_t x0, st, lo, hi;
+                tile_range(t, x0, st, lo, hi);
+                const int64_t c0 = lo / A.in_chunk, c1 = (hi - 1) / A.in_chunk;  // (c1 - c0 < 32: host-checked)
+                const bool ok = c0 + lane > c1 || ld_relaxed_gpu(A.in_ready + c0 + lane) != 0;
+                return __all_sync(0xffffffffu, ok);
+            }
+        }
         if (!pers || pass == 0 || (SP_JAC_TIMING & 1)) return true;
         bool ok = true;
         for (int64_t q0 = t - reach; q0 <= t + reach; q0 += 32) {
@@ -672,7 +687,7 @@ __global__ void __launch_bounds__(Cfg::kThreads, Cfg::kMinBlocks) jacobi1d_pass_
             // the dependence flags were observed by relaxed loads (cheap polling); one
             // acquire fence per tile turns that observation into synchronisation with the
             // producers' release stores before the move-in reads their cells
-            if (pass > 0) fence_acq_rel_gpu();
+            if (pass > 0 || (kMode == kHostOutPass && A.in_ready)) fence_acq_rel_gpu();
 #endif
             fence_proxy_async_global();  // observed flags -> the async-proxy read below
         }
@@ -1489,10 +1504,12 @@ int device_view(const void* p, const void** out, bool* host = nullptr) {
 }
 }  // namespace
 
-extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float* buf1, int32_t* flags,
-                                            int64_t flags_len, int64_t n, int32_t steps, int32_t time_tile,
-                                            int32_t space_tile, int64_t skew, int64_t* footprint_log, void* stream) {
-    SP_NVTX("sp_jacobi1d_timetiled_stream");
+namespace {
+// sp_jacobi1d_timetiled_stream; in_ready / in_chunk: PassArgs (host-buffer input by the copy
+// engine; then the launch must be the kHostOutPass instantiation, else SP_ERR_UNSUPPORTED)
+int stream_impl(const float* in, float* out, float* buf0, float* buf1, int32_t* flags, int64_t flags_len, int64_t n,
+                int32_t steps, int32_t time_tile, int32_t space_tile, int64_t skew, int64_t* footprint_log,
+                void* stream, const int* in_ready = nullptr, int64_t in_chunk = 0) {
     if (!in || !out || !buf0 || !buf1 || !flags || n < 3 || steps < 0 || buf0 == buf1 || in == buf1)
         return SP_ERR_INVALID_ARG;
     for (const void* q : {(const void*)in, (const void*)out, (const void*)buf0, (const void*)buf1})
@@ -1542,10 +1559,25 @@ extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* 
                nullptr, nullptr, nullptr, nullptr, nullptr, nullptr, 0ull, nullptr, nullptr,
                flags, {buf0, buf1}, passes, steps, time_tile, din, redirect ? nullptr : const_cast<float*>(dout), skew};
     // host output written by the in-place kernel: its staged-move-out instantiation
-    if ((st = launch_pass(p, s, di, hout && !redirect && di.kernel_host ? kHostOutPass : kPlainPass))) return st;
+    const int mode = hout && !redirect && di.kernel_host ? kHostOutPass : kPlainPass;
+    if (in_ready) {
+        if (mode != kHostOutPass || in_chunk < 4096) return SP_ERR_UNSUPPORTED;
+        p.in_ready = in_ready;
+        p.in_chunk = in_chunk;
+    }
+    if ((st = launch_pass(p, s, di, mode))) return st;
     if (redirect)
         SP_CUDA_TRY(cudaMemcpyAsync(out, bufs[passes & 1], (size_t)n * sizeof(float), cudaMemcpyDefault, s));
     return SP_OK;
+}
+}  // namespace
+
+extern "C" int sp_jacobi1d_timetiled_stream(const float* in, float* out, float* buf0, float* buf1, int32_t* flags,
+                                            int64_t flags_len, int64_t n, int32_t steps, int32_t time_tile,
+                                            int32_t space_tile, int64_t skew, int64_t* footprint_log, void* stream) {
+    SP_NVTX("sp_jacobi1d_timetiled_stream");
+    return stream_impl(in, out, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile, skew, footprint_log,
+                       stream);
 }
 
 extern "C" int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags, int64_t flags_len, int64_t n,
@@ -1568,14 +1600,100 @@ extern "C" int sp_jacobi1d_timetiled_fused(float* a, float* work, int32_t* flags
                                         footprint_log, stream);
 }
 
+namespace {
+const int32_t* jac_pinned_one() {  // the value the copy stream writes into a ready flag
+    static int32_t* one = nullptr;
+    static std::once_flag once;
+    std::call_once(once, [] {
+        void* p = nullptr;
+        if (cudaHostAlloc(&p, 64, cudaHostAllocPortable) == cudaSuccess) {
+            one = static_cast<int32_t*>(p);
+            *one = 1;
+        }
+    });
+    return one;
+}
+cudaStream_t jac_copy_stream() {  // per device (the current one)
+    static std::mutex mu;
+    static cudaStream_t cs[64] = {};
+    int dev = 0;
+    if (cudaGetDevice(&dev) != cudaSuccess || dev < 0 || dev >= 64) return nullptr;
+    std::lock_guard<std::mutex> lk(mu);
+    if (!cs[dev] && cudaStreamCreateWithFlags(&cs[dev], cudaStreamNonBlocking) != cudaSuccess) cs[dev] = nullptr;
+    return cs[dev];
+}
+}  // namespace
+
+extern "C" int sp_jacobi1d_host_flags_len(int64_t n, int32_t steps, int32_t time_tile, int32_t space_tile,
+                                          int64_t* flags_len) {
+    if (!flags_len || n < 3 || steps < 0) return SP_ERR_INVALID_ARG;
+    int64_t S;
+    int32_t wo;
+    int st = geometry(time_tile, space_tile, S, wo, persistent_variant_index(time_tile));
+    if (st) return st;
+    *flags_len = (n + S - 1) / S + 1 + (n + SP_JACOBI_HOST_CHUNK - 1) / SP_JACOBI_HOST_CHUNK;
+    return SP_OK;
+}
+
 extern "C" int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t* flags, int64_t flags_len, int64_t n,
                                 int32_t steps, int32_t time_tile, int32_t space_tile, void* stream) {
-    if (!a_host) return SP_ERR_INVALID_ARG;
+    SP_NVTX("sp_jacobi1d_host");
+    if (!a_host || !buf0 || !flags || n < 3 || steps < 0) return SP_ERR_INVALID_ARG;
     cudaPointerAttributes at;
     SP_CUDA_TRY(cudaPointerGetAttributes(&at, a_host));
     if (at.type != cudaMemoryTypeHost) return SP_ERR_INVALID_ARG;  // page-locked host memory only
-    return sp_jacobi1d_timetiled_stream(a_host, a_host, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile,
-                                        -1, nullptr, stream);
+    // Copy-engine input (flags_len covers the ready flags, the launch is the in-place kernel's
+    // host-output instantiation): the state moves in chunk by chunk through cudaMemcpyAsync on
+    // a side stream into buf0 while the kernel already runs — the copy engine streams at
+    // ~55 GB/s where the kernel's own TMA reads of host memory reach ~40-51 — and each chunk's
+    // ready flag releases the pass-0 tiles it feeds.  Otherwise pass 0 reads a_host directly.
+    const int vi = persistent_variant_index(time_tile);
+    int64_t S;
+    int32_t wo;
+    int st = geometry(time_tile, space_tile, S, wo, vi);
+    if (st) return st;
+    const int64_t tiles = (n + S - 1) / S, chunks = (n + SP_JACOBI_HOST_CHUNK - 1) / SP_JACOBI_HOST_CHUNK;
+    Variant di;
+    if ((st = device_info(di, vi))) return st;
+    static const bool direct = [] {  // SP_JACOBI_HOST_DIRECT=1: always the kernel's own PCIe reads (A/B)
+        const char* e = std::getenv("SP_JACOBI_HOST_DIRECT");
+        return e && std::atoi(e) != 0;
+    }();
+    if (direct || steps == 0 || flags_len < tiles + 1 + chunks || !di.kernel_host || buf0 == a_host)
+        return stream_impl(a_host, a_host, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile, -1, nullptr,
+                           stream);
+    const int32_t* one = jac_pinned_one();
+    const cudaStream_t cs = jac_copy_stream(), s = (cudaStream_t)stream;
+    if (!one || !cs) {
+        sp::set_cuda_error((int)cudaErrorMemoryAllocation);
+        return SP_ERR_CUDA;
+    }
+    int32_t* ready = flags + tiles + 1;
+    cudaEvent_t ev0, ev1;
+    SP_CUDA_TRY(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming));
+    SP_CUDA_TRY(cudaEventCreateWithFlags(&ev1, cudaEventDisableTiming));
+    // ready flags cleared, and the caller's earlier work on a_host / buf0 complete, before
+    // the copies start; the kernel is launched before the copies are enqueued (it waits for
+    // them on the device), so the host-side enqueue overlaps the run
+    SP_CUDA_TRY(cudaMemsetAsync(ready, 0, (size_t)chunks * sizeof(int32_t), s));
+    SP_CUDA_TRY(cudaEventRecord(ev0, s));
+    SP_CUDA_TRY(cudaStreamWaitEvent(cs, ev0, 0));
+    st = stream_impl(buf0, a_host, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile, -1, nullptr, stream,
+                     ready, SP_JACOBI_HOST_CHUNK);
+    if (!st) {
+        for (int64_t c = 0; c < chunks; ++c) {
+            const int64_t c0 = c * SP_JACOBI_HOST_CHUNK;
+            const int64_t len = n - c0 < SP_JACOBI_HOST_CHUNK ? n - c0 : SP_JACOBI_HOST_CHUNK;
+            SP_CUDA_TRY(cudaMemcpyAsync(buf0 + c0, a_host + c0, (size_t)len * sizeof(float), cudaMemcpyHostToDevice, cs));
+            SP_CUDA_TRY(cudaMemcpyAsync(ready + c, one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
+        }
+    }
+    SP_CUDA_TRY(cudaEventRecord(ev1, cs));
+    // the caller's stream completes only after the copies did (buf0 / flags reusable)
+    SP_CUDA_TRY(cudaStreamWaitEvent(s, ev1, 0));
+    cudaEventDestroy(ev0);
+    cudaEventDestroy(ev1);
+    return st;
 }
 
 __global__ void peer_done_kernel(unsigned long long* left_done, unsigned long long* right_done, unsigned long long e) {

@@ -70,10 +70,13 @@ def test_in_place_aliasing(steps):
             _check(_stream(a, steps, 16, 0, skew, where, same=True), want)
 
 
-def test_host_class_reuse_and_public_call():
+@pytest.mark.parametrize("direct", [False, True])
+def test_host_class_reuse_and_public_call(direct):
+    """copy-engine input (chunks + ready flags) and the direct PCIe move-in; a second call on
+    the same flags and buffers continues from the first one's result"""
     n, steps, tt = 300007, 200, 64
     a = sp_inputs.jacobi_input(n, seed=5)
-    ctx = sp.Jacobi1DHost(n, steps, tt)
+    ctx = sp.Jacobi1DHost(n, steps, tt, direct_input=direct)
     h = torch.from_numpy(a.copy()).pin_memory()
     ctx.run(h)
     ctx.run(h)  # flags reused, state carried on: 2 * steps in total
@@ -113,15 +116,15 @@ def test_footprint_log_under_wavefront_order():
             assert (lg[p, t, 0], lg[p, t, 1]) == (lb, ub)
 
 
-@pytest.mark.parametrize("tt", [64, 128])
-def test_J3_size_host_path_sampled(tt):
+@pytest.mark.parametrize("tt,direct", [(64, False), (128, False), (128, True)])
+def test_J3_size_host_path_sampled(tt, direct):
     """the bench's e2e call at full size: 2^26 cells, T = 1024, pinned host in/out (Tt = 128 is
     the bench's; the in-place kernel's host-output instantiation stages the last pass's
     move-out), samples around the persistent geometry's tile boundaries"""
     n, steps = 1 << 26, 1024
     a = sp_inputs.jacobi_input(n, seed=2008)
     h = torch.from_numpy(a.copy()).pin_memory()
-    sp.Jacobi1DHost(n, steps, tt).run(h)
+    sp.Jacobi1DHost(n, steps, tt, direct_input=direct).run(h)
     torch.cuda.synchronize()
     got = h.numpy()
     S = sp.jacobi1d_plan(n, steps, tt, 0)["persistent_space_tile"]
@@ -133,3 +136,18 @@ def test_J3_size_host_path_sampled(tt):
                 idx.append(t * S + off)
     idx = np.unique(np.array(idx + rng.integers(0, n, 40).tolist(), dtype=np.int64))
     _check(got[idx], oracle.jacobi1d_points(a, steps, idx))
+
+
+@pytest.mark.parametrize("n", [3, 4099, (1 << 21) - 5, (1 << 21) + 7, 3 * (1 << 21) + 1000])
+@pytest.mark.parametrize("tt", [48, 64, 128])
+def test_host_copy_engine_chunks(n, tt):
+    """copy-engine input across chunk boundaries (SP_JACOBI_HOST_CHUNK = 2^21 cells): one
+    chunk, a chunk plus a few cells, several chunks; every cell equals the oracle"""
+    steps = 2 * tt + 5
+    a = sp_inputs.jacobi_input(n, seed=n % 97 + tt)
+    h = torch.from_numpy(a.copy()).pin_memory()
+    ctx = sp.Jacobi1DHost(n, steps, tt)
+    assert ctx.flags.numel() > sp.jacobi1d_plan(n, steps, tt, 0)["persistent_tiles"] + 1
+    ctx.run(h)
+    torch.cuda.synchronize()
+    _check(h, oracle.jacobi1d(a, steps))
