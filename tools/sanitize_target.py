@@ -75,6 +75,16 @@ mark("sp.me_search_sequence (CIF +-32: 4-warp CTAs, two stages per CTA)")
 sp.me_search_sequence(fr3, 352, 288, 32)
 mark("sp.me_search_host (CIF +-32, streamed)")
 sp.MESearchHost(2, 352, 288, fr3.shape[2], 32).run(fr3.cpu().pin_memory())
+mark("sp.me_search_sequence (R = 16 class order with half-frame border searches, 4 CTAs)")
+os.environ["SP_ME_BORDER"] = "1"
+sp.me_search_sequence(fr, 352, 288, 16)
+os.environ["SP_ME_BORDER"] = "0"
+mark("sp.me_search_sequence (R = 16 plain order, 4 CTAs: both stages, byte-phase-0 tails)")
+sp.me_search_sequence(fr, 352, 288, 16)
+del os.environ["SP_ME_BORDER"]
+mark("sp.jacobi1d_host (direct PCIe move-in)")
+hd = torch.from_numpy(sp_inputs.jacobi_input(4099, seed=3)).pin_memory()
+sp.Jacobi1DHost(4099, 150, 64, 0, direct_input=True).run(hd)
 mark("sp.me_sad_search_range (flat range splitting a pair, R = 16 and 32)")
 sp.me_sad_search_range(fr, 352, 288, 16, 7, 29)
 sp.me_sad_search_range(fr3, 352, 288, 32, 3, 11)
