@@ -457,9 +457,16 @@ me_sad_kernel(const __grid_constant__ CUtensorMap ref_map, const __grid_constant
         return Pos{(int)pair, (int)byr, (int)(rem - byr * mbx)};
 #endif
     };
+    // (kStream, thread 0) highest pair seen ready: the copies land in frame order and a CTA's
+    // macroblocks come in increasing pair order, so each pair's flag is polled (and fenced)
+    // once per CTA instead of once per macroblock
+    int ready_seen = -1;
     auto issue = [&](uint32_t mb, int st) {  // single thread: stage the window + cur of mb
         const Pos q = locate(mb);
-        if (kStream) wait_ready(A.ready + q.pair);
+        if (kStream && q.pair > ready_seen) {
+            wait_ready(A.ready + q.pair);
+            ready_seen = q.pair;
+        }
         const int x0 = kMB * q.bx, y0 = kMB * (A.mb_row_begin + q.byr);
         mbar_arrive_expect_tx(&full[st], (uint32_t)(G::kCopy + kMB * kMB));
         tma_load_3d(smem + st * G::kCopy, &ref_map, x0 - R + A.pad, y0 - R - A.row0 + A.pad, q.pair - A.pair_base,
@@ -1417,14 +1424,19 @@ extern "C" int sp_me_search_host(const uint8_t* frames_host, int64_t pitch, int3
     SP_CUDA_TRY(cudaMemsetAsync(ready, 0, (size_t)pairs * sizeof(int32_t), s));
     SP_CUDA_TRY(cudaEventRecord(ev0, s));
     SP_CUDA_TRY(cudaStreamWaitEvent(cs, ev0, 0));
-    for (int32_t f = 0; f < n_frames; ++f) {
-        SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f * fbytes, frames_host + f * fbytes, fbytes, cudaMemcpyHostToDevice, cs));
-        if (f >= 1) SP_CUDA_TRY(cudaMemcpyAsync(ready + (f - 1), one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
-    }
-    SP_CUDA_TRY(cudaEventRecord(ev1, cs));
+    // the search is launched first (its move-ins wait for the ready flags on the device), so
+    // enqueueing the 2 x n_frames copies on the host overlaps the run instead of delaying it
     st = me_search_impl(frames_dev, frames_dev + fbytes, pitch, width, height, 0, height, pairs, (int64_t)fbytes, kMB,
                         range, 0, height / kMB, static_cast<int16_t*>(dmv), static_cast<uint32_t*>(dsad), nullptr,
                         stream, 0, ready);
+    if (!st) {
+        for (int32_t f = 0; f < n_frames; ++f) {
+            SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f * fbytes, frames_host + f * fbytes, fbytes,
+                                        cudaMemcpyHostToDevice, cs));
+            if (f >= 1) SP_CUDA_TRY(cudaMemcpyAsync(ready + (f - 1), one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
+        }
+    }
+    SP_CUDA_TRY(cudaEventRecord(ev1, cs));
     // the caller's stream completes only after the copies did (frames_dev / ready reusable)
     SP_CUDA_TRY(cudaStreamWaitEvent(s, ev1, 0));
     cudaEventDestroy(ev0);
