@@ -375,6 +375,42 @@ __device__ __forceinline__ void run_steps_fx(uint64_t (&P)[kK], int h, int lane,
     }
 }
 
+// Select form of the Dirichlet restore (the cluster-resident kernel's boundary warps): a lane
+// holds at most one fixed cell per component (jlo / jhi: its pair index, -1 if none), and each
+// pair is patched right after its update — edge pairs before their shuffles, so the neighbours
+// never see a stale value and no second shuffle round is needed.  Branch-free: the jump-table
+// restore's lane-divergent cases made the compiler emulate the shuffles collectively
+// (WARPSYNC.COLLECTIVE), which doubled the boundary warps' step time (ncu r5q).
+__device__ __forceinline__ uint64_t fix_sel(uint64_t q, int j, int jlo, int jhi, float vlo, float vhi) {
+    return f2_pack(j == jlo ? vlo : f2_lo(q), j == jhi ? vhi : f2_hi(q));
+}
+template <int kK>
+__device__ __forceinline__ void step_sel(const uint64_t (&P)[kK], uint64_t (&Q)[kK], uint64_t& left, uint64_t& right,
+                                         int lane, uint64_t w2, uint64_t mz, int jlo, int jhi, float vlo, float vhi) {
+    Q[0] = fix_sel(update(left, P[0], P[1], w2, mz), 0, jlo, jhi, vlo, vhi);
+    Q[kK - 1] = fix_sel(update(P[kK - 2], P[kK - 1], right, w2, mz), kK - 1, jlo, jhi, vlo, vhi);
+    neighbours<kK>(Q[0], Q[kK - 1], lane, left, right);
+#pragma unroll
+    for (int j = 1; j < kK - 1; ++j) Q[j] = fix_sel(update(P[j - 1], P[j], P[j + 1], w2, mz), j, jlo, jhi, vlo, vhi);
+}
+template <int kK>
+__device__ __forceinline__ void run_steps_sel(uint64_t (&P)[kK], int h, int lane, uint64_t w2, uint64_t mz, int jlo,
+                                              int jhi, float vlo, float vhi) {
+    uint64_t Q[kK];
+    uint64_t left, right;
+    neighbours<kK>(P[0], P[kK - 1], lane, left, right);
+    int k = 0;
+    for (; k + 2 <= h; k += 2) {
+        step_sel(P, Q, left, right, lane, w2, mz, jlo, jhi, vlo, vhi);
+        step_sel(Q, P, left, right, lane, w2, mz, jlo, jhi, vlo, vhi);
+    }
+    if (k < h) {
+        step_sel(P, Q, left, right, lane, w2, mz, jlo, jhi, vlo, vhi);
+#pragma unroll
+        for (int j = 0; j < kK; ++j) P[j] = Q[j];
+    }
+}
+
 // ---- in-place sweeps (JCfg kInPlace) ------------------------------------------------------
 // K pairs live in K + 1 registers R[0..K].  Before an ascending sweep element j is in R[j + 1];
 // the sweep computes new element j from old j - 1 (R[j]), j (R[j + 1]) and j + 1 (R[j + 2]) and
@@ -1311,8 +1347,38 @@ __global__ void __launch_bounds__(32 * kWarps, 1)
         const int64_t cu = base + lane * kK + j, cv = base + 32 * kK + lane * kK + j;
         P[j] = f2_pack(cu >= 0 && cu < n ? src[cu] : 0.f, cv >= 0 && cv < n ? src[cv] : 0.f);
     }
-    const bool boundary = (base <= 0 && 0 < base + kStrip) || (base <= n - 1 && n - 1 < base + kStrip);
+#ifndef SP_RES_NOFIX  // (timing-only build knob: no Dirichlet restore — wrong results)
+#define SP_RES_NOFIX 0
+#endif
+#ifndef SP_RES_JUMP  // (A/B build knob: the jump-table restore in every boundary warp)
+#define SP_RES_JUMP 0
+#endif
+    const bool boundary = !SP_RES_NOFIX && ((base <= 0 && 0 < base + kStrip) || (base <= n - 1 && n - 1 < base + kStrip));
     const FixedCells fc = boundary ? fixed_cells<kK>(base, n, src[0], src[n - 1]) : FixedCells{-1, -1, 0.f, 0.f, false};
+    // this lane's fixed cells for the select-form restore; both in one lane's same component
+    // (n < K - E + 1: tiny domains) keeps the jump-table form
+    int jlo = -1, jhi = -1;
+    float vlo = 0.f, vhi = 0.f;
+    // (the small shape only: with K = 28 the per-pair selects cost more than the jump table's
+    //  divergence — r5r: N = 8,064 2.41 vs 1.43 ms at T = 4,096; small shape 0.90 vs 1.13 ms)
+    bool sel = boundary && !SP_RES_JUMP && kK <= 12;
+    if (sel) {
+        const int f[2] = {fc.fx0, fc.fx1};
+        const float fv[2] = {fc.v0, fc.v1};
+        if (f[0] >= 0 && f[1] >= 0 && (f[0] >> 8) == (f[1] >> 8)) sel = false;  // same lane, same component
+#pragma unroll
+        for (int i = 0; i < 2; ++i)
+            if (f[i] >= 0 && lane == (f[i] >> 9)) {
+                if ((f[i] >> 8) & 1) {
+                    jhi = f[i] & 255;
+                    vhi = fv[i];
+                } else {
+                    jlo = f[i] & 255;
+                    vlo = fv[i];
+                }
+            }
+        sel = __all_sync(0xffffffffu, sel);  // (warp-uniform anyway: fx0 / fx1 are)
+    }
     // a one-CTA cluster synchronises with the CTA barrier (no neighbour CTA to order against):
     // J1 20.3 vs 22.4 us per call under graph replay, ~275 vs ~305 ns per step (r5i)
     const bool one = gridDim.x == 1;
@@ -1324,7 +1390,8 @@ __global__ void __launch_bounds__(32 * kWarps, 1)
     int q = 0;
     for (int done = 0; done < steps; done += kE) {
         const int h = steps - done < kE ? steps - done : kE;
-        if (boundary) run_steps_fx<true>(P, h, lane, w2, mz, fc);
+        if (sel) run_steps_sel<kK>(P, h, lane, w2, mz, jlo, jhi, vlo, vhi);
+        else if (boundary) run_steps_fx<true>(P, h, lane, w2, mz, fc);
         else run_steps_fx<false>(P, h, lane, w2, mz, fc);
         if (done + h >= steps) break;
         // exchange: edges out (strip cells [E, 2E) and [64K-2E, 64K-E)), barrier, halos in
