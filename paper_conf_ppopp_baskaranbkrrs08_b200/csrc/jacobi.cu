@@ -1740,22 +1740,21 @@ extern "C" int sp_jacobi1d_host(float* a_host, float* buf0, float* buf1, int32_t
     SP_CUDA_TRY(cudaEventCreateWithFlags(&ev0, cudaEventDisableTiming));
     SP_CUDA_TRY(cudaEventCreateWithFlags(&ev1, cudaEventDisableTiming));
     // ready flags cleared, and the caller's earlier work on a_host / buf0 complete, before
-    // the copies start; the kernel is launched before the copies are enqueued (it waits for
-    // them on the device), so the host-side enqueue overlaps the run
+    // the copies start.  The copies are enqueued BEFORE the kernel: it spins on their flags,
+    // so under a serialising tool (ncu, CUDA_LAUNCH_BLOCKING=1) copies enqueued after the
+    // launch would never run and the kernel would trap (found with ncu in session 3).
     SP_CUDA_TRY(cudaMemsetAsync(ready, 0, (size_t)chunks * sizeof(int32_t), s));
     SP_CUDA_TRY(cudaEventRecord(ev0, s));
     SP_CUDA_TRY(cudaStreamWaitEvent(cs, ev0, 0));
-    st = stream_impl(buf0, a_host, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile, -1, nullptr, stream,
-                     ready, SP_JACOBI_HOST_CHUNK);
-    if (!st) {
-        for (int64_t c = 0; c < chunks; ++c) {
-            const int64_t c0 = c * SP_JACOBI_HOST_CHUNK;
-            const int64_t len = n - c0 < SP_JACOBI_HOST_CHUNK ? n - c0 : SP_JACOBI_HOST_CHUNK;
-            SP_CUDA_TRY(cudaMemcpyAsync(buf0 + c0, a_host + c0, (size_t)len * sizeof(float), cudaMemcpyHostToDevice, cs));
-            SP_CUDA_TRY(cudaMemcpyAsync(ready + c, one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
-        }
+    for (int64_t c = 0; c < chunks; ++c) {
+        const int64_t c0 = c * SP_JACOBI_HOST_CHUNK;
+        const int64_t len = n - c0 < SP_JACOBI_HOST_CHUNK ? n - c0 : SP_JACOBI_HOST_CHUNK;
+        SP_CUDA_TRY(cudaMemcpyAsync(buf0 + c0, a_host + c0, (size_t)len * sizeof(float), cudaMemcpyHostToDevice, cs));
+        SP_CUDA_TRY(cudaMemcpyAsync(ready + c, one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
     }
     SP_CUDA_TRY(cudaEventRecord(ev1, cs));
+    st = stream_impl(buf0, a_host, buf0, buf1, flags, flags_len, n, steps, time_tile, space_tile, -1, nullptr, stream,
+                     ready, SP_JACOBI_HOST_CHUNK);
     // the caller's stream completes only after the copies did (buf0 / flags reusable)
     SP_CUDA_TRY(cudaStreamWaitEvent(s, ev1, 0));
     cudaEventDestroy(ev0);

@@ -1424,19 +1424,18 @@ extern "C" int sp_me_search_host(const uint8_t* frames_host, int64_t pitch, int3
     SP_CUDA_TRY(cudaMemsetAsync(ready, 0, (size_t)pairs * sizeof(int32_t), s));
     SP_CUDA_TRY(cudaEventRecord(ev0, s));
     SP_CUDA_TRY(cudaStreamWaitEvent(cs, ev0, 0));
-    // the search is launched first (its move-ins wait for the ready flags on the device), so
-    // enqueueing the 2 x n_frames copies on the host overlaps the run instead of delaying it
+    // The copies are enqueued BEFORE the search is launched: the kernel spins on their flags,
+    // so under a serialising tool (ncu, CUDA_LAUNCH_BLOCKING=1) copies enqueued after it would
+    // never run — a launch-first order (tried in session 3: 8.54 vs 8.56 ms on M4) deadlocks
+    // there until the kernel's trap.
+    for (int32_t f = 0; f < n_frames; ++f) {
+        SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f * fbytes, frames_host + f * fbytes, fbytes, cudaMemcpyHostToDevice, cs));
+        if (f >= 1) SP_CUDA_TRY(cudaMemcpyAsync(ready + (f - 1), one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
+    }
+    SP_CUDA_TRY(cudaEventRecord(ev1, cs));
     st = me_search_impl(frames_dev, frames_dev + fbytes, pitch, width, height, 0, height, pairs, (int64_t)fbytes, kMB,
                         range, 0, height / kMB, static_cast<int16_t*>(dmv), static_cast<uint32_t*>(dsad), nullptr,
                         stream, 0, ready);
-    if (!st) {
-        for (int32_t f = 0; f < n_frames; ++f) {
-            SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f * fbytes, frames_host + f * fbytes, fbytes,
-                                        cudaMemcpyHostToDevice, cs));
-            if (f >= 1) SP_CUDA_TRY(cudaMemcpyAsync(ready + (f - 1), one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
-        }
-    }
-    SP_CUDA_TRY(cudaEventRecord(ev1, cs));
     // the caller's stream completes only after the copies did (frames_dev / ready reusable)
     SP_CUDA_TRY(cudaStreamWaitEvent(s, ev1, 0));
     cudaEventDestroy(ev0);

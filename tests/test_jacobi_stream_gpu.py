@@ -151,3 +151,35 @@ def test_host_copy_engine_chunks(n, tt):
     ctx.run(h)
     torch.cuda.synchronize()
     _check(h, oracle.jacobi1d(a, steps))
+
+
+def test_host_paths_under_launch_blocking():
+    """The host-buffer calls stay correct when every launch is serialised
+    (CUDA_LAUNCH_BLOCKING=1, as under ncu): their kernels spin on ready flags set by copies on a
+    side stream, so those copies must be enqueued before the launch (a launch-first order
+    deadlocked until the kernel's trap)."""
+    import os
+    import subprocess
+    import sys
+    code = r"""
+import numpy as np, torch, oracle, sp_inputs
+import paper_conf_ppopp_baskaranbkrrs08_b200 as sp
+n, steps = 300007, 150
+a = sp_inputs.jacobi_input(n, seed=9)
+h = torch.from_numpy(a.copy()).pin_memory()
+sp.Jacobi1DHost(n, steps, 64).run(h)
+torch.cuda.synchronize()
+assert np.array_equal(h.numpy().view(np.uint32), oracle.jacobi1d(a, steps).view(np.uint32))
+W, H, R = 352, 288, 16
+fr = sp_inputs.me_sequence(4, W, H, R, seed=3)
+mv, sad = sp.me_search(fr, W, H, R)
+for p in range(3):
+    omv, osad, _ = oracle.me_search(fr[p], fr[p + 1], W, H, R)
+    assert np.array_equal(mv[p].numpy().reshape(-1, 2), omv)
+    assert np.array_equal(sad[p].numpy().view(np.uint32).reshape(-1), osad)
+print("ok")
+"""
+    env = dict(os.environ, CUDA_LAUNCH_BLOCKING="1")
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    r = subprocess.run([sys.executable, "-c", code], cwd=root, env=env, capture_output=True, text=True, timeout=300)
+    assert r.returncode == 0 and r.stdout.strip().endswith("ok"), r.stderr[-2000:]
