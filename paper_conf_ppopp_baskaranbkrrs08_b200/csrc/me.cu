@@ -1374,7 +1374,7 @@ const int32_t* pinned_one() {
         void* p = nullptr;
         if (cudaHostAlloc(&p, 64, cudaHostAllocPortable) == cudaSuccess) {
             one = static_cast<int32_t*>(p);
-            *one = 1;
+            for (int i = 0; i < 16; ++i) one[i] = 1;  // up to 16 ready flags per copy
         }
     });
     return one;
@@ -1428,9 +1428,19 @@ extern "C" int sp_me_search_host(const uint8_t* frames_host, int64_t pitch, int3
     // so under a serialising tool (ncu, CUDA_LAUNCH_BLOCKING=1) copies enqueued after it would
     // never run — a launch-first order (tried in session 3: 8.54 vs 8.56 ms on M4) deadlocks
     // there until the kernel's trap.
-    for (int32_t f = 0; f < n_frames; ++f) {
-        SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f * fbytes, frames_host + f * fbytes, fbytes, cudaMemcpyHostToDevice, cs));
-        if (f >= 1) SP_CUDA_TRY(cudaMemcpyAsync(ready + (f - 1), one, sizeof(int32_t), cudaMemcpyHostToDevice, cs));
+    // frames in groups — the first pair's two frames, then single frames while the search
+    // ramps up, then four at a time — each group followed by one copy of the ready flags of
+    // the pairs it completes (38 enqueued copies for M4's 65 frames instead of 130: the
+    // enqueue sits before the launch)
+    for (int32_t f0 = 0; f0 < n_frames;) {
+        const int32_t g = f0 == 0 ? 2 : f0 < 5 ? 1 : 4;
+        const int32_t f1 = f0 + g < n_frames ? f0 + g : n_frames;
+        SP_CUDA_TRY(cudaMemcpyAsync(frames_dev + f0 * fbytes, frames_host + f0 * fbytes, (size_t)(f1 - f0) * fbytes,
+                                    cudaMemcpyHostToDevice, cs));
+        const int32_t p0 = f0 > 0 ? f0 - 1 : 0, p1 = f1 - 1;  // pairs p0 .. p1-1 now have both frames
+        if (p1 > p0)
+            SP_CUDA_TRY(cudaMemcpyAsync(ready + p0, one, (size_t)(p1 - p0) * sizeof(int32_t), cudaMemcpyHostToDevice, cs));
+        f0 = f1;
     }
     SP_CUDA_TRY(cudaEventRecord(ev1, cs));
     st = me_search_impl(frames_dev, frames_dev + fbytes, pitch, width, height, 0, height, pairs, (int64_t)fbytes, kMB,
