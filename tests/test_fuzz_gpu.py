@@ -92,3 +92,32 @@ def test_me_random_frames_surfaces(seed):
             assert np.array_equal(_bits(surf[p].cpu().numpy()).reshape(-1, side * side), osurf), case
             pairs_checked += 1
     assert pairs_checked >= 4
+
+
+@pytest.mark.parametrize("seed", range(6))
+def test_me_random_frames_multi_wave(seed, monkeypatch):
+    """Random frame sizes with more macroblocks than resident CTAs (each CTA then runs
+    macroblocks from both pipeline stages), R in {16, 32}, the R = 16 class order with border
+    searches forced on or off, and with a surface (every candidate's SAD, tails included)
+    on every other draw; all pairs against the oracle."""
+    rng = np.random.default_rng(900 + seed)
+    R = 16 if seed % 3 else 32
+    W = int(rng.integers(48, 360))
+    H = int(rng.integers(48, 300))
+    mbs = (W // 16) * (H // 16)
+    P = max(2, -(-(3000 if R == 16 else 1200) // mbs))
+    border = str(int(rng.integers(0, 2)))
+    monkeypatch.setenv("SP_ME_BORDER", border)
+    surface = seed % 2 == 1
+    pitch = (W + 15) // 16 * 16
+    fr = sp_inputs.me_sequence(P + 1, W, H, R, seed=int(rng.integers(1 << 30)), pitch=pitch)
+    mv, sad, surf = sp.me_search_sequence(torch.from_numpy(fr).cuda(), W, H, R, with_surface=surface)
+    torch.cuda.synchronize()
+    side = 2 * R + 1
+    for p in range(P):
+        omv, osad, osurf = oracle.me_search(fr[p], fr[p + 1], W, H, R, with_surface=surface)
+        case = (W, H, R, P, p, border, surface)
+        assert np.array_equal(mv[p].cpu().numpy().reshape(-1, 2), omv), case
+        assert np.array_equal(_bits(sad[p].cpu().numpy()).reshape(-1), osad), case
+        if surface:
+            assert np.array_equal(_bits(surf[p].cpu().numpy()).reshape(-1, side * side), osurf), case
