@@ -53,6 +53,16 @@ def test_jacobi_plan_geometry_host_only():
         sp.jacobi1d_plan(2, 64, 16, 0)
 
 
+def test_jacobi_host_flags_len_host_only():
+    """sp_jacobi1d_host's copy-engine route needs the persistent launch's tile flags, the unit
+    counter and one ready flag per SP_JACOBI_HOST_CHUNK = 2^21 cells"""
+    for n, tt in [(3, 64), (4099, 16), (1 << 26, 128), ((1 << 21) + 1, 48)]:
+        p = sp.jacobi1d_plan(n, 1024, tt, 0)
+        assert sp.jacobi1d_host_flags_len(n, 1024, tt) == p["persistent_tiles"] + 1 + -(-n // (1 << 21))
+    with pytest.raises(sp.SPError):
+        sp.jacobi1d_host_flags_len(2, 10, 16)
+
+
 def test_jacobi_tile_footprint_closed_form():
     assert sp.jacobi1d_tile_footprint(100, 5, 0, 16) == (0, 20)
     assert sp.jacobi1d_tile_footprint(100, 5, 96, 16) == (91, 99)
